@@ -1,0 +1,393 @@
+/*
+ * oracle.c -- CPU ORACLE for the k-Hamming tabu search on the Permuted Perceptron Problem
+ * (Luong, Melab, Talbi, "Large Neighborhood Local Search Optimization on GPUs", LSPP@IPDPS 2010;
+ * text in PAPER.md).
+ *
+ * THIS IS TEST INFRASTRUCTURE. Only tests/, __graft_entry__.smoke() and bench.py's
+ * cpu_baseline / --impl reference legs may load it. It shares no code with the CUDA path
+ * (paper_conf_ipps_luongmt10_b200/csrc): no headers, helpers, tables or constants. The product
+ * path never calls it.
+ *
+ * Style: plain and slow. Every fitness is recomputed FROM SCRATCH for every neighbour; the
+ * neighbourhood is enumerated with nested loops whose loop counter IS the rank (no index
+ * formula); the tabu list is the literal "until" array. The only "trick" is the textbook
+ * identity <a, v> = n - 2 popcount(a xor v) for +-1 vectors stored as sign bits, used by the
+ * *_packed variants for speed; the scalar variants do the int8 multiply-add and the tests check
+ * that the two agree.
+ *
+ * Parity status: every function is pinned by tests/test_oracle.py:
+ *   fitness      -- hand-computed golden values, f(V*) = 0 on planted instances, brute force
+ *                   zero set == multiset equality, f >= 0, parity f = #negative rows (mod 2)
+ *   rank order   -- itertools.combinations order, the paper's worked example (n = 6,
+ *                   (2,3) -> 9), Appendix A-D formulas, C(n,k) counts
+ *   selection    -- brute-force argmin with lowest-rank tie-break, tabu invariants
+ *   trajectory   -- stop-on-zero reaches a vector whose multiset equals S
+ */
+#include <stdint.h>
+#include <stdlib.h>
+#include <string.h>
+#ifdef _OPENMP
+#include <omp.h>
+#endif
+
+/* ---------------------------------------------------------------------------------------
+ * splitmix64 (reading R12 of DESIGN.md): one draw = s += 0x9E3779B97F4A7C15, then mix.
+ * Used only to derive V0 from a seed, exactly as ppp_inputs.start_vector does.
+ * ------------------------------------------------------------------------------------- */
+uint64_t oracle_splitmix64_next(uint64_t *s)
+{
+    uint64_t z;
+    *s += 0x9E3779B97F4A7C15ULL;
+    z = *s;
+    z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ULL;
+    z = (z ^ (z >> 27)) * 0x94D049BB133111EBULL;
+    return z ^ (z >> 31);
+}
+
+/* V0 in {+1,-1}^n: ceil(n/64) draws, bit i of the stream (LSB first) = 1 -> -1. */
+void oracle_start_vector(int32_t n, uint64_t seed, int8_t *V)
+{
+    uint64_t s = seed, w = 0;
+    for (int32_t i = 0; i < n; i++) {
+        if (i % 64 == 0) w = oracle_splitmix64_next(&s);
+        V[i] = ((w >> (i % 64)) & 1) ? -1 : 1;
+    }
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Histogram of Definition 1 / PAPER.md:227-229: H_b = #{ j : S_j = b }, b = 0..n.
+ * (Reading R1: bins 0..n; reading R2: H is the histogram of the given multiset S.)
+ * ------------------------------------------------------------------------------------- */
+static void histogram_of(const int32_t *vals, int32_t m, int32_t n, int32_t *H)
+{
+    for (int32_t b = 0; b <= n; b++) H[b] = 0;
+    for (int32_t j = 0; j < m; j++)
+        if (vals[j] >= 0 && vals[j] <= n) H[vals[j]]++;
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Fitness, PAPER.md:231-237 (Section IV-A):
+ *   f(V') = 30 * sum_{j=1..m} ( |(AV')_j| - (AV')_j ) + sum_{b} | H_b - H'_b |
+ * with H' the histogram of Y' = AV' over bins b = 0..n (reading R1). Scalar int8 path.
+ * ------------------------------------------------------------------------------------- */
+static int64_t fitness_from_Y(const int32_t *Y, int32_t m, int32_t n, const int32_t *H, int32_t *Hp)
+{
+    int64_t pen = 0, hst = 0;
+    histogram_of(Y, m, n, Hp);
+    for (int32_t j = 0; j < m; j++) {
+        int64_t y = Y[j];
+        pen += (y < 0 ? -y : y) - y;
+    }
+    for (int32_t b = 0; b <= n; b++) {
+        int64_t d = (int64_t)H[b] - Hp[b];
+        hst += d < 0 ? -d : d;
+    }
+    return 30 * pen + hst;
+}
+
+int64_t oracle_fitness(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V)
+{
+    int32_t *Y = malloc(sizeof(int32_t) * (size_t)m);
+    int32_t *H = malloc(sizeof(int32_t) * (size_t)(n + 1));
+    int32_t *Hp = malloc(sizeof(int32_t) * (size_t)(n + 1));
+    histogram_of(S, m, n, H);
+    for (int32_t j = 0; j < m; j++) { /* Y = A V' (Definition 1) */
+        int32_t acc = 0;
+        for (int32_t i = 0; i < n; i++) acc += (int32_t)A[(size_t)j * n + i] * V[i];
+        Y[j] = acc;
+    }
+    int64_t f = fitness_from_Y(Y, m, n, H, Hp);
+    free(Y); free(H); free(Hp);
+    return f;
+}
+
+/* A V' for every row, by the scalar definition. */
+void oracle_matvec(const int8_t *A, int32_t m, int32_t n, const int8_t *V, int32_t *Y)
+{
+    for (int32_t j = 0; j < m; j++) {
+        int32_t acc = 0;
+        for (int32_t i = 0; i < n; i++) acc += (int32_t)A[(size_t)j * n + i] * V[i];
+        Y[j] = acc;
+    }
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Packed representation for speed: a +-1 vector is stored as sign bits (bit = 1 <=> -1), 64 per
+ * word. Textbook identity: for x, v in {+-1}^n, <x, v> = n - 2 * popcount(bits(x) xor bits(v)).
+ * ------------------------------------------------------------------------------------- */
+typedef struct {
+    int32_t m, n, nw;      /* nw = ceil(n/64) */
+    uint64_t *abits;       /* m rows x nw words */
+    int32_t *H;            /* n+1 bins of S */
+} packed_t;
+
+static void pack_instance(const int8_t *A, int32_t m, int32_t n, const int32_t *S, packed_t *P)
+{
+    P->m = m; P->n = n; P->nw = (n + 63) / 64;
+    P->abits = calloc((size_t)m * P->nw, sizeof(uint64_t));
+    P->H = malloc(sizeof(int32_t) * (size_t)(n + 1));
+    for (int32_t j = 0; j < m; j++)
+        for (int32_t i = 0; i < n; i++)
+            if (A[(size_t)j * n + i] < 0) P->abits[(size_t)j * P->nw + i / 64] |= 1ULL << (i % 64);
+    histogram_of(S, m, n, P->H);
+}
+
+static void free_packed(packed_t *P) { free(P->abits); free(P->H); }
+
+static void pack_vector(const int8_t *V, int32_t n, uint64_t *vb)
+{
+    int32_t nw = (n + 63) / 64;
+    for (int32_t w = 0; w < nw; w++) vb[w] = 0;
+    for (int32_t i = 0; i < n; i++)
+        if (V[i] < 0) vb[i / 64] |= 1ULL << (i % 64);
+}
+
+/* From-scratch fitness of the packed vector vb (scratch buffers Y, Hp of sizes m, n+1). */
+static int64_t fitness_packed(const packed_t *P, const uint64_t *vb, int32_t *Y, int32_t *Hp)
+{
+    for (int32_t j = 0; j < P->m; j++) {
+        int32_t d = 0;
+        const uint64_t *a = P->abits + (size_t)j * P->nw;
+        for (int32_t w = 0; w < P->nw; w++) d += __builtin_popcountll(a[w] ^ vb[w]);
+        Y[j] = P->n - 2 * d;
+    }
+    return fitness_from_Y(Y, P->m, P->n, P->H, Hp);
+}
+
+int64_t oracle_fitness_packed(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V)
+{
+    packed_t P;
+    pack_instance(A, m, n, S, &P);
+    uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
+    int32_t *Y = malloc(sizeof(int32_t) * (size_t)m);
+    int32_t *Hp = malloc(sizeof(int32_t) * (size_t)(n + 1));
+    pack_vector(V, n, vb);
+    int64_t f = fitness_packed(&P, vb, Y, Hp);
+    free(vb); free(Y); free(Hp); free_packed(&P);
+    return f;
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Neighbourhoods, PAPER.md:105-125 (Section II): flip 1, 2 or 3 bits. The neighbourhood
+ * index space is enumerated by NESTED LOOPS i1 < i2 < i3 in increasing order; the rank of a
+ * flip set is the loop counter (reading R6: lexicographic order, the order of Prop. 1 /
+ * Appendix A for k = 2 and of the "set of plans" of Appendix C for k = 3).
+ * first_count[i1] = number of flip sets whose smallest index is i1, counted by a loop.
+ * ------------------------------------------------------------------------------------- */
+static int64_t count_with_first(int32_t n, int32_t k, int32_t i1)
+{
+    int64_t c = 0;
+    if (k == 1) return 1;
+    for (int32_t i2 = i1 + 1; i2 < n; i2++) {
+        if (k == 2) c += 1;
+        else c += n - 1 - i2; /* the i3 loop runs over i2+1 .. n-1 */
+    }
+    return c;
+}
+
+/* Number of neighbours C(n,k), counted by the same loops. */
+int64_t oracle_neighborhood_size(int32_t n, int32_t k)
+{
+    int64_t c = 0;
+    for (int32_t i1 = 0; i1 < n; i1++) c += count_with_first(n, k, i1);
+    return c;
+}
+
+/* Flip sets of the given ranks (ascending), by walking the nested loops once. */
+int32_t oracle_flipsets(int32_t n, int32_t k, const int64_t *ranks, int64_t cnt, int32_t *out)
+{
+    int64_t r = 0, q = 0;
+    if (k < 1 || k > 3) return -1;
+    for (int32_t i1 = 0; i1 < n && q < cnt; i1++) {
+        int32_t i2s = (k >= 2) ? i1 + 1 : 0, i2e = (k >= 2) ? n : 1;
+        for (int32_t i2 = i2s; i2 < i2e && q < cnt; i2++) {
+            int32_t i3s = (k == 3) ? i2 + 1 : 0, i3e = (k == 3) ? n : 1;
+            for (int32_t i3 = i3s; i3 < i3e && q < cnt; i3++, r++) {
+                while (q < cnt && ranks[q] == r) {
+                    out[3 * q] = i1;
+                    out[3 * q + 1] = (k >= 2) ? i2 : -1;
+                    out[3 * q + 2] = (k == 3) ? i3 : -1;
+                    q++;
+                }
+            }
+        }
+    }
+    return q == cnt ? 0 : -1;
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Evaluate every neighbour of V (Figs. 7/9/10: new_fitness[move_index] = compute_fitness(V, move))
+ * from scratch. mode 0: write all fitnesses to f_all (length C(n,k)); mode 1: only return
+ * the best admissible (f, r), admissible(r) <=> until[r] < t (reading R3), lowest rank wins
+ * ties (reading R5). `sample` (sorted ranks, mode 2) evaluates only those ranks into f_all.
+ * ------------------------------------------------------------------------------------- */
+typedef struct { int64_t f, r; } fr_t;
+
+static void flip(uint64_t *vb, int32_t i) { vb[i / 64] ^= 1ULL << (i % 64); }
+
+static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k, int mode,
+                               int64_t *f_all, const int32_t *until, int64_t t,
+                               const int64_t *sample, int64_t nsample, int nthreads)
+{
+    int32_t n = P->n;
+    int64_t *base = malloc(sizeof(int64_t) * (size_t)(n + 1));
+    base[0] = 0;
+    for (int32_t i1 = 0; i1 < n; i1++) base[i1 + 1] = base[i1] + count_with_first(n, k, i1);
+    fr_t best = { INT64_MAX, -1 };
+#ifdef _OPENMP
+    if (nthreads > 0) omp_set_num_threads(nthreads);
+#endif
+#pragma omp parallel
+    {
+        fr_t mine = { INT64_MAX, -1 };
+        uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P->nw);
+        int32_t *Y = malloc(sizeof(int32_t) * (size_t)P->m);
+        int32_t *Hp = malloc(sizeof(int32_t) * (size_t)(n + 1));
+#pragma omp for schedule(dynamic, 1)
+        for (int32_t i1 = 0; i1 < n; i1++) {
+            int64_t r = base[i1];
+            int64_t q = 0;
+            if (mode == 2) { /* first sampled rank >= r */
+                int64_t lo = 0, hi = nsample;
+                while (lo < hi) { int64_t mid = (lo + hi) / 2; if (sample[mid] < r) lo = mid + 1; else hi = mid; }
+                q = lo;
+                if (q >= nsample || sample[q] >= base[i1 + 1]) continue;
+            }
+            int32_t i2s = (k >= 2) ? i1 + 1 : 0, i2e = (k >= 2) ? n : 1;
+            for (int32_t i2 = i2s; i2 < i2e; i2++) {
+                int32_t i3s = (k == 3) ? i2 + 1 : 0, i3e = (k == 3) ? n : 1;
+                for (int32_t i3 = i3s; i3 < i3e; i3++, r++) {
+                    if (mode == 2) {
+                        if (q >= nsample || sample[q] != r) continue;
+                    }
+                    if (mode == 1 && until && !(until[r] < t)) continue; /* tabu */
+                    memcpy(vb, vb0, sizeof(uint64_t) * (size_t)P->nw);
+                    flip(vb, i1);
+                    if (k >= 2) flip(vb, i2);
+                    if (k == 3) flip(vb, i3);
+                    int64_t f = fitness_packed(P, vb, Y, Hp);
+                    if (mode == 0) f_all[r] = f;
+                    else if (mode == 2) { while (q < nsample && sample[q] == r) { f_all[q] = f; q++; } }
+                    else if (f < mine.f || (f == mine.f && r < mine.r)) { mine.f = f; mine.r = r; }
+                }
+            }
+        }
+#pragma omp critical
+        {
+            if (mine.f < best.f || (mine.f == best.f && mine.r < best.r)) best = mine;
+        }
+        free(vb); free(Y); free(Hp);
+    }
+    free(base);
+    return best;
+}
+
+int32_t oracle_eval_all(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
+                        int32_t k, int64_t *f_all, int32_t nthreads)
+{
+    if (k < 1 || k > 3 || n < k) return -1;
+    packed_t P;
+    pack_instance(A, m, n, S, &P);
+    uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
+    pack_vector(V, n, vb);
+    scan_neighbourhood(&P, vb, k, 0, f_all, NULL, 0, NULL, 0, nthreads);
+    free(vb); free_packed(&P);
+    return 0;
+}
+
+/* Fitness of sampled neighbours (ranks ascending) -- for full-size parity on sampled outputs. */
+int32_t oracle_eval_ranks(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
+                          int32_t k, const int64_t *ranks, int64_t cnt, int64_t *f_out, int32_t nthreads)
+{
+    if (k < 1 || k > 3 || n < k) return -1;
+    packed_t P;
+    pack_instance(A, m, n, S, &P);
+    uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
+    pack_vector(V, n, vb);
+    scan_neighbourhood(&P, vb, k, 2, f_out, NULL, 0, ranks, cnt, nthreads);
+    free(vb); free_packed(&P);
+    return 0;
+}
+
+/* Best admissible neighbour; tabu[r] != 0 marks rank r tabu (nullable). */
+int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
+                         int32_t k, const uint8_t *tabu, int64_t *best_f, int64_t *best_r, int32_t nthreads)
+{
+    if (k < 1 || k > 3 || n < k) return -1;
+    int64_t M = oracle_neighborhood_size(n, k);
+    int32_t *until = NULL;
+    if (tabu) {
+        until = malloc(sizeof(int32_t) * (size_t)M);
+        for (int64_t r = 0; r < M; r++) until[r] = tabu[r] ? 1 : 0; /* admissible at t=1 iff until < 1 */
+    }
+    packed_t P;
+    pack_instance(A, m, n, S, &P);
+    uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
+    pack_vector(V, n, vb);
+    fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, 1, NULL, 0, nthreads);
+    *best_f = b.f == INT64_MAX ? -1 : b.f;
+    *best_r = b.r;
+    free(vb); free_packed(&P); free(until);
+    return b.r < 0 ? -6 : 0;
+}
+
+/* ---------------------------------------------------------------------------------------
+ * Tabu search, PAPER.md:241-258 (Section IV-B) after Taillard [11]; Fig. 1:
+ * at each iteration the whole neighbourhood is generated and evaluated and the best candidate
+ * replaces the current solution.
+ *   - tabu list: FIFO of the last L accepted move ranks (reading R3), implemented literally as
+ *     until[r]: a rank accepted at iteration t is tabu for t+1 .. t+L;
+ *   - no aspiration (reading R4); lowest rank wins ties (reading R5);
+ *   - stop when f = 0 if stop_on_zero (checked before every iteration, also before t = 1),
+ *     otherwise after `iters` iterations (reading R11).
+ * res[0..5] = iters_done, final_f, best_f, best_iter, first_zero_iter (-1: never), solved.
+ * ------------------------------------------------------------------------------------- */
+int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S, int32_t k,
+                        const int8_t *V0, int64_t iters, int64_t L, int32_t stop_on_zero,
+                        int64_t *trace_r, int64_t *trace_f, int8_t *V_out, int64_t *res,
+                        int32_t nthreads)
+{
+    if (k < 1 || k > 3 || n < k || m < 1 || iters < 0 || L < 0) return -1;
+    int64_t M = oracle_neighborhood_size(n, k);
+    if (L >= M) return -2;
+    packed_t P;
+    pack_instance(A, m, n, S, &P);
+    uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
+    int32_t *Y = malloc(sizeof(int32_t) * (size_t)m);
+    int32_t *Hp = malloc(sizeof(int32_t) * (size_t)(n + 1));
+    int32_t *until = calloc((size_t)M, sizeof(int32_t)); /* until[r] = 0: admissible from t = 1 */
+    pack_vector(V0, n, vb);
+    int64_t f = fitness_packed(&P, vb, Y, Hp);
+    int64_t best_f = f, best_iter = 0, first_zero = (f == 0) ? 0 : -1, t;
+    for (t = 1; t <= iters; t++) {
+        if (stop_on_zero && f == 0) break;
+        fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, t, NULL, 0, nthreads);
+        if (b.r < 0) break; /* unreachable for L < M */
+        /* apply: V <- V xor F_{r*}; flip set of r* found by walking the same nested loops */
+        int32_t F[3];
+        oracle_flipsets(n, k, &b.r, 1, F);
+        for (int32_t q = 0; q < k; q++) flip(vb, F[q]);
+        f = b.f;
+        until[b.r] = (int32_t)(t + L);
+        if (trace_r) trace_r[t - 1] = b.r;
+        if (trace_f) trace_f[t - 1] = b.f;
+        if (f < best_f) { best_f = f; best_iter = t; }
+        if (f == 0 && first_zero < 0) first_zero = t;
+    }
+    int64_t done = t - 1;
+    if (V_out)
+        for (int32_t i = 0; i < n; i++) V_out[i] = ((vb[i / 64] >> (i % 64)) & 1) ? -1 : 1;
+    res[0] = done; res[1] = f; res[2] = best_f; res[3] = best_iter; res[4] = first_zero;
+    res[5] = best_f == 0;
+    free(vb); free(Y); free(Hp); free(until); free_packed(&P);
+    return 0;
+}
+
+int32_t oracle_max_threads(void)
+{
+#ifdef _OPENMP
+    return omp_get_max_threads();
+#else
+    return 1;
+#endif
+}
