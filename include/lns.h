@@ -1,0 +1,173 @@
+/*
+ * lns.h -- C ABI of the B200 (sm_100a) large-neighbourhood tabu search for the Permuted
+ * Perceptron Problem (Luong, Melab, Talbi, "Large Neighborhood Local Search Optimization on
+ * Graphics Processing Units", LSPP @ IPDPS 2010; text in PAPER.md, cited as PAPER.md:<line>).
+ *
+ * The hot path: full evaluation of the k-Hamming neighbourhood (k = 1, 2, 3;
+ * sizes n, C(n,2), C(n,3)) of the current +-1 solution V, selection of the
+ * best non-tabu neighbour, and the move, inside a tabu search.
+ *
+ * Conventions shared by every entry point
+ *  - Problem (Definition 1): A is an m x n matrix with entries +-1, stored
+ *    ROW-MAJOR as int8 (A[j*n + i]); S is the multiset of m non-negative ints (int32); V is a
+ *    length-n int8 vector of +-1; Y = A V (int32, length m).
+ *  - Fitness: f(V) = 30 * sum_j (|Y_j| - Y_j) + sum_{b=0..n} |H_b - H'_b|,
+ *    H_b = #{j : S_j = b}, H'_b = #{j : Y_j = b}; bins 0..n (reading R1).
+ *  - Neighbour ranks: a neighbour flips the k distinct bits i1 < i2 < i3; its rank is its index
+ *    in LEXICOGRAPHIC order of (i1, i2, i3) (reading R6; the order of Prop. 1 / Appendix A for
+ *    k = 2, and of the "set of plans" of Appendix C for k = 3).
+ *  - Selection: the admissible neighbour of least fitness, ties to the LOWEST rank (R5); no
+ *    aspiration (R4). Tabu list: FIFO of the last `tenure` accepted ranks (R3); default tenure
+ *    floor(C(n,k)/6) ("m/6, m = number of neighbours").
+ *  - Pointers marked (host|device) may point to host memory or to device memory of the
+ *    context's device; the library detects which with cudaPointerGetAttributes. The caller
+ *    owns every buffer it passes; the library copies what it keeps.
+ *  - `stream` is a cudaStream_t (NULL = legacy default stream). Entry points that return
+ *    results to the host synchronise that stream before returning.
+ *  - Errors: every call returns an lns_status; the library never aborts. Asynchronous CUDA
+ *    errors surface at the next synchronisation as LNS_ECUDA. lns_strerror() names a code;
+ *    lns_last_error() gives a message for the last failure on the calling thread.
+ *  - Limits: 1 <= n, 1 <= m; C(n,k) < 2^32 - 1 (n <= 2954 for k = 3); 60 m n + 2 m < 2^31
+ *    (so fitness fits int32 and the (fitness, rank) key fits 63 bits); the bit-packed A of
+ *    ceil(m/32) * n words must fit in shared memory (m*n <= ~1.3e6, e.g. 1024 x 1024).
+ */
+#ifndef LNS_H
+#define LNS_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef int32_t lns_status;
+#define LNS_OK 0
+#define LNS_EINVAL (-1)         /* bad argument (k not in {1,2,3}, n < k, A not +-1, S outside [0,n], Y != A V, ...) */
+#define LNS_ERANGE (-2)         /* size limit exceeded (see Limits), or tenure >= C(n,k) */
+#define LNS_ENOMEM (-3)         /* device or host allocation failed */
+#define LNS_ECUDA (-4)          /* CUDA runtime error (message in lns_last_error) */
+#define LNS_ENCCL (-5)          /* NCCL missing or failed */
+#define LNS_ENOADMISSIBLE (-6)  /* every neighbour is tabu (best_rank = -1) */
+
+#define LNS_STOP_ON_ZERO 1      /* stop the search when f = 0 */
+#define LNS_FORCE_STEPPED 2     /* run one launch sequence per iteration instead of the persistent kernel */
+
+typedef struct lns_ctx lns_ctx;
+
+/* Outcome of one tabu search (PAPER.md:256-258 report fitness, #iterations and success). */
+typedef struct {
+    int64_t iters_done;      /* iterations performed (an iteration = evaluate all C(n,k) + move) */
+    int64_t final_f;         /* fitness of the final solution */
+    int64_t best_f;          /* least fitness seen, including the start vector */
+    int64_t best_iter;       /* first iteration reaching best_f (0 = start vector) */
+    int64_t first_zero_iter; /* first iteration with f = 0 (0 = start, -1 = never) */
+    int32_t solved;          /* best_f == 0 */
+    int32_t reserved;
+} lns_result;
+
+/* lns_create -- upload one PPP instance (Definition 1) to `device`.
+ *   A: (host|device) m x n int8 row-major, entries +-1.  S: (host|device) m int32 in [0, n].
+ *   The library bit-packs A and builds the histogram H of S; the caller
+ *   keeps A and S. *out receives a context owned by the library until lns_destroy.
+ *   Errors: EINVAL (m < 1, n < 1, entry of A not +-1, S_j outside [0,n]), ERANGE (limits),
+ *   ENOMEM, ECUDA. */
+lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, int32_t device,
+                      lns_ctx **out);
+
+/* lns_destroy -- free everything the context owns (NULL is a no-op). */
+void lns_destroy(lns_ctx *ctx);
+
+/* lns_eval_neighborhood -- evaluate all C(n,k) neighbours of V (Figs. 7/9/10, PAPER.md:212-216,
+ *   371-383, 405-413) and return the admissible neighbour of least fitness, lowest rank on ties.
+ *   V: (host|device) n int8 +-1.  Y: (host|device) m int32, must equal A V (verified on the
+ *   device; EINVAL otherwise).  tabu_bits: (host|device) ceil(C(n,k)/32) uint32 words,
+ *   bit r%32 of word r/32 set <=> rank r is tabu; NULL = nothing tabu.  If a partition was set
+ *   (lns_set_partition / lns_attach_comm) only that slice of ranks is evaluated.
+ *   best_fitness, best_rank: host int64 outputs. Synchronous.
+ *   Errors: EINVAL, ERANGE, ENOADMISSIBLE (all evaluated ranks tabu: best_rank = -1,
+ *   best_fitness = -1), ECUDA. */
+lns_status lns_eval_neighborhood(lns_ctx *ctx, int32_t k, const int8_t *V, const int32_t *Y,
+                                 const uint32_t *tabu_bits, int64_t *best_fitness,
+                                 int64_t *best_rank, void *stream);
+
+/* lns_eval_all -- the fitness of every neighbour of V, by rank (the paper's new_fitness[]
+ *   array).  fitness_out: (host|device) C(n,k) int32.  Ignores partitions.
+ *   Synchronous. Errors: EINVAL, ERANGE, ECUDA. */
+lns_status lns_eval_all(lns_ctx *ctx, int32_t k, const int8_t *V, int32_t *fitness_out, void *stream);
+
+/* lns_tabu_run -- tabu search of PAPER.md:241-258: `iters` iterations (or until f = 0 when
+ *   flags & LNS_STOP_ON_ZERO), each evaluating every neighbour and moving to the best
+ *   admissible one (tie -> lowest rank), with a FIFO tabu list of `tenure` ranks
+ *   (tenure < 0 -> floor(C(n,k)/6)).
+ *   V0: (host|device) n int8 +-1, or NULL -> drawn from `seed` (splitmix64, reading R12:
+ *   ceil(n/64) draws, bit i LSB-first, 1 -> -1).
+ *   V_out: (host|device) n int8 final solution, nullable.  trace_rank, trace_fit:
+ *   (host|device) int64 arrays of length `iters`, nullable; entry t-1 = (rank, fitness) accepted
+ *   at iteration t.  res: host, required.  With a communicator attached (lns_attach_comm) every
+ *   rank of the communicator must call this with identical arguments: each GPU evaluates its
+ *   slice of ranks and one NCCL u64-MIN all-reduce per iteration picks the global move; the
+ *   trajectory is identical for any number of GPUs.  Synchronous.
+ *   Errors: EINVAL, ERANGE (limits, tenure >= C(n,k)), ENOMEM, ECUDA, ENCCL. */
+lns_status lns_tabu_run(lns_ctx *ctx, int32_t k, int64_t iters, int64_t tenure, uint64_t seed,
+                        const int8_t *V0, int32_t flags, int8_t *V_out, int64_t *trace_rank,
+                        int64_t *trace_fit, lns_result *res, void *stream);
+
+/* lns_tabu_run_batch -- R independent searches (restarts) of lns_tabu_run on this device.
+ *   Restart r starts from V0 + r*n when V0 != NULL, else from the splitmix64 vector of
+ *   seed_r = first splitmix64 output of a stream seeded with seed + r (reading R12).
+ *   V_out: (host|device) R x n int8, nullable.  res: host, R entries.  Ignores partitions and
+ *   communicators (restarts are sharded across GPUs by the caller).  Synchronous.
+ *   Errors: as lns_tabu_run. */
+lns_status lns_tabu_run_batch(lns_ctx *ctx, int32_t k, int32_t R, int64_t iters, int64_t tenure,
+                              uint64_t seed, const int8_t *V0, int32_t flags, int8_t *V_out,
+                              lns_result *res, void *stream);
+
+/* lns_unrank -- flip sets of ranks (device kernel; used by tests of the rank order).
+ *   ranks: (host|device) count int64 in [0, C(n,k)).  out: (host|device) count x 3 int32,
+ *   unused slots -1.  Synchronous. Errors: EINVAL (rank out of range), ERANGE, ECUDA. */
+lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count, int32_t *out,
+                      void *stream);
+
+/* lns_set_partition -- restrict evaluation to slice `part` of `nparts` of the rank space
+ *   ("partitioning the neighborhood set, where each partition is executed on
+ *   a single GPU"). Slice g = [B(g), B(g+1)), B(g) = 32 * floor(C(n,k) * g / (32 nparts)),
+ *   B(nparts) = C(n,k). Errors: EINVAL. */
+lns_status lns_set_partition(lns_ctx *ctx, int32_t part, int32_t nparts);
+
+/* lns_attach_comm -- borrow an NCCL communicator (ncclComm_t of the libnccl already loaded in
+ *   the process, e.g. torch's) for multi-GPU lns_tabu_run; sets the partition to (rank, world).
+ *   The communicator is not freed by the library. comm = NULL detaches. Errors: ENCCL. */
+lns_status lns_attach_comm(lns_ctx *ctx, void *nccl_comm, int32_t rank, int32_t world);
+
+/* Stepped interface (one iteration at a time; used by multi-process drivers that own the
+ * collective, e.g. torch.distributed):
+ *   lns_step_begin  -- start a search (arguments as lns_tabu_run; trace capacity = max_iters).
+ *   lns_step_eval   -- evaluate this context's slice for the current iteration and store the
+ *                      partial best key ((fitness << 32) | rank, or INT64_MAX if nothing is
+ *                      admissible) into key_dev[0] (device int64). Asynchronous on `stream`.
+ *   lns_step_apply  -- key_dev[0] now holds the GLOBAL minimum key (after an all-reduce MIN):
+ *                      apply that move, update the tabu list and the trace. Asynchronous.
+ *   lns_step_end    -- copy out V_out / traces / result as lns_tabu_run does. Synchronous.
+ * Iterations after f = 0 (with LNS_STOP_ON_ZERO) are no-ops on the device. */
+lns_status lns_step_begin(lns_ctx *ctx, int32_t k, int64_t max_iters, int64_t tenure, uint64_t seed,
+                          const int8_t *V0, int32_t flags, void *stream);
+lns_status lns_step_eval(lns_ctx *ctx, int64_t *key_dev, void *stream);
+lns_status lns_step_apply(lns_ctx *ctx, const int64_t *key_dev, void *stream);
+lns_status lns_step_end(lns_ctx *ctx, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit,
+                        lns_result *res, void *stream);
+
+/* lns_last_kernel_ms -- device time (CUDA events) of the hot kernel(s) of the last run or eval. */
+double lns_last_kernel_ms(lns_ctx *ctx);
+
+/* lns_config -- override launch parameters (0 = automatic): blocks per search. */
+lns_status lns_config(lns_ctx *ctx, int32_t blocks);
+
+int64_t lns_neighborhood_size(int32_t n, int32_t k); /* C(n,k), or -1 if k not in {1,2,3} */
+const char *lns_strerror(lns_status status);
+const char *lns_last_error(void);
+int32_t lns_version(void); /* major*10000 + minor*100 + patch */
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* LNS_H */

@@ -1,0 +1,295 @@
+"""B200-native k-Hamming tabu search for the Permuted Perceptron Problem.
+
+Thin ctypes binding of the C ABI in ``include/lns.h`` (same names, argument marshalling only):
+every step of the hot path -- neighbourhood evaluation, best-move selection, the move and the
+tabu bookkeeping -- runs in the sm_100a kernels of ``csrc/lns.cu`` inside ``liblns.so``.
+There is no CPU fallback: if the library or a CUDA device is missing, calls raise.
+
+Buffers may be numpy arrays (host), torch CPU tensors or torch CUDA tensors; they are passed by
+pointer (the library copies host data itself). Paper: Luong, Melab, Talbi, LSPP@IPDPS 2010
+(PAPER.md); see DESIGN.md for the readings of the paper this follows.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+from typing import Any, Optional
+
+import numpy as np
+
+from . import _build
+
+LNS_OK = 0
+LNS_EINVAL = -1
+LNS_ERANGE = -2
+LNS_ENOMEM = -3
+LNS_ECUDA = -4
+LNS_ENCCL = -5
+LNS_ENOADMISSIBLE = -6
+LNS_STOP_ON_ZERO = 1
+LNS_FORCE_STEPPED = 2
+KEY_NONE = (1 << 63) - 1
+
+RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_iter", "solved")
+
+
+class LnsError(RuntimeError):
+    def __init__(self, status: int, where: str, detail: str):
+        super().__init__(f"{where}: {detail} (status {status})")
+        self.status = status
+
+
+class lns_result(ctypes.Structure):
+    _fields_ = [("iters_done", ctypes.c_int64), ("final_f", ctypes.c_int64), ("best_f", ctypes.c_int64),
+                ("best_iter", ctypes.c_int64), ("first_zero_iter", ctypes.c_int64),
+                ("solved", ctypes.c_int32), ("reserved", ctypes.c_int32)]
+
+    def as_dict(self) -> dict:
+        return {f: int(getattr(self, f)) for f in RESULT_FIELDS}
+
+
+_lib = None
+_vp, _i32, _i64, _u64 = ctypes.c_void_p, ctypes.c_int32, ctypes.c_int64, ctypes.c_uint64
+_SIGS = {
+    "lns_create": (_i32, [_vp, _i32, _i32, _vp, _i32, ctypes.POINTER(_vp)]),
+    "lns_destroy": (None, [_vp]),
+    "lns_eval_neighborhood": (_i32, [_vp, _i32, _vp, _vp, _vp, ctypes.POINTER(_i64), ctypes.POINTER(_i64), _vp]),
+    "lns_eval_all": (_i32, [_vp, _i32, _vp, _vp, _vp]),
+    "lns_tabu_run": (_i32, [_vp, _i32, _i64, _i64, _u64, _vp, _i32, _vp, _vp, _vp, ctypes.POINTER(lns_result), _vp]),
+    "lns_tabu_run_batch": (_i32, [_vp, _i32, _i32, _i64, _i64, _u64, _vp, _i32, _vp, _vp, _vp]),
+    "lns_unrank": (_i32, [_i32, _i32, _vp, _i64, _vp, _vp]),
+    "lns_set_partition": (_i32, [_vp, _i32, _i32]),
+    "lns_attach_comm": (_i32, [_vp, _vp, _i32, _i32]),
+    "lns_step_begin": (_i32, [_vp, _i32, _i64, _i64, _u64, _vp, _i32, _vp]),
+    "lns_step_eval": (_i32, [_vp, _vp, _vp]),
+    "lns_step_apply": (_i32, [_vp, _vp, _vp]),
+    "lns_step_end": (_i32, [_vp, _vp, _vp, _vp, ctypes.POINTER(lns_result), _vp]),
+    "lns_last_kernel_ms": (ctypes.c_double, [_vp]),
+    "lns_config": (_i32, [_vp, _i32]),
+    "lns_neighborhood_size": (_i64, [_i32, _i32]),
+    "lns_strerror": (ctypes.c_char_p, [_i32]),
+    "lns_last_error": (ctypes.c_char_p, []),
+    "lns_version": (_i32, []),
+}
+
+
+def library_path() -> str:
+    return _build.LIB
+
+
+def load(build_if_missing: bool = True):
+    """Load liblns.so (building it with nvcc first if it is missing or stale)."""
+    global _lib
+    if _lib is None:
+        if build_if_missing and _build.stale():
+            _build.build()
+        if not os.path.exists(_build.LIB):
+            raise RuntimeError(f"CUDA extension {_build.LIB} is missing; run _build.build()")
+        lib = ctypes.CDLL(_build.LIB)
+        for name, (res, args) in _SIGS.items():
+            fn = getattr(lib, name)
+            fn.restype = res
+            fn.argtypes = args
+        _lib = lib
+    return _lib
+
+
+def _check(status: int, where: str):
+    if status != LNS_OK:
+        lib = load()
+        raise LnsError(status, where, (lib.lns_last_error() or b"").decode() or lib.lns_strerror(status).decode())
+
+
+# --------------------------------------------------------------------------- marshalling
+def _ptr(x, dtype) -> tuple[Optional[int], Any]:
+    """(pointer, keep-alive) for numpy arrays / torch tensors; None -> NULL."""
+    if x is None:
+        return None, None
+    if isinstance(x, np.ndarray):
+        a = np.ascontiguousarray(x, dtype=dtype)
+        return a.ctypes.data, a
+    try:
+        import torch
+    except ImportError:  # pragma: no cover
+        torch = None
+    if torch is not None and isinstance(x, torch.Tensor):
+        tdt = {np.int8: torch.int8, np.int32: torch.int32, np.int64: torch.int64, np.uint32: torch.int32}[dtype]
+        t = x.contiguous()
+        if t.dtype != tdt:
+            t = t.to(tdt)
+        return t.data_ptr(), t
+    a = np.ascontiguousarray(np.asarray(x), dtype=dtype)
+    return a.ctypes.data, a
+
+
+def _out_ptr(x, dtype):
+    """Output buffers must already have the right dtype and be contiguous (written in place)."""
+    if x is None:
+        return None
+    if isinstance(x, np.ndarray):
+        assert x.dtype == dtype and x.flags.c_contiguous, "output array must be contiguous " + str(dtype)
+        return x.ctypes.data
+    import torch
+
+    assert isinstance(x, torch.Tensor) and x.is_contiguous()
+    want = {np.int8: torch.int8, np.int32: torch.int32, np.int64: torch.int64}[dtype]
+    assert x.dtype == want, f"output tensor must be {want}"
+    return x.data_ptr()
+
+
+def _stream(stream) -> Optional[int]:
+    if stream is None:
+        return None
+    if isinstance(stream, int):
+        return stream
+    return int(stream.cuda_stream)  # torch.cuda.Stream
+
+
+# --------------------------------------------------------------------------- C ABI, same names
+def lns_version() -> int:
+    return int(load().lns_version())
+
+
+def lns_strerror(status: int) -> str:
+    return load().lns_strerror(status).decode()
+
+
+def lns_neighborhood_size(n: int, k: int) -> int:
+    return int(load().lns_neighborhood_size(n, k))
+
+
+def lns_create(A, S, device: int = 0) -> int:
+    """Upload an instance (A: m x n of +-1, S: m ints in [0, n]); returns the context handle."""
+    shape = tuple(A.shape)
+    m, n = int(shape[0]), int(shape[1])
+    pa, ka = _ptr(A, np.int8)
+    ps, ks = _ptr(S, np.int32)
+    out = _vp()
+    _check(load().lns_create(pa, m, n, ps, device, ctypes.byref(out)), "lns_create")
+    return out.value
+
+
+def lns_destroy(ctx: int) -> None:
+    load().lns_destroy(ctx)
+
+
+def lns_config(ctx: int, blocks: int = 0) -> None:
+    _check(load().lns_config(ctx, blocks), "lns_config")
+
+
+def lns_last_kernel_ms(ctx: int) -> float:
+    return float(load().lns_last_kernel_ms(ctx))
+
+
+def lns_set_partition(ctx: int, part: int, nparts: int) -> None:
+    _check(load().lns_set_partition(ctx, part, nparts), "lns_set_partition")
+
+
+def lns_attach_comm(ctx: int, comm_ptr: Optional[int], rank: int, world: int) -> None:
+    _check(load().lns_attach_comm(ctx, comm_ptr, rank, world), "lns_attach_comm")
+
+
+def lns_eval_neighborhood(ctx: int, k: int, V, Y, tabu_bits=None, stream=None) -> tuple[int, int]:
+    """(best fitness, best rank) over admissible neighbours; raises LnsError(ENOADMISSIBLE)."""
+    pv, kv = _ptr(V, np.int8)
+    py, ky = _ptr(Y, np.int32)
+    pt, kt = _ptr(tabu_bits, np.uint32)
+    bf, br = _i64(), _i64()
+    _check(load().lns_eval_neighborhood(ctx, k, pv, py, pt, ctypes.byref(bf), ctypes.byref(br), _stream(stream)),
+           "lns_eval_neighborhood")
+    return int(bf.value), int(br.value)
+
+
+def lns_eval_all(ctx: int, k: int, V, out=None, stream=None):
+    """Fitness of every neighbour by rank (int32); `out` may be a device tensor."""
+    if out is None:
+        n = len(V)
+        out = np.empty(lns_neighborhood_size(n, k), dtype=np.int32)
+    pv, kv = _ptr(V, np.int8)
+    _check(load().lns_eval_all(ctx, k, pv, _out_ptr(out, np.int32), _stream(stream)), "lns_eval_all")
+    return out
+
+
+def lns_tabu_run(ctx: int, k: int, iters: int, tenure: int = -1, seed: int = 0, V0=None,
+                 flags: int = LNS_STOP_ON_ZERO, V_out=None, trace_rank=None, trace_fit=None, stream=None) -> dict:
+    pv, kv = _ptr(V0, np.int8)
+    res = lns_result()
+    _check(load().lns_tabu_run(ctx, k, iters, tenure, seed & ((1 << 64) - 1), pv, flags, _out_ptr(V_out, np.int8),
+                               _out_ptr(trace_rank, np.int64), _out_ptr(trace_fit, np.int64), ctypes.byref(res),
+                               _stream(stream)), "lns_tabu_run")
+    return res.as_dict()
+
+
+def lns_tabu_run_batch(ctx: int, k: int, R: int, iters: int, tenure: int = -1, seed: int = 0, V0=None,
+                       flags: int = LNS_STOP_ON_ZERO, V_out=None, stream=None) -> list[dict]:
+    pv, kv = _ptr(V0, np.int8)
+    res = (lns_result * max(R, 1))()
+    _check(load().lns_tabu_run_batch(ctx, k, R, iters, tenure, seed & ((1 << 64) - 1), pv, flags,
+                                     _out_ptr(V_out, np.int8), res, _stream(stream)), "lns_tabu_run_batch")
+    return [res[i].as_dict() for i in range(R)]
+
+
+def lns_unrank(n: int, k: int, ranks, out=None, stream=None):
+    pr, kr = _ptr(ranks, np.int64)
+    cnt = int(len(ranks))
+    if out is None:
+        out = np.empty((cnt, 3), dtype=np.int32)
+    _check(load().lns_unrank(n, k, pr, cnt, _out_ptr(out, np.int32), _stream(stream)), "lns_unrank")
+    return out
+
+
+def lns_step_begin(ctx: int, k: int, max_iters: int, tenure: int = -1, seed: int = 0, V0=None,
+                   flags: int = LNS_STOP_ON_ZERO, stream=None) -> None:
+    pv, kv = _ptr(V0, np.int8)
+    _check(load().lns_step_begin(ctx, k, max_iters, tenure, seed & ((1 << 64) - 1), pv, flags, _stream(stream)),
+           "lns_step_begin")
+
+
+def lns_step_eval(ctx: int, key_dev, stream=None) -> None:
+    """key_dev: a CUDA int64 tensor (>= 1 element) that receives the partial best key."""
+    _check(load().lns_step_eval(ctx, _out_ptr(key_dev, np.int64), _stream(stream)), "lns_step_eval")
+
+
+def lns_step_apply(ctx: int, key_dev, stream=None) -> None:
+    _check(load().lns_step_apply(ctx, _out_ptr(key_dev, np.int64), _stream(stream)), "lns_step_apply")
+
+
+def lns_step_end(ctx: int, V_out=None, trace_rank=None, trace_fit=None, stream=None) -> dict:
+    res = lns_result()
+    _check(load().lns_step_end(ctx, _out_ptr(V_out, np.int8), _out_ptr(trace_rank, np.int64),
+                               _out_ptr(trace_fit, np.int64), ctypes.byref(res), _stream(stream)), "lns_step_end")
+    return res.as_dict()
+
+
+class Instance:
+    """RAII wrapper of an lns context (owning the handle)."""
+
+    def __init__(self, A, S, device: int = 0):
+        self.m, self.n = int(A.shape[0]), int(A.shape[1])
+        self.ctx = lns_create(A, S, device)
+
+    def close(self):
+        if getattr(self, "ctx", None):
+            lns_destroy(self.ctx)
+            self.ctx = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *exc):
+        self.close()
+
+    def tabu_run(self, k, iters, tenure=-1, seed=0, V0=None, stop_on_zero=True, trace=True, stream=None, flags=0):
+        tr = np.full(max(iters, 1), -1, np.int64) if trace else None
+        tf = np.full(max(iters, 1), -1, np.int64) if trace else None
+        Vo = np.empty(self.n, np.int8)
+        fl = (LNS_STOP_ON_ZERO if stop_on_zero else 0) | flags
+        res = lns_tabu_run(self.ctx, k, iters, tenure, seed, V0, fl, Vo, tr, tf, stream)
+        it = res["iters_done"]
+        return (tr[:it] if trace else None), (tf[:it] if trace else None), Vo, res

@@ -1,0 +1,69 @@
+"""CPU-side checks of the C ABI boundary: the library builds for sm_100a, loads, and exports
+every entry point include/lns.h declares; host-only entry points behave as documented."""
+import os
+import re
+import subprocess
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _declared():
+    src = open(os.path.join(ROOT, "include", "lns.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(lns_[a-z_]+)\s*\(", src)))
+
+
+def test_header_declares_the_boundary_calls():
+    names = _declared()
+    for need in ("lns_create", "lns_eval_neighborhood", "lns_tabu_run", "lns_tabu_run_batch",
+                 "lns_attach_comm", "lns_destroy", "lns_strerror", "lns_version", "lns_unrank"):
+        assert need in names
+
+
+def test_library_exports_every_declared_symbol():
+    import paper_conf_ipps_luongmt10_b200 as L
+
+    lib = L.load()
+    out = subprocess.run(["nm", "-D", "--defined-only", L.library_path()], capture_output=True, text=True,
+                         check=True).stdout
+    exported = set(re.findall(r"\bT (lns_\w+)", out))
+    for name in _declared():
+        assert name in exported, name
+        getattr(lib, name)
+    assert set(L._SIGS) == set(_declared())
+
+
+def test_library_is_sm100a():
+    import paper_conf_ipps_luongmt10_b200 as L
+
+    L.load()
+    out = subprocess.run(["cuobjdump", "--list-elf", L.library_path()], capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+
+
+def test_host_only_entry_points():
+    import paper_conf_ipps_luongmt10_b200 as L
+    from math import comb
+
+    assert L.lns_version() >= 100
+    for n in (1, 3, 21, 117, 1024, 2954):
+        for k in (1, 2, 3):
+            assert L.lns_neighborhood_size(n, k) == comb(n, k)
+    assert L.lns_neighborhood_size(10, 4) == -1
+    assert L.lns_strerror(L.LNS_ENOADMISSIBLE) == "no admissible neighbour"
+
+
+def test_no_cpu_fallback_without_gpu():
+    """On a host without a GPU the product path must fail loudly, never compute on the CPU."""
+    import torch
+
+    if torch.cuda.is_available():
+        pytest.skip("GPU present")
+    import numpy as np
+
+    import paper_conf_ipps_luongmt10_b200 as L
+
+    with pytest.raises(L.LnsError):
+        L.lns_create(np.ones((2, 3), np.int8), np.array([3, 3], np.int32))

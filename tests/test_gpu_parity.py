@@ -1,0 +1,300 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle, element by element.
+
+All work is integer, so every comparison is exact (bit-exact fitness values, ranks and whole
+trajectories). Inputs are the seeded planted instances of ppp_inputs.
+"""
+from math import comb
+
+import numpy as np
+import pytest
+
+import ppp_inputs as pi
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def L():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_luongmt10_b200 as lib
+
+    lib.load()
+    return lib
+
+
+def _rand_pm1(rng, n):
+    return np.where(rng.random(n) < 0.5, -1, 1).astype(np.int8)
+
+
+def _states(inst, rng, count=3):
+    """Random V, near-solution V (secret with 1-3 flips), and V = -secret (every row negative)."""
+    n = inst.n
+    out = [_rand_pm1(rng, n) for _ in range(count)]
+    near = inst.secret.copy()
+    near[rng.choice(n, size=min(3, n), replace=False)] *= -1
+    out.append(near)
+    out.append((-inst.secret).astype(np.int8))
+    out.append(inst.secret.copy())
+    return out
+
+
+# ------------------------------------------------------------------------------ unranking
+@pytest.mark.parametrize("k", [1, 2, 3])
+def test_unrank_exhaustive_small(L, orc, k):
+    for n in (3, 4, 5, 7, 31, 32, 33, 60):
+        M = comb(n, k)
+        r = np.arange(M, dtype=np.int64)
+        assert np.array_equal(L.lns_unrank(n, k, r), orc.flipsets(n, k, r))
+
+
+def test_unrank_exhaustive_C4(L, orc):
+    n, k = 117, 3
+    r = np.arange(comb(n, k), dtype=np.int64)
+    assert np.array_equal(L.lns_unrank(n, k, r), orc.flipsets(n, k, r))
+
+
+@pytest.mark.parametrize("n", [1024, 2954])
+def test_unrank_sampled_large(L, orc, n):
+    """Full-size rank spaces (C5: 1.78e8 ranks; the largest n with C(n,3) < 2^32): random ranks
+    plus every plan boundary (first/last rank of each smallest index)."""
+    k = 3
+    M = comb(n, k)
+    rng = np.random.default_rng(n)
+    firsts = [0]
+    for a in range(n - 3):
+        firsts.append(firsts[-1] + comb(n - 1 - a, 2))
+    bnd = np.array(firsts, dtype=np.int64)
+    ranks = np.unique(np.concatenate([bnd, bnd - 1, bnd + 1, rng.integers(0, M, 200000), [M - 1]]))
+    ranks = ranks[(ranks >= 0) & (ranks < M)]
+    assert np.array_equal(L.lns_unrank(n, k, ranks), orc.flipsets(n, k, ranks))
+
+
+# ------------------------------------------------------------------------------ evaluation
+SHAPES = [(21, 21, 1), (73, 73, 2), (19, 23, 3), (33, 40, 3), (64, 64, 3), (30, 30, 2), (65, 66, 1),
+          (81, 81, 3), (101, 117, 3), (1, 5, 3), (32, 3, 3), (200, 50, 3)]
+
+
+@pytest.mark.parametrize("m,n,k", SHAPES)
+def test_eval_all_matches_oracle(L, orc, m, n, k):
+    inst = pi.planted_instance(m, n, 7000 + m * 31 + n)
+    rng = np.random.default_rng(m * n + k)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        for V in _states(inst, rng, count=2):
+            got = L.lns_eval_all(ctx, k, V)
+            want = orc.eval_all(inst.A, inst.S, V, k)
+            assert np.array_equal(got.astype(np.int64), want)
+    finally:
+        L.lns_destroy(ctx)
+
+
+def test_eval_all_forced_ties_duplicate_columns(L, orc):
+    inst = pi.planted_instance(40, 30, 99)
+    A = inst.A.copy()
+    A[:, 7] = A[:, 3]
+    A[:, 20] = -A[:, 11]
+    ctx = L.lns_create(A, inst.S)
+    try:
+        rng = np.random.default_rng(1)
+        for k in (1, 2, 3):
+            V = _rand_pm1(rng, 30)
+            assert np.array_equal(L.lns_eval_all(ctx, k, V).astype(np.int64), orc.eval_all(A, inst.S, V, k))
+    finally:
+        L.lns_destroy(ctx)
+
+
+@pytest.mark.parametrize("m,n,k", [(21, 21, 1), (73, 73, 2), (81, 81, 3), (101, 117, 3), (47, 33, 3)])
+def test_eval_neighborhood_best_with_tabu(L, orc, m, n, k):
+    inst = pi.planted_instance(m, n, 4242 + n)
+    rng = np.random.default_rng(n)
+    M = comb(n, k)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        for V in _states(inst, rng, count=1):
+            Y = (inst.A.astype(np.int32) @ V.astype(np.int32)).astype(np.int32)
+            for frac in (0.0, 0.5, 1.0):
+                tabu = rng.random(M) < frac
+                if frac == 1.0:
+                    tabu[rng.integers(M)] = False  # exactly one admissible rank
+                bits = np.packbits(tabu, bitorder="little")
+                bits = np.concatenate([bits, np.zeros((-len(bits)) % 4, np.uint8)]).view(np.uint32)
+                got = L.lns_eval_neighborhood(ctx, k, V, Y, bits)
+                assert got == orc.eval_best(inst.A, inst.S, V, k, tabu)
+    finally:
+        L.lns_destroy(ctx)
+
+
+def test_eval_neighborhood_errors(L):
+    inst = pi.planted_instance(21, 21, 1)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        V = inst.secret
+        Y = (inst.A.astype(np.int32) @ V).astype(np.int32)
+        with pytest.raises(L.LnsError) as e:
+            L.lns_eval_neighborhood(ctx, 1, V, Y + 2)
+        assert e.value.status == L.LNS_EINVAL
+        with pytest.raises(L.LnsError) as e:
+            L.lns_eval_neighborhood(ctx, 4, V, Y)
+        assert e.value.status == L.LNS_EINVAL
+        allbits = np.full(1, 0xFFFFFFFF, np.uint32)
+        with pytest.raises(L.LnsError) as e:
+            L.lns_eval_neighborhood(ctx, 1, V, Y, allbits)
+        assert e.value.status == L.LNS_ENOADMISSIBLE
+        with pytest.raises(L.LnsError) as e:
+            L.lns_tabu_run(ctx, 1, 10, tenure=21)
+        assert e.value.status == L.LNS_ERANGE
+    finally:
+        L.lns_destroy(ctx)
+    with pytest.raises(L.LnsError) as e:
+        L.lns_create(np.zeros((2, 2), np.int8), np.zeros(2, np.int32))
+    assert e.value.status == L.LNS_EINVAL
+    with pytest.raises(L.LnsError) as e:
+        L.lns_create(np.ones((2, 2), np.int8), np.array([0, 3], np.int32))
+    assert e.value.status == L.LNS_EINVAL
+
+
+def test_eval_C5_sampled(L, orc):
+    """C5 (1024 x 1024, k = 3, 1.78e8 neighbours): sampled fitnesses against the oracle, and the
+    returned best equals the minimum of the full GPU array and has the oracle's fitness."""
+    import torch
+
+    inst = pi.config_instance("C5")
+    rng = np.random.default_rng(5)
+    V = pi.start_vector(1024, pi.config_seed("C5"))
+    M = comb(1024, 3)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        out = torch.empty(M, dtype=torch.int32, device="cuda")
+        L.lns_eval_all(ctx, 3, V, out)
+        ranks = np.unique(np.concatenate([rng.integers(0, M, 3000), [0, M - 1]]))
+        got = out[torch.from_numpy(ranks).cuda()].cpu().numpy().astype(np.int64)
+        assert np.array_equal(got, orc.eval_ranks(inst.A, inst.S, V, 3, ranks))
+        Y = (inst.A.astype(np.int32) @ V.astype(np.int32)).astype(np.int32)
+        bf, br = L.lns_eval_neighborhood(ctx, 3, V, Y)
+        mn = int(out.min().item())
+        first = int(torch.nonzero(out == mn)[0].item())
+        assert (bf, br) == (mn, first)
+        assert orc.eval_ranks(inst.A, inst.S, V, 3, [br])[0] == bf
+    finally:
+        L.lns_destroy(ctx)
+
+
+# ------------------------------------------------------------------------------ trajectories
+TRAJ = [("C1", 1000, True), ("C1", 1000, False), ("C2", 10000, False), ("C3", 1000, False), ("C4", 400, False)]
+
+
+@pytest.mark.parametrize("cfg,iters,stop", TRAJ)
+def test_tabu_trajectory_bit_exact(L, orc, cfg, iters, stop):
+    c = pi.CONFIGS[cfg]
+    inst = pi.config_instance(cfg)
+    seed = pi.config_seed(cfg)
+    V0 = pi.start_vector(inst.n, seed)
+    L_ten = pi.default_tenure(inst.n, c["k"])
+    with L.Instance(inst.A, inst.S) as I:
+        tr, tf, Vo, res = I.tabu_run(c["k"], iters, -1, seed=seed, V0=None, stop_on_zero=stop)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, c["k"], V0, iters, L_ten, stop_on_zero=stop)
+    assert res == ores
+    assert np.array_equal(tr, otr)
+    assert np.array_equal(tf, otf)
+    assert np.array_equal(Vo, oVo)
+
+
+@pytest.mark.parametrize("k,L_ten", [(1, 0), (2, 1), (2, 2), (3, 5), (3, 0)])
+def test_trajectory_short_tenures_and_forced_stepped(L, orc, k, L_ten):
+    """Tenures 0, 1, 2 exercise the ring-buffer edge cases; the stepped launch sequence (the
+    multi-GPU code path) must give the same trajectory as the persistent kernel."""
+    inst = pi.planted_instance(37, 29, 555 + k)
+    V0 = pi.start_vector(29, 11 + k)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0, 150, L_ten, stop_on_zero=False)
+    with L.Instance(inst.A, inst.S) as I:
+        for flags in (0, L.LNS_FORCE_STEPPED):
+            tr, tf, Vo, res = I.tabu_run(k, 150, L_ten, V0=V0, stop_on_zero=False, flags=flags)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+            assert np.array_equal(Vo, oVo)
+
+
+@pytest.mark.parametrize("blocks", [1, 2, 7, 148])
+def test_trajectory_independent_of_grid_size(L, orc, blocks):
+    inst = pi.config_instance("C3")
+    V0 = pi.start_vector(81, 4)
+    otr, otf, _, ores = orc.tabu_run(inst.A, inst.S, 3, V0, 60, pi.default_tenure(81, 3), stop_on_zero=False)
+    with L.Instance(inst.A, inst.S) as I:
+        L.lns_config(I.ctx, blocks)
+        tr, tf, _, res = I.tabu_run(3, 60, -1, V0=V0, stop_on_zero=False)
+    assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+
+
+@pytest.mark.parametrize("G", [2, 3, 8])
+def test_partitioned_search_emulated_on_one_gpu(L, orc, G):
+    """The multi-GPU protocol (PAPER.md:448-454 partitioning): G contexts each own a slice of the
+    rank space; per iteration every slice's partial key is min-reduced and applied everywhere.
+    The trajectory must equal the single-partition one (a u64 MIN of exact keys is associative)."""
+    import torch
+
+    inst = pi.config_instance("C4")
+    V0 = pi.start_vector(117, 5)
+    iters = 40
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0, iters, pi.default_tenure(117, 3), stop_on_zero=False)
+    ctxs = [L.lns_create(inst.A, inst.S) for _ in range(G)]
+    try:
+        keys = torch.empty((G, 1), dtype=torch.int64, device="cuda")
+        for g, c in enumerate(ctxs):
+            L.lns_set_partition(c, g, G)
+            L.lns_step_begin(c, 3, iters, -1, 0, V0, 0)
+        for _ in range(iters):
+            for g, c in enumerate(ctxs):
+                L.lns_step_eval(c, keys[g])
+            keys.copy_(keys.min(dim=0, keepdim=True).values.expand(G, 1))
+            for g, c in enumerate(ctxs):
+                L.lns_step_apply(c, keys[g])
+        torch.cuda.synchronize()
+        for c in ctxs:
+            tr = np.empty(iters, np.int64)
+            tf = np.empty(iters, np.int64)
+            Vo = np.empty(117, np.int8)
+            res = L.lns_step_end(c, Vo, tr, tf)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+            assert np.array_equal(Vo, oVo)
+    finally:
+        for c in ctxs:
+            L.lns_destroy(c)
+
+
+def test_batch_restarts_match_single_runs(L, orc):
+    inst = pi.config_instance("C2")
+    with L.Instance(inst.A, inst.S) as I:
+        R = 4
+        Vo = np.empty((R, 73), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, 2, R, 300, -1, 17, None, L.LNS_STOP_ON_ZERO, Vo)
+        for r in range(R):
+            V0 = pi.start_vector(73, pi.restart_seed(17, r))
+            _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, 2, V0, 300, pi.default_tenure(73, 2))
+            assert batch[r] == ores
+            assert np.array_equal(Vo[r], oVo)
+
+
+def test_C5_two_iterations_properties(L, orc):
+    """C5 trajectories are beyond the oracle (1.9e14 ops per iteration); check the first two
+    iterations by sampled properties: each accepted fitness equals the oracle's from-scratch
+    fitness of the resulting vector, and is <= every sampled admissible neighbour's fitness."""
+    inst = pi.config_instance("C5")
+    seed = pi.config_seed("C5")
+    V = pi.start_vector(1024, seed)
+    rng = np.random.default_rng(55)
+    M = comb(1024, 3)
+    with L.Instance(inst.A, inst.S) as I:
+        tr, tf, Vo, res = I.tabu_run(3, 2, -1, seed=seed, stop_on_zero=False)
+    assert res["iters_done"] == 2
+    for t in range(2):
+        sample = np.unique(rng.integers(0, M, 2000))
+        sample = sample[~np.isin(sample, tr[:t])]
+        fs = orc.eval_ranks(inst.A, inst.S, V, 3, sample)
+        assert tf[t] <= fs.min()
+        (f3,) = orc.flipsets(1024, 3, [tr[t]])
+        V = V.copy()
+        V[f3] *= -1
+        assert orc.fitness(inst.A, inst.S, V, packed=True) == tf[t]
+    assert np.array_equal(V, Vo)
