@@ -74,18 +74,20 @@ _SIGS = {
 
 
 def library_path() -> str:
-    return _build.LIB
+    """liblns.so in the package (LNS_LIB may point at a variant build, e.g. the profiling one)."""
+    return os.environ.get("LNS_LIB") or _build.LIB
 
 
 def load(build_if_missing: bool = True):
     """Load liblns.so (building it with nvcc first if it is missing or stale)."""
     global _lib
     if _lib is None:
-        if build_if_missing and _build.stale():
+        path = library_path()
+        if build_if_missing and path == _build.LIB and _build.stale():
             _build.build()
-        if not os.path.exists(_build.LIB):
-            raise RuntimeError(f"CUDA extension {_build.LIB} is missing; run _build.build()")
-        lib = ctypes.CDLL(_build.LIB)
+        if not os.path.exists(path):
+            raise RuntimeError(f"CUDA extension {path} is missing; run _build.build()")
+        lib = ctypes.CDLL(path)
         for name, (res, args) in _SIGS.items():
             fn = getattr(lib, name)
             fn.restype = res

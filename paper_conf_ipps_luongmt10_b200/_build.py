@@ -32,19 +32,23 @@ def stale() -> bool:
     return any(os.path.getmtime(p) > t for p in SRC + HDR)
 
 
-def build(force: bool = False, verbose: bool = False) -> str:
-    if not force and not stale():
+LIB_PROF = os.path.join(PKG, "liblns_prof.so")  # -DLNS_PHASE_TIMING variant for tools/profiling
+
+
+def build(force: bool = False, verbose: bool = False, profiling: bool = False) -> str:
+    lib = LIB_PROF if profiling else LIB
+    if not force and not profiling and not stale():
         return LIB
-    tmp = LIB + f".tmp{os.getpid()}"
-    cmd = [nvcc(), *NVCC_FLAGS, "-I", os.path.join(ROOT, "include"), "-o", tmp, *SRC, "-ldl"]
+    tmp = lib + f".tmp{os.getpid()}"
+    extra = ["-DLNS_PHASE_TIMING"] if profiling else []
+    cmd = [nvcc(), *NVCC_FLAGS, *extra, "-I", os.path.join(ROOT, "include"), "-o", tmp, *SRC, "-ldl"]
     if verbose:
         cmd.insert(1, "-Xptxas=-v")
         print(" ".join(cmd), file=sys.stderr)
     subprocess.check_call(cmd)
-    os.replace(tmp, LIB)
-    return LIB
+    os.replace(tmp, lib)
+    return lib
 
 
 if __name__ == "__main__":
-    build(force="--force" in sys.argv, verbose="-v" in sys.argv)
-    print(LIB)
+    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, profiling="--profiling" in sys.argv))

@@ -4,25 +4,29 @@
 // Design:
 //  * A is bit-packed once (sign bits, bit = 1 <=> -1). Per iteration every CTA builds, in shared
 //    memory, a "plan" of the current state: rows sorted by Y (counting sort over the lattice
-//    Y = vmin + 2u), the sign bits X = (A o V)'s "-1" indicator permuted into that row order and
-//    stored [row-word][column], the segment boundaries of equal-Y rows, and per-bin constants.
+//    Y = vmin + 2u), the sign bits x_jc = [A_jc V_c = -1] permuted into that row order and stored
+//    [row-word][column], the pieces (segment x row-word) of equal-Y rows, and per-bin constants.
 //  * A neighbour F = {a<b<c} moves row j to Y'_j = Y_j - 2k + 4 t_j, t_j = #{i in F : x_ji = 1}
 //    (PAPER.md:227-229 with V' = V xor F). All rows of one Y-segment land in the same k+1 bins, so
 //    the new histogram H' only needs, per segment, how many rows have t = 0..k.
-//    Those counts come from bit-sliced t (LOP3) and POPC over the segment's row words; a sliding
-//    window over the segment lattice turns them into H'(b) and the fitness (30-weighted penalty on
-//    negative bins, |H - H'| on bins 0..n), exactly, in integers.
+//    Those counts come from bit-sliced t (LOP3) and POPC over the segment's row words; a shift
+//    register over the segment lattice turns them into H'(b) and the fitness (60|b|-weighted
+//    penalty on negative bins, |H - H'| on bins 0..n), exactly, in integers.
 //  * Ranks are lexicographic (reading R6); each lane unranks exactly (integer combinatorial number
 //    system, float estimate + integer correction). The (fitness, rank) pair is packed into one
 //    63-bit key, so a u64 MIN gives "least fitness, lowest rank" (reading R5) at warp, CTA, grid and
 //    (NCCL) multi-GPU level.
-//  * The whole tabu search runs in ONE persistent cooperative kernel: one grid barrier per
-//    iteration; every CTA applies the winning move to its own shared-memory copy of (V, Y).
+//  * The whole tabu search runs in ONE persistent cooperative kernel. Per iteration each CTA
+//    publishes its best key into a parity-tagged slot and polls all slots (one exchange, no
+//    separate barrier); every CTA applies the winning move to its own shared copy of (V, Y).
+//    The tabu list is the literal until[] array of the oracle (rank r is tabu while
+//    until[r] >= t), each CTA owning (and caching in shared memory) the slice it evaluates.
 #include "lns.h"
 
 #include <cuda_runtime.h>
 #include <dlfcn.h>
 
+#include <algorithm>
 #include <climits>
 #include <cmath>
 #include <cstdio>
@@ -30,24 +34,46 @@
 #include <string>
 #include <vector>
 
-#define LNS_VERSION_NUM 100
+#define LNS_VERSION_NUM 200
 
 namespace {
 
 constexpr int64_t KEY_NONE = INT64_MAX;
-constexpr int NT = 512;           // threads per CTA
+#ifndef LNS_NT
+#define LNS_NT 1024
+#endif
+constexpr int NT = LNS_NT;  // threads per CTA
 constexpr int NWARP = NT / 32;
 constexpr unsigned FULL = 0xffffffffu;
+constexpr int MAX_SLOTS = 1024;  // CTAs per search that can exchange keys
 
 thread_local std::string g_err;
+
+// Optional per-phase cycle accounting (compile with -DLNS_PHASE_TIMING; tools/profiling only).
+#ifdef LNS_PHASE_TIMING
+constexpr int NPH = 8;
+__shared__ long long s_ph[NPH];
+__shared__ long long s_last;
+__device__ unsigned long long g_ph[NPH];
+#define PH(i)                                                        \
+    do {                                                             \
+        if (threadIdx.x == 0) {                                      \
+            const long long _now = clock64();                        \
+            s_ph[i] += _now - s_last;                                \
+            s_last = _now;                                           \
+        }                                                            \
+    } while (0)
+#else
+#define PH(i) do { } while (0)
+#endif
 
 // ------------------------------------------------------------------------------------------
 // Device data
 // ------------------------------------------------------------------------------------------
 struct DevInst {
-    int32_t m, n, W, NWn;      // W = ceil(m/32) row words, NWn = ceil(n/32) column words
-    const uint32_t *Arow;      // m x NWn, bit (i%32) of word i/32 = 1 <=> A[j][i] = -1
-    const int32_t *H;          // n+1 bins of S
+    int32_t m, n, W, NWn;  // W = ceil(m/32) row words, NWn = ceil(n/32) column words
+    const uint32_t *Arow;  // m x NWn, bit (i%32) of word i/32 = 1 <=> A[j][i] = -1
+    const int32_t *H;      // n+1 bins of S
 };
 
 // fstate layout (int64): current f, iterations done, best f, best iter, first zero iter, done, error
@@ -55,49 +81,58 @@ enum { FS_F = 0, FS_T, FS_BEST, FS_BESTIT, FS_ZERO, FS_DONE, FS_ERR, FS_N };
 
 struct SearchArgs {
     DevInst I;
-    uint32_t M;          // C(n,k)
-    uint32_t lo, hi;     // rank slice of this device
-    int64_t iters;       // iterations to run (persistent) / capacity (stepped)
-    int64_t L;           // tenure
+    uint32_t M;             // C(n,k)
+    uint32_t lo, hi;        // rank slice of this device
+    int64_t iters;          // iterations to run (persistent) / capacity (stepped)
+    int64_t L;              // tenure
     int32_t stop_on_zero;
-    uint32_t *vb;        // state: NWn words of V's sign bits
-    int32_t *Y;          // state: m
-    int64_t *fs;         // FS_N
-    uint32_t *tabu;      // ceil(M/32) words (only this device's slice is used)
-    uint32_t *ring;      // L+1 entries: rank accepted at iteration t sits in ring[t % (L+1)]
-    int64_t *keys;       // 3 slots (persistent) / accumulator (stepped)
-    unsigned *bar;       // grid barrier (count, generation) / stepped: last-block counter
+    int32_t a_in_smem;      // stage A's bit rows in shared memory
+    int32_t until_smem;     // cache the CTA's until[] slice in shared memory (capacity in entries, 0 = no)
+    uint32_t *vb;           // state: NWn words of V's sign bits
+    int32_t *Y;             // state: m
+    int64_t *fs;            // FS_N
+    uint32_t *until;        // M entries: rank r is tabu at iteration t iff until[r] >= t
+    int64_t *slots;         // 3 x MAX_SLOTS parity-tagged keys (persistent) / accumulator (stepped)
+    unsigned *counter;      // stepped: last-CTA counter
     int64_t *trace_r, *trace_f;
 };
 
-// Shared-memory carve-up (identical on host and device).
+// Shared-memory carve-up (identical on host and device). The bit-packed A (Ar) and the until[]
+// slice are staged only when they fit.
 struct Smem {
-    int X, Y, vb, H, seg, cur, rowAt, bins, total;
+    int X, Y, vb, H, cnt, seg, cur, pofs, rowAt, bins, pieces, pstart, base_end, Ar, a_end;
 };
 
 __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
 
-__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K)
+__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem)
 {
     Smem s;
     int o = 0;
-    s.X = o;     o = align16(o + 4 * W * n);
-    s.Y = o;     o = align16(o + 4 * m);
-    s.vb = o;    o = align16(o + 4 * NWn);
-    s.H = o;     o = align16(o + 4 * (n + 1));
-    s.seg = o;   o = align16(o + 4 * (n + 4));          // Upad + 1 <= n + 3
-    s.cur = o;   o = align16(o + 4 * (n + 4));
-    s.rowAt = o; o = align16(o + 4 * m);
-    s.bins = o;  o = align16(o + 8 * (n + 4 + 2 * K));  // Upad + 2K bins
-    s.total = o;
+    s.X = o;      o = align16(o + 4 * W * n);
+    s.Y = o;      o = align16(o + 4 * m);
+    s.vb = o;     o = align16(o + 4 * NWn);
+    s.H = o;      o = align16(o + 4 * (n + 1));
+    s.cnt = o;    o = align16(o + 4 * (n + 2 + 2 * K));  // conservative lattice Uc <= n + 1 + 2K
+    s.seg = o;    o = align16(o + 4 * (n + 2));          // seg[0..U], U <= n + 1
+    s.cur = o;    o = align16(o + 4 * (n + 2 + 2 * K));
+    s.pofs = o;   o = align16(o + 4 * (n + 2));
+    s.rowAt = o;  o = align16(o + 4 * m);
+    s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
+    s.pieces = o; o = align16(o + 8 * (n + 1 + W));      // P <= U + W - 1 pieces
+    s.pstart = o; o = align16(o + 4 * (W + 1));
+    s.base_end = o;
+    s.Ar = o;
+    if (a_in_smem) o = align16(o + 4 * m * NWn);
+    s.a_end = o;  // the until[] slice (if cached) follows
     return s;
 }
 
 struct PlanScalars {
-    int vmin, Upad, base;
-    int64_t key;
+    int vmin, U, NB, P, ufirst;
+    int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
+    unsigned long long key, gkey;
     int red[2 * NWARP + 2];
-    unsigned long long redk[NWARP];
 };
 
 __device__ __forceinline__ uint64_t C2(uint64_t y) { return y * (y - 1) / 2; }
@@ -139,10 +174,6 @@ __device__ __forceinline__ int warp_max_i(int v) {
     for (int o = 16; o; o >>= 1) v = max(v, __shfl_xor_sync(FULL, v, o));
     return v;
 }
-__device__ __forceinline__ int warp_sum_i(int v) {
-    for (int o = 16; o; o >>= 1) v += __shfl_xor_sync(FULL, v, o);
-    return v;
-}
 __device__ __forceinline__ unsigned long long warp_min_k(unsigned long long v) {
     for (int o = 16; o; o >>= 1) {
         unsigned long long w = __shfl_xor_sync(FULL, v, o);
@@ -151,43 +182,14 @@ __device__ __forceinline__ unsigned long long warp_min_k(unsigned long long v) {
     return v;
 }
 
-// Block-wide min of a key; result valid in all threads.
-__device__ unsigned long long block_min_key(unsigned long long v, PlanScalars &ps)
+// Value range of Y: every thread passes its partial (min, max); a __syncthreads, then warp 0 sets
+// the lattice ps.vlo / Uc of the next plan; callers must __syncthreads before reading them. (Written with min and max,
+// not min(-y): nvcc 12.9 miscompiled an unrolled "mx = min(mx, -y)" into a 3-input min that
+// dropped one negation.)
+template <int K>
+__device__ __forceinline__ void range_publish(int mn, int mx, PlanScalars &ps)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    v = warp_min_k(v);
-    if (lane == 0) ps.redk[warp] = v;
-    __syncthreads();
-    if (warp == 0) {
-        unsigned long long w = lane < NWARP ? ps.redk[lane] : (unsigned long long)KEY_NONE;
-        w = warp_min_k(w);
-        if (lane == 0) ps.key = (int64_t)w;
-    }
-    __syncthreads();
-    return (unsigned long long)ps.key;
-}
-
-// ------------------------------------------------------------------------------------------
-// Plan: per-iteration shared-memory structures of the current state (Y, V).
-// ------------------------------------------------------------------------------------------
-template <int K>
-__device__ void build_plan(const DevInst &I, unsigned char *sm, const Smem &L, PlanScalars &ps)
-{
-    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
-    const int m = I.m, n = I.n;
-    const int *Ys = (const int *)(sm + L.Y);
-    const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
-    const int *Hs = (const int *)(sm + L.H);
-    int *seg = (int *)(sm + L.seg);
-    int *cur = (int *)(sm + L.cur);
-    int *rowAt = (int *)(sm + L.rowAt);
-    int2 *bins = (int2 *)(sm + L.bins);
-    uint32_t *X = (uint32_t *)(sm + L.X);
-
-    // 1. value range of Y. (Written with min and max, not min(-y): nvcc 12.9 miscompiled the
-    //    unrolled "mx = min(mx, -y)" into a 3-input min that dropped one negation.)
-    int mn = INT_MAX, mx = INT_MIN;
-    for (int j = tid; j < m; j += NT) { int y = Ys[j]; mn = min(mn, y); mx = max(mx, y); }
     mn = warp_min_i(mn); mx = warp_max_i(mx);
     if (lane == 0) { ps.red[warp] = mn; ps.red[NWARP + warp] = mx; }
     __syncthreads();
@@ -195,158 +197,225 @@ __device__ void build_plan(const DevInst &I, unsigned char *sm, const Smem &L, P
         int a = lane < NWARP ? ps.red[lane] : INT_MAX, b = lane < NWARP ? ps.red[NWARP + lane] : INT_MIN;
         a = warp_min_i(a); b = warp_max_i(b);
         if (lane == 0) {
-            int U = (b - a) / 2 + 1;
-            ps.vmin = a;
-            ps.Upad = (U + 1) & ~1;
+            ps.vlo = a;
+            ps.Uc = (b - a) / 2 + 1;
         }
     }
+}
+
+// ------------------------------------------------------------------------------------------
+// Plan: per-iteration shared-memory structures of the current state (Y, V). Requires cnt[] = 0
+// and a lattice ps.vlo / Uc covering every Y (the exact range after load_state, or the previous
+// plan's range widened by 2k after a move: |Y'_j - Y_j| <= 2k). The exact range is found here.
+//   cnt/cur   rows per conservative lattice point (Y = vlo + 2u)
+//   seg       start of segment u - ufirst in sorted-row order (exact lattice, Y = vmin + 2u)
+//   pieces    (mask, fin | len << 16): the part of one segment inside one 32-row word, in row
+//             order; fin > 0 on a segment's last piece = number of bins finalised after it
+//             (1 + the empty lattice points that follow, or + the 2K trailing bins)
+//   pstart    first piece of each row word
+//   bins      (H_b, w_b) of bin beta <-> b = vmin + 2(beta - K): w_b = 60|b| - 1 for b < 0
+//   X[w][c]   sign bits x_jc = [A_jc V_c = -1] of sorted rows 32w..32w+31, column c
+// Leaves cnt[] zeroed, ps.key / gkey = KEY_NONE and ps.vlo / Uc set for the next plan.
+// ------------------------------------------------------------------------------------------
+template <int K>
+__device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps)
+{
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int m = I.m, n = I.n, W = I.W, NWn = I.NWn;
+    const int *Ys = (const int *)(sm + L.Y);
+    const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
+    const int *Hs = (const int *)(sm + L.H);
+    int *cnt = (int *)(sm + L.cnt);
+    int *seg = (int *)(sm + L.seg);
+    int *cur = (int *)(sm + L.cur);
+    int *pofs = (int *)(sm + L.pofs);
+    int *rowAt = (int *)(sm + L.rowAt);
+    int2 *bins = (int2 *)(sm + L.bins);
+    uint2 *pieces = (uint2 *)(sm + L.pieces);
+    int *pstart = (int *)(sm + L.pstart);
+    uint32_t *X = (uint32_t *)(sm + L.X);
+    const int vlo = ps.vlo, Uc = ps.Uc;
+
+    // A. counting sort over the conservative lattice
+    for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
     __syncthreads();
-    const int vmin = ps.vmin, Upad = ps.Upad, NB = Upad + 2 * K;
-    // 2. counting sort over the lattice u = (y - vmin)/2
-    for (int u = tid; u <= Upad; u += NT) seg[u] = 0;
-    __syncthreads();
-    for (int j = tid; j < m; j += NT) atomicAdd(&seg[(Ys[j] - vmin) >> 1], 1);
-    // bins: bin beta <-> value b = vmin + 2(beta - K); cost(h) = |h - Hb| + wb h
-    int hsum = 0;
-    for (int beta = tid; beta < NB; beta += NT) {
-        int b = vmin + 2 * (beta - K);
-        int2 bn;
-        if (b < 0) bn = make_int2(0, 60 * (-b) - 1);     // 30 (|y| - y) = 60 |y| for y < 0
-        else if (b <= n) { bn = make_int2(Hs[b], 0); hsum += Hs[b]; }
-        else bn = make_int2(0, 0);
-        bins[beta] = bn;
-    }
-    hsum = warp_sum_i(hsum);
-    if (lane == 0) ps.red[warp] = hsum;
-    __syncthreads();
-    // 3. exclusive scan of the counts (warp 0), base = m - (H mass inside the bin window)
+    PH(0);
+    // B. warp 0: exact range (first / last non-empty point), exclusive scans of the row and piece
+    //    offsets over it, and the lattice of the next plan
     if (warp == 0) {
-        int run = 0;
-        for (int b0 = 0; b0 <= Upad; b0 += 32) {
-            int u = b0 + lane;
-            int v = (u < Upad) ? seg[u] : 0;
+        int uf = -1, ul = -1;
+        for (int b0 = 0; b0 < Uc; b0 += 32) {
+            const unsigned bal = __ballot_sync(FULL, b0 + lane < Uc && cnt[b0 + lane] > 0);
+            if (bal) {
+                if (uf < 0) uf = b0 + __ffs(bal) - 1;
+                ul = b0 + 31 - __clz(bal);
+            }
+        }
+        const int U = ul - uf + 1;
+        int runr = 0, runp = 0;
+        for (int b0 = 0; b0 < U; b0 += 32) {
+            const int v_ = b0 + lane;
+            const int u = uf + v_;
+            const int v = v_ < U ? cnt[u] : 0;
             int inc = v;
             for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, inc, o); if (lane >= o) inc += t; }
-            if (u <= Upad) { seg[u] = run + inc - v; cur[u] = run + inc - v; }
-            run += __shfl_sync(FULL, inc, 31);
+            const int st = runr + inc - v, en = runr + inc;
+            const int np = v > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : 0;
+            int incp = np;
+            for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, incp, o); if (lane >= o) incp += t; }
+            if (v_ < U) { seg[v_] = st; cur[u] = st; pofs[v_] = runp + incp - np; }
+            runr += __shfl_sync(FULL, inc, 31);
+            runp += __shfl_sync(FULL, incp, 31);
         }
-        int hs = lane < NWARP ? ps.red[lane] : 0;
-        hs = warp_sum_i(hs);
-        if (lane == 0) ps.base = m - hs;
+        if (lane == 0) {
+            const int vmin = vlo + 2 * uf;
+            seg[U] = runr; ps.P = runp; pstart[W] = runp;
+            ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
+            ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
+            ps.key = (unsigned long long)KEY_NONE;
+            ps.gkey = (unsigned long long)KEY_NONE;
+        }
     }
     __syncthreads();
-    // 4. place rows
+    PH(1);
+    // C. place rows; emit pieces (one thread per segment); bin constants
+    const int vmin = ps.vmin, U = ps.U, NB = ps.NB, uf = ps.ufirst;
     for (int j = tid; j < m; j += NT) {
-        int p = atomicAdd(&cur[(Ys[j] - vmin) >> 1], 1);
+        const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
         rowAt[p] = j;
     }
-    __syncthreads();
-    // 5. X[w][c] = bits x_{rowAt[32w+l], c} (x = 1 <=> A_jc V_c = -1), one warp per row word
-    for (int w = warp; w < I.W; w += NWARP) {
-        int p = 32 * w + lane;
-        bool valid = p < m;
-        const uint32_t *ar = I.Arow + (size_t)(valid ? rowAt[p] : 0) * I.NWn;
-        for (int cw = 0; cw < I.NWn; cw++) {
-            uint32_t word = valid ? (__ldg(ar + cw) ^ vbs[cw]) : 0u;
-            uint32_t mine = 0;
-#pragma unroll
-            for (int cc = 0; cc < 32; cc++) {
-                uint32_t bal = __ballot_sync(FULL, (word >> cc) & 1u);
-                if (lane == cc) mine = bal;
-            }
-            int c = 32 * cw + lane;
-            if (c < n) X[w * n + c] = mine;
+    for (int v = tid; v < U; v += NT) {
+        if (cnt[uf + v] == 0) continue;
+        const int st = seg[v], en = seg[v + 1];
+        const int w0 = st >> 5, w1 = (en - 1) >> 5;
+        int q = v + 1;
+        while (q < U && cnt[uf + q] == 0) q++;
+        const int fin_last = (q >= U ? NB : q) - v;
+        int p = pofs[v];
+        for (int w = w0; w <= w1; w++, p++) {
+            const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
+            const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
+            pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? fin_last : 0) | ((uint32_t)(en - st) << 16));
+            if (w > w0 || (st & 31) == 0) pstart[w] = p;
         }
     }
+    for (int beta = tid; beta < NB; beta += NT) {
+        const int b = vmin + 2 * (beta - K);
+        bins[beta] = make_int2((b >= 0 && b <= n) ? Hs[b] : 0, b < 0 ? 60 * (-b) - 1 : 0);
+    }
     __syncthreads();
+    PH(2);
+    // D. X[w][c]: per (row word, column word) pair, lane l loads sorted row 32w+l's sign bits of
+    //    columns 32cw..32cw+31 and a 5-round shuffle transpose turns rows into columns; zero cnt[]
+    for (int u = tid; u < Uc; u += NT) cnt[u] = 0;
+    for (int pr = warp; pr < W * NWn; pr += NWARP) {
+        const int w = pr / NWn, cw = pr - w * NWn;
+        const int p = 32 * w + lane;
+        uint32_t x = p < m ? (Ar[(size_t)rowAt[p] * NWn + cw] ^ vbs[cw]) : 0u;
+#pragma unroll
+        for (int j = 16; j >= 1; j >>= 1) {
+            const uint32_t mk = j == 16 ? 0x0000FFFFu : j == 8 ? 0x00FF00FFu : j == 4 ? 0x0F0F0F0Fu
+                              : j == 2 ? 0x33333333u : 0x55555555u;
+            const uint32_t y = __shfl_xor_sync(FULL, x, j);
+            x = (lane & j) ? ((x & ~mk) | ((y & ~mk) >> j)) : ((x & mk) | ((y & mk) << j));
+        }
+        const int c = 32 * cw + lane;
+        if (c < n) X[w * n + c] = x;
+    }
+    __syncthreads();
+    PH(3);
 }
 
-// Fitness of neighbour (a, b, c) from the plan (exact; see file header).
+// Fitness of neighbour (a, b, c) from the plan, word-major: the lane's columns of one row word
+// are loaded once, bit-sliced into t = #flipped "-1" entries (lo, hi planes), and every piece of
+// that word adds its POPC counts. On a segment's last piece its row counts N_t (t = 0..k) are
+// known; they land in bins beta + 2t, and a 2k-long shift register finalises one bin per segment.
+//   f = 2m + sum_beta ( w_beta h_beta - 2 min(h_beta, H_beta) )
+// (|h - H| = h + H - 2 min(h, H) summed over b = 0..n; every row lands in exactly one bin.)
 template <int K>
-__device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const int *__restrict__ seg,
-                                        const int2 *__restrict__ bins, int n, int Upad, int base,
-                                        int a, int b, int c)
+__device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
+                                        const int *__restrict__ pstart, const int2 *__restrict__ bins,
+                                        int n, int W, int m2, int a, int b, int c)
 {
-    int f = base;
-    int ce[K], co[K];
+    int f = m2, smin = 0;
+    int R[2 * K];
 #pragma unroll
-    for (int q = 0; q < K; q++) { ce[q] = 0; co[q] = 0; }
-    int st = seg[0];
-    for (int u = 0; u < Upad + 2 * K; u += 2) {
+    for (int i = 0; i < 2 * K; i++) R[i] = 0;
+    int c1 = 0, c2 = 0, c3 = 0;
+    int beta = 0, p = 0;
+    for (int w = 0; w < W; w++) {
+        const uint32_t *xr = X + w * n;
+        uint32_t lo, hi = 0, lh = 0;
+        if (K == 1) {
+            lo = xr[a];
+        } else if (K == 2) {
+            const uint32_t xa = xr[a], xb = xr[b];
+            lo = xa ^ xb; hi = xa & xb;
+        } else {
+            const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+            lo = xa ^ xb ^ xc;
+            hi = (xa & xb) | (xc & (xa ^ xb));
+            lh = lo & hi;
+        }
+        const int pend = pstart[w + 1];
+        for (; p < pend; p++) {
+            const uint2 rec = pieces[p];
+            c1 += __popc(lo & rec.x);
+            if (K >= 2) c2 += __popc(hi & rec.x);
+            if (K == 3) c3 += __popc(lh & rec.x);
+            const int fin = rec.y & 0xffffu;
+            if (fin) {
+                const int len = rec.y >> 16;
+                int N[K + 1];
+                if (K == 1) { N[1] = c1; N[0] = len - c1; }
+                else if (K == 2) { N[2] = c2; N[1] = c1; N[0] = len - c1 - c2; }
+                else { N[3] = c3; N[2] = c2 - c3; N[1] = c1 - c3; N[0] = len - c1 - c2 + c3; }
+                int h = R[0] + N[0];
 #pragma unroll
-        for (int par = 0; par < 2; par++) {
-            const int uu = u + par;
-            int en = (uu < Upad) ? seg[uu + 1] : st;
-            int c1 = 0, c2 = 0, c3 = 0;
-            if (st < en) {
-                const int w0 = st >> 5, w1 = (en - 1) >> 5;
-                for (int w = w0; w <= w1; w++) {
-                    uint32_t mask = FULL;
-                    if (w == w0) mask &= FULL << (st & 31);
-                    if (w == w1) mask &= FULL >> (31 - ((en - 1) & 31));
-                    const uint32_t *xr = X + w * n;
-                    uint32_t xa = xr[a];
-                    if (K == 1) {
-                        c1 += __popc(xa & mask);
-                    } else if (K == 2) {
-                        uint32_t xb = xr[b];
-                        c1 += __popc((xa ^ xb) & mask);
-                        c2 += __popc((xa & xb) & mask);
-                    } else {
-                        uint32_t xb = xr[b], xc = xr[c];
-                        uint32_t lo = xa ^ xb ^ xc;
-                        uint32_t hi = (xa & xb) | (xc & (xa ^ xb));
-                        c1 += __popc(lo & mask);
-                        c2 += __popc(hi & mask);
-                        c3 += __popc(lo & hi & mask);
-                    }
+                for (int i = 0; i < 2 * K - 1; i++) R[i] = (i & 1) ? R[i + 1] + N[(i + 1) >> 1] : R[i + 1];
+                R[2 * K - 1] = N[K];
+                int2 bn = bins[beta++];
+                f += bn.y * h;
+                smin += min(h, bn.x);
+                c1 = 0; c2 = 0; c3 = 0;
+                for (int e = 1; e < fin; e++) {
+                    h = R[0];
+#pragma unroll
+                    for (int i = 0; i < 2 * K - 1; i++) R[i] = R[i + 1];
+                    R[2 * K - 1] = 0;
+                    bn = bins[beta++];
+                    f += bn.y * h;
+                    smin += min(h, bn.x);
                 }
             }
-            // N_t = rows of this segment with t flipped "-1" entries; they land in bin uu + 2t
-            int N[K + 1];
-            const int len = en - st;
-            if (K == 1) { N[1] = c1; N[0] = len - c1; }
-            else if (K == 2) { N[2] = c2; N[1] = c1; N[0] = len - c1 - c2; }
-            else { N[3] = c3; N[2] = c2 - c3; N[1] = c1 - c3; N[0] = len - c1 - c2 + c3; }
-            int h;
-            int *ch = par ? co : ce;
-            h = ch[0] + N[0];
-#pragma unroll
-            for (int q = 0; q < K - 1; q++) ch[q] = ch[q + 1] + N[q + 1];
-            ch[K - 1] = N[K];
-            const int2 bn = bins[uu];
-            f += abs(h - bn.x) + bn.y * h;
-            st = en;
         }
     }
-    return f;
+    return f - 2 * smin;
 }
 
-__device__ __forceinline__ uint32_t ldcg_u32(const uint32_t *p) { return __ldcg(p); }
-
-// Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA; returns this thread's best key.
+// Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
+// key. until (nullable) is indexed by r - ubase: rank r is tabu iff until[r - ubase] >= t.
 template <int K, bool WRITE_ALL>
 __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
-                                         const PlanScalars &ps, uint32_t M, uint32_t blo, uint32_t bhi,
-                                         const uint32_t *tabu, int32_t *fit_out)
+                                         uint32_t M, uint32_t blo, uint32_t bhi, const uint32_t *until,
+                                         uint32_t ubase, uint32_t t, int32_t *fit_out)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
-    const int *seg = (const int *)(sm + L.seg);
+    const uint2 *pieces = (const uint2 *)(sm + L.pieces);
+    const int *pstart = (const int *)(sm + L.pstart);
     const int2 *bins = (const int2 *)(sm + L.bins);
-    const int Upad = ps.Upad, base = ps.base;
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
         if (r < bhi) {
-            bool is_tabu = false;
-            if (tabu) is_tabu = (ldcg_u32(tabu + (r >> 5)) >> (r & 31)) & 1u;
+            const bool is_tabu = until && until[r - ubase] >= t;
             if (!is_tabu || WRITE_ALL) {
                 int a, b, c;
                 unrank<K>(r, I.n, M, a, b, c);
-                int f = eval_fit<K>(X, seg, bins, I.n, Upad, base, a, b, c);
+                const int f = eval_fit<K>(X, pieces, pstart, bins, I.n, I.W, 2 * I.m, a, b, c);
                 if (WRITE_ALL) fit_out[r] = f;
-                unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
+                const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 if (!is_tabu && key < best) best = key;
             }
         }
@@ -355,15 +424,16 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
 }
 
 // Apply the move F to the CTA's shared copy of (Y, V): Y'_j = Y_j - 2 sum_{i in F} B_ji,
-// B_ji = V_i A_ji, then flip the bits of V.
+// B_ji = V_i A_ji, then flip the bits of V. The flip is ordered before the
+// next reads of V (plan step D) by the plan's own barriers.
 template <int K>
-__device__ void apply_move(const DevInst &I, int *Ys, uint32_t *vbs, int a, int b, int c)
+__device__ void apply_move(const DevInst &I, const uint32_t *Ar, int *Ys, uint32_t *vbs, int a, int b, int c)
 {
     for (int j = threadIdx.x; j < I.m; j += NT) {
-        const uint32_t *ar = I.Arow + (size_t)j * I.NWn;
-        int d = (((__ldg(ar + (a >> 5)) ^ vbs[a >> 5]) >> (a & 31)) & 1u) ? -1 : 1;
-        if (K >= 2) d += (((__ldg(ar + (b >> 5)) ^ vbs[b >> 5]) >> (b & 31)) & 1u) ? -1 : 1;
-        if (K == 3) d += (((__ldg(ar + (c >> 5)) ^ vbs[c >> 5]) >> (c & 31)) & 1u) ? -1 : 1;
+        const uint32_t *ar = Ar + (size_t)j * I.NWn;
+        int d = (((ar[a >> 5] ^ vbs[a >> 5]) >> (a & 31)) & 1u) ? -1 : 1;
+        if (K >= 2) d += (((ar[b >> 5] ^ vbs[b >> 5]) >> (b & 31)) & 1u) ? -1 : 1;
+        if (K == 3) d += (((ar[c >> 5] ^ vbs[c >> 5]) >> (c & 31)) & 1u) ? -1 : 1;
         Ys[j] -= 2 * d;
     }
     __syncthreads();
@@ -372,27 +442,6 @@ __device__ void apply_move(const DevInst &I, int *Ys, uint32_t *vbs, int a, int 
         if (K >= 2) vbs[b >> 5] ^= 1u << (b & 31);
         if (K == 3) vbs[c >> 5] ^= 1u << (c & 31);
     }
-    __syncthreads();
-}
-
-__device__ __forceinline__ void grid_barrier(unsigned *bar, unsigned nblocks)
-{
-    __syncthreads();
-    if (threadIdx.x == 0) {
-        volatile unsigned *gen = bar + 1;
-        unsigned g = *gen;
-        __threadfence();
-        unsigned arrived = atomicAdd(bar, 1u);
-        if (arrived == nblocks - 1) {
-            atomicExch(bar, 0u);
-            __threadfence();
-            atomicAdd(bar + 1, 1u);
-        } else {
-            while (*gen == g) { }
-        }
-        __threadfence();
-    }
-    __syncthreads();
 }
 
 // Slice [blo, bhi) of CTA `b` of `nb` inside [lo, hi), boundaries on multiples of 32.
@@ -403,15 +452,34 @@ __device__ __forceinline__ void cta_slice(uint32_t lo, uint32_t hi, unsigned b, 
     bhi = (b + 1 == nb) ? hi : lo + 32u * (uint32_t)((span * (b + 1) / nb) / 32);
 }
 
-__device__ void load_state(const SearchArgs &A, unsigned char *sm, const Smem &L)
+// Stage the state (and A's bits when A.a_in_smem) into shared memory, zero cnt[] and publish the
+// range of Y; returns A's bit rows.
+template <int K>
+__device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, const Smem &L, PlanScalars &ps)
 {
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
     int *Hs = (int *)(sm + L.H);
-    for (int j = threadIdx.x; j < A.I.m; j += NT) Ys[j] = A.Y[j];
+    int *cnt = (int *)(sm + L.cnt);
+    int mn = INT_MAX, mx = INT_MIN;
+    for (int j = threadIdx.x; j < A.I.m; j += NT) {
+        const int y = A.Y[j];
+        Ys[j] = y;
+        mn = min(mn, y); mx = max(mx, y);
+    }
     for (int w = threadIdx.x; w < A.I.NWn; w += NT) vbs[w] = A.vb[w];
     for (int b = threadIdx.x; b <= A.I.n; b += NT) Hs[b] = A.I.H[b];
+    for (int u = threadIdx.x; u < A.I.n + 2 + 2 * K; u += NT) cnt[u] = 0;
+    const uint32_t *Ar = A.I.Arow;
+    if (A.a_in_smem) {
+        uint32_t *As = (uint32_t *)(sm + L.Ar);
+        const int nw = A.I.m * A.I.NWn;
+        for (int q = threadIdx.x; q < nw; q += NT) As[q] = __ldg(A.I.Arow + q);
+        Ar = As;
+    }
+    range_publish<K>(mn, mx, ps);
     __syncthreads();
+    return Ar;
 }
 
 // ------------------------------------------------------------------------------------------
@@ -424,49 +492,46 @@ __global__ void __launch_bounds__(NT) k_init(DevInst I, const int8_t *V0, uint32
                                              const int32_t *Ycheck, int64_t *fs)
 {
     __shared__ int hist[4096 + 1];
-    __shared__ int s_bad;
-    __shared__ long long s_pen;
+    __shared__ int s_bad, s_hd;
+    __shared__ unsigned long long s_pen;
     const int tid = threadIdx.x;
-    if (tid == 0) { s_bad = 0; s_pen = 0; }
+    if (tid == 0) { s_bad = 0; s_pen = 0; s_hd = 0; }
+    for (int b = tid; b <= I.n; b += NT) hist[b] = 0;
+    __syncthreads();
     for (int w = tid; w < I.NWn; w += NT) {
         uint32_t word = 0;
         for (int q = 0; q < 32; q++) {
-            int i = 32 * w + q;
+            const int i = 32 * w + q;
             if (i < I.n) {
-                int8_t v = V0[i];
+                const int8_t v = V0[i];
                 if (v != 1 && v != -1) s_bad = 1;
                 if (v < 0) word |= 1u << q;
             }
         }
         vb[w] = word;
     }
-    const bool use_hist = I.n <= 4096;
-    for (int b = tid; b <= I.n && use_hist; b += NT) hist[b] = 0;
     __syncthreads();
-    long long pen = 0;
+    unsigned long long pen = 0;
     for (int j = tid; j < I.m; j += NT) {
         const uint32_t *ar = I.Arow + (size_t)j * I.NWn;
         int d = 0;
         for (int w = 0; w < I.NWn; w++) d += __popc(__ldg(ar + w) ^ vb[w]);
-        int y = I.n - 2 * d;  // <a_j, v> = n - 2 popcount(a xor v)
+        const int y = I.n - 2 * d;  // <a_j, v> = n - 2 popcount(a xor v)
         Y[j] = y;
         if (Ycheck && Ycheck[j] != y) s_bad = 1;
-        if (y < 0) pen += -2 * (long long)y;
-        if (y >= 0 && y <= I.n && use_hist) atomicAdd(&hist[y], 1);
+        if (y < 0) pen += (unsigned long long)(-2 * y);
+        if (y >= 0) atomicAdd(&hist[y], 1);
     }
-    atomicAdd((unsigned long long *)&s_pen, (unsigned long long)pen);
+    atomicAdd(&s_pen, pen);
     __syncthreads();
     int hd = 0;
-    for (int b = tid; b <= I.n && use_hist; b += NT) hd += abs(I.H[b] - hist[b]);
-    __shared__ int s_hd;
-    if (tid == 0) s_hd = 0;
-    __syncthreads();
+    for (int b = tid; b <= I.n; b += NT) hd += abs(I.H[b] - hist[b]);
     atomicAdd(&s_hd, hd);
     __syncthreads();
     if (tid == 0) {
-        int64_t f = 30 * (int64_t)s_pen + s_hd;
+        const int64_t f = 30 * (int64_t)s_pen + s_hd;
         fs[FS_F] = f; fs[FS_T] = 0; fs[FS_BEST] = f; fs[FS_BESTIT] = 0;
-        fs[FS_ZERO] = (f == 0) ? 0 : -1; fs[FS_DONE] = 0; fs[FS_ERR] = (s_bad || !use_hist) ? 1 : 0;
+        fs[FS_ZERO] = (f == 0) ? 0 : -1; fs[FS_DONE] = 0; fs[FS_ERR] = s_bad ? 1 : 0;
     }
 }
 
@@ -476,14 +541,27 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
-    const unsigned nb = gridDim.x, bid = blockIdx.x;
+    const int nb = (int)gridDim.x, bid = (int)blockIdx.x;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const bool leader = (bid == 0 && threadIdx.x == 0);
-    load_state(A, sm, L);
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, bid, nb, blo, bhi);
+    // the CTA's until[] slice: shared-memory copy when it fits, else the global array
+    uint32_t *until = A.until;
+    uint32_t ubase = 0;
+    if (A.until_smem) {
+        uint32_t *us = (uint32_t *)(sm + L.a_end);
+        for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) us[r - blo] = A.until[r];
+        until = us;
+        ubase = blo;
+    }
+    const uint32_t *Ar = load_state<K>(A, sm, L, ps);
+#ifdef LNS_PHASE_TIMING
+    if (threadIdx.x == 0) { for (int i = 0; i < NPH; i++) s_ph[i] = 0; s_last = clock64(); }
+#endif
     int64_t f = A.fs[FS_F];
     int64_t best_f = A.fs[FS_BEST], best_it = A.fs[FS_BESTIT], zero_it = A.fs[FS_ZERO];
     const int64_t t0 = A.fs[FS_T];
@@ -491,38 +569,55 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     bool failed = false;
     for (; t <= t0 + A.iters; t++) {
         if (A.stop_on_zero && f == 0) break;
-        build_plan<K>(A.I, sm, L, ps);
-        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, A.L > 0 ? A.tabu : nullptr, nullptr);
-        unsigned long long bk = block_min_key(mine, ps);
-        if (threadIdx.x == 0 && bk != (unsigned long long)KEY_NONE)
-            atomicMin((unsigned long long *)&A.keys[t % 3], bk);
-        grid_barrier(A.bar, nb);
-        if (threadIdx.x == 0) ps.key = (int64_t)__ldcg((const unsigned long long *)&A.keys[t % 3]);
-        if (leader) A.keys[(t + 2) % 3] = KEY_NONE;
+        build_plan<K>(A.I, Ar, sm, L, ps);
+        unsigned long long mine = eval_range<K, false>(A.I, sm, L, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr);
+        mine = warp_min_k(mine);
+        if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
         __syncthreads();
-        const int64_t key = ps.key;
-        if (key == KEY_NONE) { failed = true; break; }
-        const uint32_t r = (uint32_t)(key & 0xffffffffu);
-        f = key >> 32;
-        int a, b, c;
-        unrank<K>(r, A.I.n, A.M, a, b, c);
-        apply_move<K>(A.I, Ys, vbs, a, b, c);
-        if (threadIdx.x == 0 && A.L > 0) {
-            const int64_t R1 = A.L + 1;
-            if (t > A.L) {
-                uint32_t old = __ldcg(&A.ring[(t - A.L) % R1]);
-                if (old >= blo && old < bhi) atomicAnd(&A.tabu[old >> 5], ~(1u << (old & 31)));
+        PH(4);
+        unsigned long long key = ps.key;
+        if (nb > 1) {
+            // exchange: u64 MIN of this CTA's key into slot t%3 (each slot on its own 128-B line),
+            // then one arrival on a monotonic 64-bit counter; when the counter reaches
+            // nb * (t - t0) every CTA's MIN has landed and the slot holds the global minimum.
+            // Slot (t+2)%3 was last read in iteration t-1 by CTAs that have all arrived at t, so
+            // CTA 0 resets it here for iteration t+2.
+            if (threadIdx.x == 0) {
+                unsigned long long *slot = (unsigned long long *)A.slots + 16 * (t % 3);
+                if (key != (unsigned long long)KEY_NONE) atomicMin(slot, key);
+                __threadfence();
+                atomicAdd((unsigned long long *)A.slots + 48, 1ull);
+                const unsigned long long target = (unsigned long long)nb * (unsigned long long)(t - t0);
+                volatile unsigned long long *ctr = (volatile unsigned long long *)A.slots + 48;
+                while (*ctr < target) { }
+                ps.gkey = *(volatile unsigned long long *)slot;
+                if (bid == 0) *((volatile unsigned long long *)A.slots + 16 * ((t + 2) % 3)) = (unsigned long long)KEY_NONE;
             }
-            if (r >= blo && r < bhi) atomicOr(&A.tabu[r >> 5], 1u << (r & 31));
-            if (bid == 0) { A.ring[t % R1] = r; __threadfence(); }
+            __syncthreads();
+            key = ps.gkey;
         }
+        PH(5);
+        if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
+        const uint32_t r = (uint32_t)(key & 0xffffffffu);
+        f = (int64_t)(key >> 32);
+        if (threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
         if (leader) {
             if (A.trace_r) A.trace_r[t - 1] = r;
             if (A.trace_f) A.trace_f[t - 1] = f;
             if (f < best_f) { best_f = f; best_it = t; }
             if (f == 0 && zero_it < 0) zero_it = t;
         }
+        int a, b, c;
+        unrank<K>(r, A.I.n, A.M, a, b, c);
+        apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
+        PH(6);
     }
+#ifdef LNS_PHASE_TIMING
+    if (threadIdx.x == 0)
+        for (int i = 0; i < NPH; i++) atomicAdd(&g_ph[i], (unsigned long long)s_ph[i]);
+#endif
+    if (A.until_smem)
+        for (uint32_t q = blo + threadIdx.x; q < bhi; q += NT) A.until[q] = until[q - ubase];
     if (bid == 0) {
         for (int j = threadIdx.x; j < A.I.m; j += NT) A.Y[j] = Ys[j];
         for (int w = threadIdx.x; w < A.I.NWn; w += NT) A.vb[w] = vbs[w];
@@ -534,34 +629,36 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     }
 }
 
-// Stepped mode, evaluation: partial best key of this device's slice into key_out[0].
-// The last CTA to finish publishes the accumulator and resets it (no extra launch).
+// Stepped mode, evaluation of iteration t = fs[FS_T] + 1: partial best key of this device's slice
+// into key_out[0]. The last CTA to finish publishes the accumulator and resets it (no extra launch).
 template <int K, bool WRITE_ALL>
 __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_out, int32_t *fit_out)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    __shared__ bool s_last;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
+    const int lane = threadIdx.x & 31;
     if (!WRITE_ALL && A.fs[FS_DONE]) {
         if (blockIdx.x == 0 && threadIdx.x == 0) *key_out = KEY_NONE;
         return;
     }
-    load_state(A, sm, L);
+    const uint32_t *Ar = load_state<K>(A, sm, L, ps);
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, blockIdx.x, gridDim.x, blo, bhi);
-    build_plan<K>(A.I, sm, L, ps);
-    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps, A.M, blo, bhi, A.tabu, fit_out);
-    unsigned long long bk = block_min_key(mine, ps);
+    build_plan<K>(A.I, Ar, sm, L, ps);
+    const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
+    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, A.M, blo, bhi, A.until, 0, t, fit_out);
+    mine = warp_min_k(mine);
+    if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
+    __syncthreads();
     if (threadIdx.x == 0) {
-        if (bk != (unsigned long long)KEY_NONE) atomicMin((unsigned long long *)A.keys, bk);
+        if (ps.key != (unsigned long long)KEY_NONE) atomicMin((unsigned long long *)A.slots, ps.key);
         __threadfence();
-        unsigned done = atomicAdd(A.bar, 1u);
-        s_last = (done == gridDim.x - 1);
-        if (s_last) {
+        const unsigned done = atomicAdd(A.counter, 1u);
+        if (done == gridDim.x - 1) {
             __threadfence();
-            *key_out = (int64_t)atomicExch((unsigned long long *)A.keys, (unsigned long long)KEY_NONE);
-            A.bar[0] = 0;
+            *key_out = (int64_t)atomicExch((unsigned long long *)A.slots, (unsigned long long)KEY_NONE);
+            *A.counter = 0;
         }
     }
 }
@@ -596,15 +693,7 @@ __global__ void __launch_bounds__(NT) k_step_apply(SearchArgs A, const int64_t *
         A.vb[a >> 5] ^= 1u << (a & 31);
         if (K >= 2) A.vb[b >> 5] ^= 1u << (b & 31);
         if (K == 3) A.vb[c >> 5] ^= 1u << (c & 31);
-        if (A.L > 0) {
-            const int64_t R1 = A.L + 1;
-            if (t > A.L) {
-                uint32_t old = A.ring[(t - A.L) % R1];
-                if (old >= A.lo && old < A.hi) A.tabu[old >> 5] &= ~(1u << (old & 31));
-            }
-            if (r >= A.lo && r < A.hi) A.tabu[r >> 5] |= 1u << (r & 31);
-            A.ring[t % R1] = r;
-        }
+        if (r >= A.lo && r < A.hi) A.until[r] = (uint32_t)(t + A.L);
         if (A.trace_r) A.trace_r[t - 1] = r;
         if (A.trace_f) A.trace_f[t - 1] = f;
         A.fs[FS_F] = f; A.fs[FS_T] = t;
@@ -614,24 +703,28 @@ __global__ void __launch_bounds__(NT) k_step_apply(SearchArgs A, const int64_t *
     }
 }
 
-// Debug: dump the plan of the current state (one CTA): [vmin, Upad, base, H[0..n], seg[0..Upad], bins.x, bins.y]
+// Debug: dump the plan of the current state (one CTA):
+// [vmin, U, NB, P, seg[0..U], bins (NB x {H, w}), pieces (P x {mask, meta}), pstart[0..W]]
 template <int K>
 __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K);
-    load_state(A, sm, L);
-    build_plan<K>(A.I, sm, L, ps);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
+    const uint32_t *Ar = load_state<K>(A, sm, L, ps);
+    const int *segp = (const int *)(sm + L.seg);
+    build_plan<K>(A.I, Ar, sm, L, ps);
+    const int U = ps.U;
     if (threadIdx.x == 0) {
-        const int *Hs = (const int *)(sm + L.H);
-        const int *seg = (const int *)(sm + L.seg);
         const int2 *bins = (const int2 *)(sm + L.bins);
+        const uint2 *pieces = (const uint2 *)(sm + L.pieces);
+        const int *pstart = (const int *)(sm + L.pstart);
         int o = 0;
-        out[o++] = ps.vmin; out[o++] = ps.Upad; out[o++] = ps.base;
-        for (int b = 0; b <= A.I.n; b++) out[o++] = Hs[b];
-        for (int u = 0; u <= ps.Upad; u++) out[o++] = seg[u];
-        for (int q = 0; q < ps.Upad + 2 * K; q++) { out[o++] = bins[q].x; out[o++] = bins[q].y; }
+        out[o++] = ps.vmin; out[o++] = U; out[o++] = ps.NB; out[o++] = ps.P;
+        for (int u = 0; u <= U; u++) out[o++] = segp[u];
+        for (int q = 0; q < ps.NB; q++) { out[o++] = bins[q].x; out[o++] = bins[q].y; }
+        for (int q = 0; q < ps.P; q++) { out[o++] = (int)pieces[q].x; out[o++] = (int)pieces[q].y; }
+        for (int w = 0; w <= A.I.W; w++) out[o++] = pstart[w];
     }
 }
 
@@ -639,7 +732,7 @@ template <int K>
 __global__ void k_unrank(int n, uint32_t M, const int64_t *ranks, int64_t count, int32_t *out, int32_t *bad)
 {
     for (int64_t q = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; q < count; q += (int64_t)gridDim.x * blockDim.x) {
-        int64_t r = ranks[q];
+        const int64_t r = ranks[q];
         if (r < 0 || r >= (int64_t)M) { *bad = 1; out[3 * q] = out[3 * q + 1] = out[3 * q + 2] = -1; continue; }
         int a, b, c;
         unrank<K>((uint32_t)r, n, M, a, b, c);
@@ -650,6 +743,13 @@ __global__ void k_unrank(int n, uint32_t M, const int64_t *ranks, int64_t count,
 __global__ void k_fill_i64(int64_t *p, int64_t v, int64_t cnt)
 {
     for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < cnt; i += (int64_t)gridDim.x * blockDim.x) p[i] = v;
+}
+
+// until[r] = bit r of the caller's tabu bitmap (tabu at t = 1 <=> until >= 1).
+__global__ void k_bits_to_until(const uint32_t *bits, uint32_t *until, uint32_t M)
+{
+    for (uint32_t r = blockIdx.x * blockDim.x + threadIdx.x; r < M; r += gridDim.x * blockDim.x)
+        until[r] = bits ? (bits[r >> 5] >> (r & 31)) & 1u : 0u;
 }
 
 }  // namespace
@@ -673,12 +773,12 @@ struct lns_ctx {
     uint32_t *d_vb = nullptr;
     int32_t *d_Y = nullptr;
     int64_t *d_fs = nullptr;
-    int64_t *d_keys = nullptr;  // 3 persistent slots + 1 stepped accumulator + 1 eval output
-    unsigned *d_bar = nullptr;  // [0..1] grid barrier, [2] stepped counter
+    int64_t *d_slots = nullptr;  // 3 x MAX_SLOTS persistent slots, then stepped accumulator, eval output
+    unsigned *d_counter = nullptr;
     int8_t *d_V = nullptr;
     int32_t *d_Yin = nullptr;
-    uint32_t *d_tabu = nullptr; size_t tabu_cap = 0;
-    uint32_t *d_ring = nullptr; size_t ring_cap = 0;
+    uint32_t *d_bits = nullptr; size_t bits_cap = 0;
+    uint32_t *d_until = nullptr; size_t until_cap = 0;
     int64_t *d_tr = nullptr, *d_tf = nullptr; size_t trace_cap = 0, trace_cap_f = 0;
     int32_t *d_fit = nullptr; size_t fit_cap = 0;
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
@@ -689,6 +789,10 @@ struct lns_ctx {
 };
 
 namespace {
+
+constexpr int SLOT_ACC = 3 * MAX_SLOTS;  // stepped accumulator
+constexpr int SLOT_OUT = 3 * MAX_SLOTS + 1;  // eval output key
+constexpr int SLOT_N = 3 * MAX_SLOTS + 2;
 
 struct DeviceGuard {
     int prev = -1;
@@ -753,52 +857,54 @@ void slice_of(uint32_t M, int part, int nparts, uint32_t &lo, uint32_t &hi)
     hi = B(part + 1);
 }
 
-template <int K>
-void set_smem_attr(size_t bytes)
-{
-    cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)bytes);
-    cudaFuncSetAttribute(k_step_eval<K, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)bytes);
-    cudaFuncSetAttribute(k_step_eval<K, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)bytes);
-}
+// Launch geometry of one search: k, shared-memory bytes, A staged or not, until cached or not.
+struct Geometry {
+    uint32_t M = 0;
+    int a_in_smem = 0;
+    size_t smem_eval = 0;  // bytes for the stepped / eval kernels
+};
 
-lns_status check_k(const lns_ctx *c, int k, uint32_t &M, size_t &smem)
+lns_status check_k(const lns_ctx *c, int k, Geometry &g)
 {
     if (!c) return fail(LNS_EINVAL, "null context");
     if (k < 1 || k > 3) return fail(LNS_EINVAL, "k must be 1, 2 or 3");
     if (c->n < k) return fail(LNS_EINVAL, "n < k");
-    int64_t Mk = comb_k(c->n, k);
+    const int64_t Mk = comb_k(c->n, k);
     if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
-    M = (uint32_t)Mk;
-    Smem L = smem_layout(c->m, c->n, c->W, c->NWn, k);
-    smem = (size_t)L.total;
-    if ((int)smem > c->smemOptin - (int)sizeof(PlanScalars) - 64) return fail(LNS_ERANGE, "bit-packed A does not fit in shared memory");
+    g.M = (uint32_t)Mk;
+    const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
+    const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1);
+    const Smem without = smem_layout(c->m, c->n, c->W, c->NWn, k, 0);
+    if (with.a_end <= budget) { g.a_in_smem = 1; g.smem_eval = (size_t)with.a_end; }
+    else if (without.a_end <= budget) { g.a_in_smem = 0; g.smem_eval = (size_t)without.a_end; }
+    else return fail(LNS_ERANGE, "bit-packed A does not fit in shared memory");
     return LNS_OK;
 }
 
-// Blocks per search for the persistent kernel.
 int search_blocks(const lns_ctx *c, uint32_t span, int occ)
 {
-    int cap = c->numSMs * occ;
+    const int cap = std::min(c->numSMs * occ, MAX_SLOTS);
     if (c->blocks_override > 0) return std::min(c->blocks_override, cap);
-    int nb = (int)std::min<int64_t>((int64_t)cap, std::max<int64_t>(1, span / 1024));
+    const int nb = (int)std::min<int64_t>((int64_t)cap, std::max<int64_t>(1, span / 1024));
     return std::max(1, nb);
 }
 
-SearchArgs make_args(lns_ctx *c, uint32_t M, int64_t iters, int64_t L, int flags)
+SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, int flags)
 {
     SearchArgs A;
     A.I = dev_inst(c);
-    A.M = M;
-    slice_of(M, c->part, c->nparts, A.lo, A.hi);
+    A.M = g.M;
+    slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
-    A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.tabu = c->d_tabu; A.ring = c->d_ring;
-    A.keys = c->d_keys; A.bar = c->d_bar; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
+    A.a_in_smem = g.a_in_smem;
+    A.until_smem = 0;
+    A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
+    A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     return A;
 }
 
-// Prepare a search: V0 -> state, tabu/ring/trace buffers cleared.
-lns_status search_setup(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L, uint64_t seed,
-                        const int8_t *V0, cudaStream_t st)
+// Prepare a search: V0 -> state, until[] cleared, trace buffers sized.
+lns_status search_setup(lns_ctx *c, const Geometry &g, int64_t iters, uint64_t seed, const int8_t *V0, cudaStream_t st)
 {
     lns_status s;
     std::vector<int8_t> hv;
@@ -808,25 +914,20 @@ lns_status search_setup(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L,
         vector_from_seed(c->n, seed, hv.data());
         CK(cudaMemcpyAsync(c->d_V, hv.data(), c->n, cudaMemcpyHostToDevice, st));
     }
-    size_t tw = (M + 31) / 32;
-    if ((s = grow(c->d_tabu, c->tabu_cap, tw)) != LNS_OK) return s;
-    CK(cudaMemsetAsync(c->d_tabu, 0, tw * 4, st));
-    if (L > 0) {
-        if ((s = grow(c->d_ring, c->ring_cap, (size_t)L + 1)) != LNS_OK) return s;
-    }
-    size_t tc = (size_t)std::max<int64_t>(iters, 1);
+    if ((s = grow(c->d_until, c->until_cap, g.M)) != LNS_OK) return s;
+    CK(cudaMemsetAsync(c->d_until, 0, (size_t)g.M * 4, st));
+    const size_t tc = (size_t)std::max<int64_t>(iters, 1);
     if ((s = grow(c->d_tr, c->trace_cap, tc)) != LNS_OK) return s;
     if ((s = grow(c->d_tf, c->trace_cap_f, tc)) != LNS_OK) return s;
-    k_fill_i64<<<1, 32, 0, st>>>(c->d_keys, KEY_NONE, 5);
-    CK(cudaMemsetAsync(c->d_bar, 0, 4 * sizeof(unsigned), st));
+    k_fill_i64<<<1, 32, 0, st>>>(c->d_slots + SLOT_ACC, KEY_NONE, 2);
+    CK(cudaMemsetAsync(c->d_counter, 0, sizeof(unsigned), st));
     k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, nullptr, c->d_fs);
     CK(cudaGetLastError());
-    (void)k;
     return LNS_OK;
 }
 
-lns_status search_finish(lns_ctx *c, int64_t iters, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit,
-                         lns_result *res, cudaStream_t st)
+lns_status search_finish(lns_ctx *c, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit, lns_result *res,
+                         cudaStream_t st)
 {
     int64_t fs[FS_N];
     CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
@@ -835,16 +936,16 @@ lns_status search_finish(lns_ctx *c, int64_t iters, int8_t *V_out, int64_t *trac
     CK(cudaStreamSynchronize(st));
     if (fs[FS_ERR] == 1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
     if (fs[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
-    int64_t done = fs[FS_T];
+    const int64_t done = fs[FS_T];
     if (trace_rank && done > 0) CK(cudaMemcpyAsync(trace_rank, c->d_tr, done * 8, cudaMemcpyDefault, st));
     if (trace_fit && done > 0) CK(cudaMemcpyAsync(trace_fit, c->d_tf, done * 8, cudaMemcpyDefault, st));
+    std::vector<int8_t> hv;
     if (V_out) {
-        std::vector<int8_t> hv(c->n);
+        hv.resize(c->n);
         for (int i = 0; i < c->n; i++) hv[i] = ((vb[i / 32] >> (i % 32)) & 1) ? -1 : 1;
         CK(cudaMemcpyAsync(V_out, hv.data(), c->n, cudaMemcpyDefault, st));
     }
     CK(cudaStreamSynchronize(st));
-    (void)iters;
     if (res) {
         res->iters_done = done; res->final_f = fs[FS_F]; res->best_f = fs[FS_BEST];
         res->best_iter = fs[FS_BESTIT]; res->first_zero_iter = fs[FS_ZERO];
@@ -854,15 +955,26 @@ lns_status search_finish(lns_ctx *c, int64_t iters, int8_t *V_out, int64_t *trac
 }
 
 template <int K>
-lns_status launch_search(lns_ctx *c, const SearchArgs &A, size_t smem, cudaStream_t st)
+lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st)
 {
-    set_smem_attr<K>(smem);
+    // persistent geometry: first the CTA count at the eval footprint, then cache the until[]
+    // slice in shared memory if it fits next to it
+    const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
+    CK(cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, budget));
     int occ = 0;
-    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, smem));
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
-    int nb = search_blocks(c, A.hi - A.lo, occ);
-    SearchArgs a = A;
-    void *args[] = {&a};
+    const int nb = search_blocks(c, A.hi - A.lo, 1);
+    const uint64_t slice = ((uint64_t)(A.hi - A.lo) + nb - 1) / nb + 64;
+    size_t smem = g.smem_eval;
+    if (g.smem_eval + 4 * slice <= (size_t)budget) {
+        A.until_smem = 1;
+        smem = g.smem_eval + 4 * slice;
+    }
+    // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
+    k_fill_i64<<<1, 64, 0, st>>>(c->d_slots, KEY_NONE, 48);
+    CK(cudaMemsetAsync(c->d_slots + 48, 0, 8, st));
+    void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
     CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
@@ -870,22 +982,22 @@ lns_status launch_search(lns_ctx *c, const SearchArgs &A, size_t smem, cudaStrea
 }
 
 template <int K>
-lns_status launch_step_eval(lns_ctx *c, const SearchArgs &A, size_t smem, int64_t *key_out, int32_t *fit_out,
+lns_status launch_step_eval(lns_ctx *c, const SearchArgs &A, const Geometry &g, int64_t *key_out, int32_t *fit_out,
                             bool all, cudaStream_t st)
 {
-    set_smem_attr<K>(smem);
+    CK(cudaFuncSetAttribute(k_step_eval<K, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)g.smem_eval));
+    CK(cudaFuncSetAttribute(k_step_eval<K, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)g.smem_eval));
     int occ = 0;
-    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_step_eval<K, false>, NT, smem));
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_step_eval<K, false>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "eval kernel does not fit on an SM");
     SearchArgs a = A;
-    a.keys = c->d_keys + 3;
-    a.bar = c->d_bar + 2;
+    a.slots = c->d_slots + SLOT_ACC;
     int nb = search_blocks(c, A.hi - A.lo, occ);
     if (all) {
         nb = (int)std::min<int64_t>(std::max<int64_t>(1, (A.hi - A.lo) / 1024), 4LL * c->numSMs * occ);
-        k_step_eval<K, true><<<nb, NT, smem, st>>>(a, key_out, fit_out);
+        k_step_eval<K, true><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     } else {
-        k_step_eval<K, false><<<nb, NT, smem, st>>>(a, key_out, fit_out);
+        k_step_eval<K, false><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     }
     CK(cudaGetLastError());
     return LNS_OK;
@@ -899,21 +1011,21 @@ lns_status launch_step_apply(const SearchArgs &A, const int64_t *key, cudaStream
     return LNS_OK;
 }
 
-lns_status dispatch_search(lns_ctx *c, int k, const SearchArgs &A, size_t smem, cudaStream_t st)
+lns_status dispatch_search(lns_ctx *c, int k, const SearchArgs &A, const Geometry &g, cudaStream_t st)
 {
     switch (k) {
-    case 1: return launch_search<1>(c, A, smem, st);
-    case 2: return launch_search<2>(c, A, smem, st);
-    default: return launch_search<3>(c, A, smem, st);
+    case 1: return launch_search<1>(c, A, g, st);
+    case 2: return launch_search<2>(c, A, g, st);
+    default: return launch_search<3>(c, A, g, st);
     }
 }
-lns_status dispatch_step_eval(lns_ctx *c, int k, const SearchArgs &A, size_t smem, int64_t *key_out,
+lns_status dispatch_step_eval(lns_ctx *c, int k, const SearchArgs &A, const Geometry &g, int64_t *key_out,
                               int32_t *fit_out, bool all, cudaStream_t st)
 {
     switch (k) {
-    case 1: return launch_step_eval<1>(c, A, smem, key_out, fit_out, all, st);
-    case 2: return launch_step_eval<2>(c, A, smem, key_out, fit_out, all, st);
-    default: return launch_step_eval<3>(c, A, smem, key_out, fit_out, all, st);
+    case 1: return launch_step_eval<1>(c, A, g, key_out, fit_out, all, st);
+    case 2: return launch_step_eval<2>(c, A, g, key_out, fit_out, all, st);
+    default: return launch_step_eval<3>(c, A, g, key_out, fit_out, all, st);
     }
 }
 lns_status dispatch_step_apply(int k, const SearchArgs &A, const int64_t *key, cudaStream_t st)
@@ -955,6 +1067,7 @@ const char *lns_strerror(lns_status s)
 
 const char *lns_last_error(void) { return g_err.c_str(); }
 int32_t lns_version(void) { return LNS_VERSION_NUM; }
+
 int64_t lns_neighborhood_size(int32_t n, int32_t k)
 {
     if (k < 1 || k > 3) return -1;
@@ -966,6 +1079,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     if (!out || !A || !S) return fail(LNS_EINVAL, "null argument");
     *out = nullptr;
     if (m < 1 || n < 1) return fail(LNS_EINVAL, "m and n must be >= 1");
+    if (m > 65535) return fail(LNS_ERANGE, "m > 65535");
     if (60LL * m * n + 2LL * m >= (int64_t)INT32_MAX) return fail(LNS_ERANGE, "60 m n + 2 m >= 2^31");
     if (n > 4096) return fail(LNS_ERANGE, "n > 4096");
     int ndev = 0;
@@ -981,7 +1095,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     std::vector<int32_t> H(n + 1, 0);
     for (int j = 0; j < m; j++) {
         for (int i = 0; i < n; i++) {
-            int8_t a = hA[(size_t)j * n + i];
+            const int8_t a = hA[(size_t)j * n + i];
             if (a != 1 && a != -1) return fail(LNS_EINVAL, "A entries must be +1 or -1");
             if (a < 0) arow[(size_t)j * NWn + i / 32] |= 1u << (i % 32);
         }
@@ -996,15 +1110,15 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
         return cleanup(fail(LNS_ECUDA, "device attributes"));
     if (cudaMalloc(&c->d_Arow, arow.size() * 4) != cudaSuccess || cudaMalloc(&c->d_H, (n + 1) * 4) != cudaSuccess ||
         cudaMalloc(&c->d_vb, NWn * 4) != cudaSuccess || cudaMalloc(&c->d_Y, m * 4) != cudaSuccess ||
-        cudaMalloc(&c->d_fs, FS_N * 8) != cudaSuccess || cudaMalloc(&c->d_keys, 8 * 8) != cudaSuccess ||
-        cudaMalloc(&c->d_bar, 4 * sizeof(unsigned)) != cudaSuccess || cudaMalloc(&c->d_V, n) != cudaSuccess ||
+        cudaMalloc(&c->d_fs, FS_N * 8) != cudaSuccess || cudaMalloc(&c->d_slots, SLOT_N * 8) != cudaSuccess ||
+        cudaMalloc(&c->d_counter, sizeof(unsigned)) != cudaSuccess || cudaMalloc(&c->d_V, n) != cudaSuccess ||
         cudaMalloc(&c->d_Yin, m * 4) != cudaSuccess) {
         cudaGetLastError();
         return cleanup(fail(LNS_ENOMEM, "cudaMalloc failed"));
     }
     if (cudaMemcpy(c->d_Arow, arow.data(), arow.size() * 4, cudaMemcpyHostToDevice) != cudaSuccess ||
         cudaMemcpy(c->d_H, H.data(), (n + 1) * 4, cudaMemcpyHostToDevice) != cudaSuccess ||
-        cudaMemset(c->d_bar, 0, 4 * sizeof(unsigned)) != cudaSuccess ||
+        cudaMemset(c->d_counter, 0, sizeof(unsigned)) != cudaSuccess ||
         cudaEventCreate(&c->ev0) != cudaSuccess || cudaEventCreate(&c->ev1) != cudaSuccess)
         return cleanup(fail(LNS_ECUDA, "upload"));
     *out = c;
@@ -1016,8 +1130,8 @@ void lns_destroy(lns_ctx *c)
     if (!c) return;
     DeviceGuard g(c->device);
     cudaFree(c->d_Arow); cudaFree(c->d_H); cudaFree(c->d_vb); cudaFree(c->d_Y); cudaFree(c->d_fs);
-    cudaFree(c->d_keys); cudaFree(c->d_bar); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_tabu);
-    cudaFree(c->d_ring); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
+    cudaFree(c->d_slots); cudaFree(c->d_counter); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_bits);
+    cudaFree(c->d_until); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
     delete c;
@@ -1057,28 +1171,32 @@ lns_status lns_attach_comm(lns_ctx *c, void *comm, int32_t rank, int32_t world)
 lns_status lns_eval_neighborhood(lns_ctx *c, int32_t k, const int8_t *V, const int32_t *Y, const uint32_t *tabu_bits,
                                  int64_t *best_fitness, int64_t *best_rank, void *stream)
 {
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, k, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
     if (!V || !Y || !best_fitness || !best_rank) return fail(LNS_EINVAL, "null argument");
-    DeviceGuard g(c->device);
+    DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
-    size_t tw = (M + 31) / 32;
-    if ((s = grow(c->d_tabu, c->tabu_cap, tw)) != LNS_OK) return s;
-    if (tabu_bits) CK(cudaMemcpyAsync(c->d_tabu, tabu_bits, tw * 4, cudaMemcpyDefault, st));
-    else CK(cudaMemsetAsync(c->d_tabu, 0, tw * 4, st));
+    const size_t tw = (g.M + 31) / 32;
+    if ((s = grow(c->d_until, c->until_cap, g.M)) != LNS_OK) return s;
+    if (tabu_bits) {
+        if ((s = grow(c->d_bits, c->bits_cap, tw)) != LNS_OK) return s;
+        CK(cudaMemcpyAsync(c->d_bits, tabu_bits, tw * 4, cudaMemcpyDefault, st));
+    }
+    k_bits_to_until<<<std::min<uint32_t>(4096, (g.M + 255) / 256), 256, 0, st>>>(tabu_bits ? c->d_bits : nullptr,
+                                                                                c->d_until, g.M);
     CK(cudaMemcpyAsync(c->d_V, V, c->n, cudaMemcpyDefault, st));
     CK(cudaMemcpyAsync(c->d_Yin, Y, 4 * (size_t)c->m, cudaMemcpyDefault, st));
-    k_fill_i64<<<1, 32, 0, st>>>(c->d_keys, KEY_NONE, 5);
-    CK(cudaMemsetAsync(c->d_bar, 0, 4 * sizeof(unsigned), st));
+    k_fill_i64<<<1, 32, 0, st>>>(c->d_slots + SLOT_ACC, KEY_NONE, 2);
+    CK(cudaMemsetAsync(c->d_counter, 0, sizeof(unsigned), st));
     k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, c->d_Yin, c->d_fs);
     CK(cudaGetLastError());
-    SearchArgs A = make_args(c, M, 1, 0, 0);
+    SearchArgs A = make_args(c, g, 1, 0, 0);
     CK(cudaEventRecord(c->ev0, st));
-    if ((s = dispatch_step_eval(c, k, A, smem, c->d_keys + 4, nullptr, false, st)) != LNS_OK) return s;
+    if ((s = dispatch_step_eval(c, k, A, g, c->d_slots + SLOT_OUT, nullptr, false, st)) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev1, st));
     int64_t key, fs[FS_N];
-    CK(cudaMemcpyAsync(&key, c->d_keys + 4, 8, cudaMemcpyDeviceToHost, st));
+    CK(cudaMemcpyAsync(&key, c->d_slots + SLOT_OUT, 8, cudaMemcpyDeviceToHost, st));
     CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
     CK(cudaStreamSynchronize(st));
     float ms = 0; cudaEventElapsedTime(&ms, c->ev0, c->ev1); c->last_ms = ms;
@@ -1091,28 +1209,26 @@ lns_status lns_eval_neighborhood(lns_ctx *c, int32_t k, const int8_t *V, const i
 
 lns_status lns_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness_out, void *stream)
 {
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, k, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
     if (!V || !fitness_out) return fail(LNS_EINVAL, "null argument");
-    DeviceGuard g(c->device);
+    DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
-    if ((s = grow(c->d_fit, c->fit_cap, M)) != LNS_OK) return s;
-    size_t tw = (M + 31) / 32;
-    if ((s = grow(c->d_tabu, c->tabu_cap, tw)) != LNS_OK) return s;
-    CK(cudaMemsetAsync(c->d_tabu, 0, tw * 4, st));
+    if ((s = grow(c->d_fit, c->fit_cap, g.M)) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V, V, c->n, cudaMemcpyDefault, st));
-    k_fill_i64<<<1, 32, 0, st>>>(c->d_keys, KEY_NONE, 5);
-    CK(cudaMemsetAsync(c->d_bar, 0, 4 * sizeof(unsigned), st));
+    k_fill_i64<<<1, 32, 0, st>>>(c->d_slots + SLOT_ACC, KEY_NONE, 2);
+    CK(cudaMemsetAsync(c->d_counter, 0, sizeof(unsigned), st));
     k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, nullptr, c->d_fs);
-    SearchArgs A = make_args(c, M, 1, 0, 0);
-    A.lo = 0; A.hi = M;
+    SearchArgs A = make_args(c, g, 1, 0, 0);
+    A.lo = 0; A.hi = g.M;
+    A.until = nullptr;
     CK(cudaEventRecord(c->ev0, st));
-    if ((s = dispatch_step_eval(c, k, A, smem, c->d_keys + 4, c->d_fit, true, st)) != LNS_OK) return s;
+    if ((s = dispatch_step_eval(c, k, A, g, c->d_slots + SLOT_OUT, c->d_fit, true, st)) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev1, st));
     int64_t fs[FS_N];
     CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
-    CK(cudaMemcpyAsync(fitness_out, c->d_fit, 4 * (size_t)M, cudaMemcpyDefault, st));
+    CK(cudaMemcpyAsync(fitness_out, c->d_fit, 4 * (size_t)g.M, cudaMemcpyDefault, st));
     CK(cudaStreamSynchronize(st));
     float ms = 0; cudaEventElapsedTime(&ms, c->ev0, c->ev1); c->last_ms = ms;
     if (fs[FS_ERR]) return fail(LNS_EINVAL, "V must be +-1");
@@ -1122,14 +1238,14 @@ lns_status lns_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness
 lns_status lns_step_begin(lns_ctx *c, int32_t k, int64_t max_iters, int64_t tenure, uint64_t seed, const int8_t *V0,
                           int32_t flags, void *stream)
 {
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, k, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
     if (max_iters < 0) return fail(LNS_EINVAL, "iters < 0");
     int64_t L;
-    if ((s = resolve_tenure(M, tenure, L)) != LNS_OK) return s;
-    DeviceGuard g(c->device);
-    if ((s = search_setup(c, k, M, max_iters, L, seed, V0, (cudaStream_t)stream)) != LNS_OK) return s;
+    if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
+    DeviceGuard dg(c->device);
+    if ((s = search_setup(c, g, max_iters, seed, V0, (cudaStream_t)stream)) != LNS_OK) return s;
     c->step_active = true; c->step_K = k; c->step_iters = max_iters; c->step_L = L; c->step_flags = flags;
     return LNS_OK;
 }
@@ -1137,59 +1253,60 @@ lns_status lns_step_begin(lns_ctx *c, int32_t k, int64_t max_iters, int64_t tenu
 lns_status lns_step_eval(lns_ctx *c, int64_t *key_dev, void *stream)
 {
     if (!c || !c->step_active || !key_dev) return fail(LNS_EINVAL, "no active stepped search");
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, c->step_K, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, c->step_K, g);
     if (s != LNS_OK) return s;
-    DeviceGuard g(c->device);
-    SearchArgs A = make_args(c, M, c->step_iters, c->step_L, c->step_flags);
-    return dispatch_step_eval(c, c->step_K, A, smem, key_dev, nullptr, false, (cudaStream_t)stream);
+    DeviceGuard dg(c->device);
+    SearchArgs A = make_args(c, g, c->step_iters, c->step_L, c->step_flags);
+    return dispatch_step_eval(c, c->step_K, A, g, key_dev, nullptr, false, (cudaStream_t)stream);
 }
 
 lns_status lns_step_apply(lns_ctx *c, const int64_t *key_dev, void *stream)
 {
     if (!c || !c->step_active || !key_dev) return fail(LNS_EINVAL, "no active stepped search");
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, c->step_K, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, c->step_K, g);
     if (s != LNS_OK) return s;
-    DeviceGuard g(c->device);
-    SearchArgs A = make_args(c, M, c->step_iters, c->step_L, c->step_flags);
+    DeviceGuard dg(c->device);
+    SearchArgs A = make_args(c, g, c->step_iters, c->step_L, c->step_flags);
     return dispatch_step_apply(c->step_K, A, key_dev, (cudaStream_t)stream);
 }
 
 lns_status lns_step_end(lns_ctx *c, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit, lns_result *res, void *stream)
 {
     if (!c || !c->step_active) return fail(LNS_EINVAL, "no active stepped search");
-    DeviceGuard g(c->device);
+    DeviceGuard dg(c->device);
     c->step_active = false;
-    return search_finish(c, c->step_iters, V_out, trace_rank, trace_fit, res, (cudaStream_t)stream);
+    return search_finish(c, V_out, trace_rank, trace_fit, res, (cudaStream_t)stream);
 }
 
 lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, uint64_t seed, const int8_t *V0,
                         int32_t flags, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit, lns_result *res,
                         void *stream)
 {
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, k, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
     if (!res) return fail(LNS_EINVAL, "res is required");
-    if (iters < 0) return fail(LNS_EINVAL, "iters < 0");
+    if (iters < 0 || iters >= (int64_t)INT32_MAX) return fail(LNS_EINVAL, "iters must be in [0, 2^31)");
     int64_t L;
-    if ((s = resolve_tenure(M, tenure, L)) != LNS_OK) return s;
-    DeviceGuard g(c->device);
+    if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
+    if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
-    if ((s = search_setup(c, k, M, iters, L, seed, V0, st)) != LNS_OK) return s;
-    SearchArgs A = make_args(c, M, iters, L, flags);
+    if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
+    SearchArgs A = make_args(c, g, iters, L, flags);
     const bool stepped = c->comm != nullptr || c->nparts > 1 || (flags & LNS_FORCE_STEPPED);
     if (!stepped) {
-        if (iters > 0 && (s = dispatch_search(c, k, A, smem, st)) != LNS_OK) return s;
+        if (iters > 0 && (s = dispatch_search(c, k, A, g, st)) != LNS_OK) return s;
     } else {
         if (c->nparts > 1 && !c->comm) return fail(LNS_EINVAL, "partitioned run needs a communicator (or use the stepped API)");
-        int64_t *kb = c->d_keys + 4;
+        int64_t *kb = c->d_slots + SLOT_OUT;
         CK(cudaEventRecord(c->ev0, st));
         for (int64_t t = 0; t < iters; t++) {
-            if ((s = dispatch_step_eval(c, k, A, smem, kb, nullptr, false, st)) != LNS_OK) return s;
+            if ((s = dispatch_step_eval(c, k, A, g, kb, nullptr, false, st)) != LNS_OK) return s;
             if (c->comm) {
-                int rc = c->nccl_allreduce(kb, kb, 1, /*ncclUint64*/ 5, /*ncclMin*/ 3, c->comm, st);
+                const int rc = c->nccl_allreduce(kb, kb, 1, /*ncclUint64*/ 5, /*ncclMin*/ 3, c->comm, st);
                 if (rc != 0) return fail(LNS_ENCCL, "ncclAllReduce failed");
             }
             if ((s = dispatch_step_apply(k, A, kb, st)) != LNS_OK) return s;
@@ -1202,7 +1319,7 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         }
         CK(cudaEventRecord(c->ev1, st));
     }
-    s = search_finish(c, iters, V_out, trace_rank, trace_fit, res, st);
+    s = search_finish(c, V_out, trace_rank, trace_fit, res, st);
     float ms = 0;
     if (iters > 0 && cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
     cudaGetLastError();
@@ -1213,14 +1330,14 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
                               const int8_t *V0, int32_t flags, int8_t *V_out, lns_result *res, void *stream)
 {
     if (!c || !res || R < 0) return fail(LNS_EINVAL, "bad argument");
-    int savep = c->part, saven = c->nparts;
+    const int savep = c->part, saven = c->nparts;
     void *savec = c->comm;
     c->part = 0; c->nparts = 1; c->comm = nullptr;
     lns_status s = LNS_OK;
     double total_ms = 0;
     for (int r = 0; r < R && s == LNS_OK; r++) {
         uint64_t st = seed + (uint64_t)r;
-        uint64_t seed_r = splitmix64_next(st);
+        const uint64_t seed_r = splitmix64_next(st);
         const int8_t *v0 = V0 ? V0 + (size_t)r * c->n : nullptr;
         int8_t *vo = V_out ? V_out + (size_t)r * c->n : nullptr;
         s = lns_tabu_run(c, k, iters, tenure, seed_r, v0, flags & ~LNS_FORCE_STEPPED, vo, nullptr, nullptr, &res[r], stream);
@@ -1231,21 +1348,33 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     return s;
 }
 
+#ifdef LNS_PHASE_TIMING
+// Profiling build only: read (and reset) the per-phase cycle sums over CTAs and iterations.
+lns_status lns_debug_phases(unsigned long long *out8)
+{
+    CK(cudaMemcpyFromSymbol(out8, g_ph, sizeof(unsigned long long) * NPH));
+    unsigned long long z[NPH] = {0};
+    CK(cudaMemcpyToSymbol(g_ph, z, sizeof(z)));
+    return LNS_OK;
+}
+#endif
+
 // Undocumented debug export (tests/tools only): plan of V for neighbourhood k, see k_debug_plan.
 lns_status lns_debug_plan(lns_ctx *c, int32_t k, const int8_t *V, int32_t *out_host, int64_t cap)
 {
-    uint32_t M; size_t smem;
-    lns_status s = check_k(c, k, M, smem);
+    Geometry g;
+    lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
-    DeviceGuard g(c->device);
+    DeviceGuard dg(c->device);
     int32_t *d_out = nullptr;
     CK(cudaMalloc(&d_out, cap * 4));
     CK(cudaMemcpy(c->d_V, V, c->n, cudaMemcpyDefault));
     k_init<<<1, NT>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, nullptr, c->d_fs);
-    SearchArgs A = make_args(c, M, 1, 0, 0);
-    if (k == 1) { cudaFuncSetAttribute(k_debug_plan<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem); k_debug_plan<1><<<1, NT, smem>>>(A, d_out); }
-    else if (k == 2) { cudaFuncSetAttribute(k_debug_plan<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem); k_debug_plan<2><<<1, NT, smem>>>(A, d_out); }
-    else { cudaFuncSetAttribute(k_debug_plan<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem); k_debug_plan<3><<<1, NT, smem>>>(A, d_out); }
+    SearchArgs A = make_args(c, g, 1, 0, 0);
+    const int sm = (int)g.smem_eval;
+    if (k == 1) { cudaFuncSetAttribute(k_debug_plan<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, sm); k_debug_plan<1><<<1, NT, sm>>>(A, d_out); }
+    else if (k == 2) { cudaFuncSetAttribute(k_debug_plan<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, sm); k_debug_plan<2><<<1, NT, sm>>>(A, d_out); }
+    else { cudaFuncSetAttribute(k_debug_plan<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, sm); k_debug_plan<3><<<1, NT, sm>>>(A, d_out); }
     CK(cudaMemcpy(out_host, d_out, cap * 4, cudaMemcpyDeviceToHost));
     cudaFree(d_out);
     return LNS_OK;
@@ -1255,11 +1384,12 @@ lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count,
 {
     if (k < 1 || k > 3 || n < k) return fail(LNS_EINVAL, "bad n/k");
     if (count < 0 || (count > 0 && (!ranks || !out))) return fail(LNS_EINVAL, "bad buffers");
-    int64_t Mk = comb_k(n, k);
+    const int64_t Mk = comb_k(n, k);
     if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
     if (count == 0) return LNS_OK;
     cudaStream_t st = (cudaStream_t)stream;
-    int64_t *d_r = nullptr; int32_t *d_o = nullptr, *d_bad = nullptr;
+    int64_t *d_r = nullptr;
+    int32_t *d_o = nullptr, *d_bad = nullptr;
     if (cudaMalloc(&d_r, count * 8) != cudaSuccess || cudaMalloc(&d_o, count * 12) != cudaSuccess ||
         cudaMalloc(&d_bad, 4) != cudaSuccess) {
         cudaFree(d_r); cudaFree(d_o); cudaGetLastError();
@@ -1268,13 +1398,13 @@ lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count,
     int bad = 0;
     cudaMemcpyAsync(d_r, ranks, count * 8, cudaMemcpyDefault, st);
     cudaMemsetAsync(d_bad, 0, 4, st);
-    int blocks = (int)std::min<int64_t>((count + 255) / 256, 4096);
+    const int blocks = (int)std::min<int64_t>((count + 255) / 256, 4096);
     if (k == 1) k_unrank<1><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
     else if (k == 2) k_unrank<2><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
     else k_unrank<3><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
     cudaMemcpyAsync(out, d_o, count * 12, cudaMemcpyDefault, st);
     cudaMemcpyAsync(&bad, d_bad, 4, cudaMemcpyDeviceToHost, st);
-    cudaError_t e = cudaStreamSynchronize(st);
+    const cudaError_t e = cudaStreamSynchronize(st);
     cudaFree(d_r); cudaFree(d_o); cudaFree(d_bad);
     if (e != cudaSuccess) return fail(LNS_ECUDA, cudaGetErrorString(e));
     if (bad) return fail(LNS_EINVAL, "rank out of range");
