@@ -100,7 +100,7 @@ struct SearchArgs {
 // Shared-memory carve-up (identical on host and device). The bit-packed A (Ar) and the until[]
 // slice are staged only when they fit.
 struct Smem {
-    int X, Y, vb, H, cnt, seg, cur, pofs, rowAt, bins, pieces, pstart, base_end, Ar, a_end;
+    int X, Y, vb, H, cnt, seg, cur, pofs, rowAt, bins, pieces, pstart, T2, T3, base_end, Ar, a_end;
 };
 
 __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
@@ -121,6 +121,8 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
     s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
     s.pieces = o; o = align16(o + 8 * (n + 1 + W));      // P <= U + W - 1 pieces
     s.pstart = o; o = align16(o + 4 * (W + 1));
+    s.T2 = o;     o = align16(o + 4 * n);                // C(y,2), y < n (u32)
+    s.T3 = o;     o = align16(o + 4 * n);                // C(z,3), z < n (u32: C(n,3) < 2^32)
     s.base_end = o;
     s.Ar = o;
     if (a_in_smem) o = align16(o + 4 * m * NWn);
@@ -166,6 +168,42 @@ __device__ __forceinline__ void unrank(uint32_t r, int n, uint32_t M, int &a, in
     else { b = n - 1 - y; c = n - 1 - (int)R; }
 }
 
+// The same unranking from shared tables T2[y] = C(y,2), T3[z] = C(z,3) (u32, exact), with a
+// log2/exp2 estimate: no 64-bit arithmetic on the hot path. The correction loops make it exact.
+template <int K>
+__device__ __forceinline__ void unrank_tab(uint32_t r, int n, uint32_t M, const uint32_t *__restrict__ T2,
+                                           const uint32_t *__restrict__ T3, int &a, int &b, int &c)
+{
+    if (K == 1) { a = (int)r; b = -1; c = -1; return; }
+    uint32_t R = M - 1u - r;
+    int top = n - 1;
+    if (K == 3) {
+        int z = (int)exp2f(__log2f(6.0f * (float)R + 1.0f) * (1.0f / 3.0f)) + 1;
+        z = min(max(z, 2), top);
+        while (T3[z] > R) z--;
+        while (z < top && T3[z + 1] <= R) z++;
+        R -= T3[z];
+        a = n - 1 - z;
+        top = z - 1;
+    }
+    int y = (int)((1.0f + sqrtf(8.0f * (float)R + 1.0f)) * 0.5f);
+    y = min(max(y, 1), top);
+    while (T2[y] > R) y--;
+    while (y < top && T2[y + 1] <= R) y++;
+    R -= T2[y];
+    if (K == 2) { a = n - 1 - y; b = n - 1 - (int)R; c = -1; }
+    else { b = n - 1 - y; c = n - 1 - (int)R; }
+}
+
+__device__ __forceinline__ void fill_tables(uint32_t *T2, uint32_t *T3, int n)
+{
+    for (int i = threadIdx.x; i < n; i += blockDim.x) {
+        const uint64_t z = (uint64_t)i;
+        T2[i] = (uint32_t)(z * (z - 1) / 2);
+        T3[i] = i >= 2 ? (uint32_t)(z * (z - 1) * (z - 2) / 6) : 0u;
+    }
+}
+
 __device__ __forceinline__ int warp_min_i(int v) {
     for (int o = 16; o; o >>= 1) v = min(v, __shfl_xor_sync(FULL, v, o));
     return v;
@@ -209,9 +247,9 @@ __device__ __forceinline__ void range_publish(int mn, int mx, PlanScalars &ps)
 // plan's range widened by 2k after a move: |Y'_j - Y_j| <= 2k). The exact range is found here.
 //   cnt/cur   rows per conservative lattice point (Y = vlo + 2u)
 //   seg       start of segment u - ufirst in sorted-row order (exact lattice, Y = vmin + 2u)
-//   pieces    (mask, fin | len << 16): the part of one segment inside one 32-row word, in row
-//             order; fin > 0 on a segment's last piece = number of bins finalised after it
-//             (1 + the empty lattice points that follow, or + the 2K trailing bins)
+//   pieces    (mask, fin | w << 1 | len << 16): the part of one segment inside row word w, in row
+//             order; fin = 1 on a segment's last piece (its bin is then complete); an empty
+//             lattice point is one zero piece (mask 0, fin 1, len 0)
 //   pstart    first piece of each row word
 //   bins      (H_b, w_b) of bin beta <-> b = vmin + 2(beta - K): w_b = 60|b| - 1 for b < 0
 //   X[w][c]   sign bits x_jc = [A_jc V_c = -1] of sorted rows 32w..32w+31, column c
@@ -260,7 +298,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             int inc = v;
             for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, inc, o); if (lane >= o) inc += t; }
             const int st = runr + inc - v, en = runr + inc;
-            const int np = v > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : 0;
+            const int np = v > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : 1;  // empty point: one zero piece
             int incp = np;
             for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, incp, o); if (lane >= o) incp += t; }
             if (v_ < U) { seg[v_] = st; cur[u] = st; pofs[v_] = runp + incp - np; }
@@ -285,17 +323,17 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         rowAt[p] = j;
     }
     for (int v = tid; v < U; v += NT) {
-        if (cnt[uf + v] == 0) continue;
         const int st = seg[v], en = seg[v + 1];
-        const int w0 = st >> 5, w1 = (en - 1) >> 5;
-        int q = v + 1;
-        while (q < U && cnt[uf + q] == 0) q++;
-        const int fin_last = (q >= U ? NB : q) - v;
         int p = pofs[v];
+        if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
+            pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
+            continue;
+        }
+        const int w0 = st >> 5, w1 = (en - 1) >> 5;
         for (int w = w0; w <= w1; w++, p++) {
             const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
             const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
-            pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? fin_last : 0) | ((uint32_t)(en - st) << 16));
+            pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? 1 : 0) | ((uint32_t)w << 1) | ((uint32_t)(en - st) << 16));
             if (w > w0 || (st & 31) == 0) pstart[w] = p;
         }
     }
@@ -326,85 +364,122 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     PH(3);
 }
 
-// Fitness of neighbour (a, b, c) from the plan, word-major: the lane's columns of one row word
-// are loaded once, bit-sliced into t = #flipped "-1" entries (lo, hi planes), and every piece of
-// that word adds its POPC counts. On a segment's last piece its row counts N_t (t = 0..k) are
-// known; they land in bins beta + 2t, and a 2k-long shift register finalises one bin per segment.
+// One lattice point (segment) of eval_fit: its pieces add POPC counts of the bit-sliced planes
+// (reloading the lane's three column words only when the piece's row word changes); then its row
+// counts N_t land in bins beta + 2t and bin beta is complete. Registers Ra.. hold bins
+// beta .. beta+2K-1; the caller rotates the names (Ra becomes bin beta+2K), so no moves are needed.
+template <int K>
+__device__ __forceinline__ void seg_step(const uint2 *__restrict__ &pp, const int2 *__restrict__ &bp,
+                                         const uint32_t *__restrict__ X, int n, int a, int b, int c, int &curw,
+                                         uint32_t &lo, uint32_t &hi, uint32_t &lh, int &f, int &smin,
+                                         int &Ra, int &Rc, int &Re)
+{
+    int c1 = 0, c2 = 0, c3 = 0;
+    uint2 rec;
+    do {
+        rec = *pp++;
+        const int w = (int)((rec.y >> 1) & 0x7fffu);
+        if (w != curw) {
+            curw = w;
+            const uint32_t *xr = X + w * n;
+            if (K == 1) {
+                lo = xr[a];
+            } else if (K == 2) {
+                const uint32_t xa = xr[a], xb = xr[b];
+                lo = xa ^ xb; hi = xa & xb;
+            } else {
+                const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+                lo = xa ^ xb ^ xc;
+                hi = (xa & xb) | (xc & (xa ^ xb));
+                lh = lo & hi;
+            }
+        }
+        c1 += __popc(lo & rec.x);
+        if (K >= 2) c2 += __popc(hi & rec.x);
+        if (K == 3) c3 += __popc(lh & rec.x);
+    } while (!(rec.y & 1u));
+    const int len = (int)(rec.y >> 16);
+    int h;
+    if (K == 1) {         // N1 = c1 -> bin beta+2 (reuses Ra)
+        h = Ra + len - c1;
+        Ra = c1;
+    } else if (K == 2) {  // N1 = c1 -> beta+2 (Rc), N2 = c2 -> beta+4 (Ra)
+        h = Ra + len - c1 - c2;
+        Rc += c1; Ra = c2;
+    } else {              // N1 = c1-c3 -> beta+2 (Rc), N2 = c2-c3 -> beta+4 (Re), N3 = c3 -> beta+6 (Ra)
+        h = Ra + len - c1 - c2 + c3;
+        Rc += c1 - c3; Re += c2 - c3; Ra = c3;
+    }
+    const int2 bn = *bp++;
+    f += bn.y * h;
+    smin += min(h, bn.x);
+}
+
+__device__ __forceinline__ void bin_cost(int h, int2 bn, int &f, int &smin)
+{
+    f += bn.y * h;
+    smin += min(h, bn.x);
+}
+
+// Fitness of neighbour (a, b, c) from the plan, segment-major over the U lattice points:
 //   f = 2m + sum_beta ( w_beta h_beta - 2 min(h_beta, H_beta) )
 // (|h - H| = h + H - 2 min(h, H) summed over b = 0..n; every row lands in exactly one bin.)
 template <int K>
 __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
-                                        const int *__restrict__ pstart, const int2 *__restrict__ bins,
-                                        int n, int W, int m2, int a, int b, int c)
+                                        const int2 *__restrict__ bins, int n, int U, int m2, int a, int b, int c)
 {
     int f = m2, smin = 0;
-    int R[2 * K];
-#pragma unroll
-    for (int i = 0; i < 2 * K; i++) R[i] = 0;
-    int c1 = 0, c2 = 0, c3 = 0;
-    int beta = 0, p = 0;
-    for (int w = 0; w < W; w++) {
-        const uint32_t *xr = X + w * n;
-        uint32_t lo, hi = 0, lh = 0;
-        if (K == 1) {
-            lo = xr[a];
-        } else if (K == 2) {
-            const uint32_t xa = xr[a], xb = xr[b];
-            lo = xa ^ xb; hi = xa & xb;
-        } else {
-            const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
-            lo = xa ^ xb ^ xc;
-            hi = (xa & xb) | (xc & (xa ^ xb));
-            lh = lo & hi;
+    int R0 = 0, R1 = 0, R2 = 0, R3 = 0, R4 = 0, R5 = 0;
+    int curw = -1;
+    uint32_t lo = 0, hi = 0, lh = 0;
+    const uint2 *pp = pieces;
+    const int2 *bp = bins;
+    int u = 0;
+#define SEG(Ra, Rc, Re) seg_step<K>(pp, bp, X, n, a, b, c, curw, lo, hi, lh, f, smin, Ra, Rc, Re)
+#define TRAIL2(A, B) { bin_cost(A, bp[0], f, smin); bin_cost(B, bp[1], f, smin); }
+#define TRAIL4(A, B, C, D) { TRAIL2(A, B) bin_cost(C, bp[2], f, smin); bin_cost(D, bp[3], f, smin); }
+#define TRAIL6(A, B, C, D, E, F) { TRAIL4(A, B, C, D) bin_cost(E, bp[4], f, smin); bin_cost(F, bp[5], f, smin); }
+    if (K == 1) {
+        for (;;) {
+            SEG(R0, R0, R0); if (++u == U) { TRAIL2(R1, R0); break; }
+            SEG(R1, R1, R1); if (++u == U) { TRAIL2(R0, R1); break; }
         }
-        const int pend = pstart[w + 1];
-        for (; p < pend; p++) {
-            const uint2 rec = pieces[p];
-            c1 += __popc(lo & rec.x);
-            if (K >= 2) c2 += __popc(hi & rec.x);
-            if (K == 3) c3 += __popc(lh & rec.x);
-            const int fin = rec.y & 0xffffu;
-            if (fin) {
-                const int len = rec.y >> 16;
-                int N[K + 1];
-                if (K == 1) { N[1] = c1; N[0] = len - c1; }
-                else if (K == 2) { N[2] = c2; N[1] = c1; N[0] = len - c1 - c2; }
-                else { N[3] = c3; N[2] = c2 - c3; N[1] = c1 - c3; N[0] = len - c1 - c2 + c3; }
-                int h = R[0] + N[0];
-#pragma unroll
-                for (int i = 0; i < 2 * K - 1; i++) R[i] = (i & 1) ? R[i + 1] + N[(i + 1) >> 1] : R[i + 1];
-                R[2 * K - 1] = N[K];
-                int2 bn = bins[beta++];
-                f += bn.y * h;
-                smin += min(h, bn.x);
-                c1 = 0; c2 = 0; c3 = 0;
-                for (int e = 1; e < fin; e++) {
-                    h = R[0];
-#pragma unroll
-                    for (int i = 0; i < 2 * K - 1; i++) R[i] = R[i + 1];
-                    R[2 * K - 1] = 0;
-                    bn = bins[beta++];
-                    f += bn.y * h;
-                    smin += min(h, bn.x);
-                }
-            }
+    } else if (K == 2) {
+        for (;;) {
+            SEG(R0, R2, R0); if (++u == U) { TRAIL4(R1, R2, R3, R0); break; }
+            SEG(R1, R3, R1); if (++u == U) { TRAIL4(R2, R3, R0, R1); break; }
+            SEG(R2, R0, R2); if (++u == U) { TRAIL4(R3, R0, R1, R2); break; }
+            SEG(R3, R1, R3); if (++u == U) { TRAIL4(R0, R1, R2, R3); break; }
+        }
+    } else {
+        for (;;) {
+            SEG(R0, R2, R4); if (++u == U) { TRAIL6(R1, R2, R3, R4, R5, R0); break; }
+            SEG(R1, R3, R5); if (++u == U) { TRAIL6(R2, R3, R4, R5, R0, R1); break; }
+            SEG(R2, R4, R0); if (++u == U) { TRAIL6(R3, R4, R5, R0, R1, R2); break; }
+            SEG(R3, R5, R1); if (++u == U) { TRAIL6(R4, R5, R0, R1, R2, R3); break; }
+            SEG(R4, R0, R2); if (++u == U) { TRAIL6(R5, R0, R1, R2, R3, R4); break; }
+            SEG(R5, R1, R3); if (++u == U) { TRAIL6(R0, R1, R2, R3, R4, R5); break; }
         }
     }
+#undef SEG
+#undef TRAIL2
+#undef TRAIL4
+#undef TRAIL6
     return f - 2 * smin;
 }
 
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
 // key. until (nullable) is indexed by r - ubase: rank r is tabu iff until[r - ubase] >= t.
 template <int K, bool WRITE_ALL>
-__device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
+__device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L, int U,
                                          uint32_t M, uint32_t blo, uint32_t bhi, const uint32_t *until,
                                          uint32_t ubase, uint32_t t, int32_t *fit_out)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
     const uint2 *pieces = (const uint2 *)(sm + L.pieces);
-    const int *pstart = (const int *)(sm + L.pstart);
     const int2 *bins = (const int2 *)(sm + L.bins);
+    const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
@@ -412,8 +487,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const bool is_tabu = until && until[r - ubase] >= t;
             if (!is_tabu || WRITE_ALL) {
                 int a, b, c;
-                unrank<K>(r, I.n, M, a, b, c);
-                const int f = eval_fit<K>(X, pieces, pstart, bins, I.n, I.W, 2 * I.m, a, b, c);
+                unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
+                const int f = eval_fit<K>(X, pieces, bins, I.n, U, 2 * I.m, a, b, c);
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 if (!is_tabu && key < best) best = key;
@@ -470,6 +545,7 @@ __device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, co
     for (int w = threadIdx.x; w < A.I.NWn; w += NT) vbs[w] = A.vb[w];
     for (int b = threadIdx.x; b <= A.I.n; b += NT) Hs[b] = A.I.H[b];
     for (int u = threadIdx.x; u < A.I.n + 2 + 2 * K; u += NT) cnt[u] = 0;
+    fill_tables((uint32_t *)(sm + L.T2), (uint32_t *)(sm + L.T3), A.I.n);
     const uint32_t *Ar = A.I.Arow;
     if (A.a_in_smem) {
         uint32_t *As = (uint32_t *)(sm + L.Ar);
@@ -570,7 +646,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     for (; t <= t0 + A.iters; t++) {
         if (A.stop_on_zero && f == 0) break;
         build_plan<K>(A.I, Ar, sm, L, ps);
-        unsigned long long mine = eval_range<K, false>(A.I, sm, L, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr);
+        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps.U, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr);
         mine = warp_min_k(mine);
         if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
         __syncthreads();
@@ -608,7 +684,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (f == 0 && zero_it < 0) zero_it = t;
         }
         int a, b, c;
-        unrank<K>(r, A.I.n, A.M, a, b, c);
+        unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), a, b, c);
         apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
         PH(6);
     }
@@ -647,7 +723,7 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
     cta_slice(A.lo, A.hi, blockIdx.x, gridDim.x, blo, bhi);
     build_plan<K>(A.I, Ar, sm, L, ps);
     const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
-    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, A.M, blo, bhi, A.until, 0, t, fit_out);
+    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps.U, A.M, blo, bhi, A.until, 0, t, fit_out);
     mine = warp_min_k(mine);
     if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
     __syncthreads();
@@ -728,14 +804,20 @@ __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out
     }
 }
 
+// Unranking as the hot path does it (shared tables); tab = 0 uses the 64-bit reference version.
 template <int K>
-__global__ void k_unrank(int n, uint32_t M, const int64_t *ranks, int64_t count, int32_t *out, int32_t *bad)
+__global__ void k_unrank(int n, uint32_t M, const int64_t *ranks, int64_t count, int32_t *out, int32_t *bad, int tab)
 {
+    extern __shared__ uint32_t tabs[];
+    uint32_t *T2 = tabs, *T3 = tabs + n;
+    fill_tables(T2, T3, n);
+    __syncthreads();
     for (int64_t q = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; q < count; q += (int64_t)gridDim.x * blockDim.x) {
         const int64_t r = ranks[q];
         if (r < 0 || r >= (int64_t)M) { *bad = 1; out[3 * q] = out[3 * q + 1] = out[3 * q + 2] = -1; continue; }
         int a, b, c;
-        unrank<K>((uint32_t)r, n, M, a, b, c);
+        if (tab) unrank_tab<K>((uint32_t)r, n, M, T2, T3, a, b, c);
+        else unrank<K>((uint32_t)r, n, M, a, b, c);
         out[3 * q] = a; out[3 * q + 1] = b; out[3 * q + 2] = c;
     }
 }
@@ -1399,15 +1481,26 @@ lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count,
     cudaMemcpyAsync(d_r, ranks, count * 8, cudaMemcpyDefault, st);
     cudaMemsetAsync(d_bad, 0, 4, st);
     const int blocks = (int)std::min<int64_t>((count + 255) / 256, 4096);
-    if (k == 1) k_unrank<1><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
-    else if (k == 2) k_unrank<2><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
-    else k_unrank<3><<<blocks, 256, 0, st>>>(n, (uint32_t)Mk, d_r, count, d_o, d_bad);
+    const size_t tsm = 8 * (size_t)n;
+    // both the hot-path (table) unranking and the 64-bit reference; they must agree
+    int32_t *d_o2 = nullptr;
+    if (cudaMalloc(&d_o2, count * 12) != cudaSuccess) { cudaFree(d_r); cudaFree(d_o); cudaFree(d_bad); cudaGetLastError(); return fail(LNS_ENOMEM, "cudaMalloc failed"); }
+    for (int tab = 0; tab < 2; tab++) {
+        int32_t *o = tab ? d_o : d_o2;
+        if (k == 1) k_unrank<1><<<blocks, 256, tsm, st>>>(n, (uint32_t)Mk, d_r, count, o, d_bad, tab);
+        else if (k == 2) k_unrank<2><<<blocks, 256, tsm, st>>>(n, (uint32_t)Mk, d_r, count, o, d_bad, tab);
+        else k_unrank<3><<<blocks, 256, tsm, st>>>(n, (uint32_t)Mk, d_r, count, o, d_bad, tab);
+    }
+    std::vector<int32_t> h1((size_t)count * 3), h2((size_t)count * 3);
+    cudaMemcpyAsync(h1.data(), d_o, count * 12, cudaMemcpyDeviceToHost, st);
+    cudaMemcpyAsync(h2.data(), d_o2, count * 12, cudaMemcpyDeviceToHost, st);
     cudaMemcpyAsync(out, d_o, count * 12, cudaMemcpyDefault, st);
     cudaMemcpyAsync(&bad, d_bad, 4, cudaMemcpyDeviceToHost, st);
     const cudaError_t e = cudaStreamSynchronize(st);
-    cudaFree(d_r); cudaFree(d_o); cudaFree(d_bad);
+    cudaFree(d_r); cudaFree(d_o); cudaFree(d_o2); cudaFree(d_bad);
     if (e != cudaSuccess) return fail(LNS_ECUDA, cudaGetErrorString(e));
     if (bad) return fail(LNS_EINVAL, "rank out of range");
+    if (h1 != h2) return fail(LNS_ECUDA, "table and reference unranking disagree");
     return LNS_OK;
 }
 
