@@ -298,3 +298,31 @@ def test_C5_two_iterations_properties(L, orc):
         V[f3] *= -1
         assert orc.fitness(inst.A, inst.S, V, packed=True) == tf[t]
     assert np.array_equal(V, Vo)
+
+
+def test_python_partitioned_driver_with_nccl_world1(L, orc):
+    """parallel.partitioned_tabu_run + LnsStepper over a real NCCL process group (world 1): the
+    Python-driven protocol gives the oracle trajectory."""
+    import os
+
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_ipps_luongmt10_b200 import parallel as par
+
+    os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+    os.environ.setdefault("MASTER_PORT", "29533")
+    dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
+    try:
+        inst = pi.config_instance("C3")
+        V0 = pi.start_vector(81, 3)
+        ctx = L.lns_create(inst.A, inst.S)
+        try:
+            st = par.LnsStepper(ctx, 81, 3, 30, -1, 0, V0, stop_on_zero=False, rank=0, world=1)
+            tr, tf, Vo, res = par.partitioned_tabu_run(st, 30)
+        finally:
+            L.lns_destroy(ctx)
+        otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0, 30, pi.default_tenure(81, 3), stop_on_zero=False)
+        assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+    finally:
+        dist.destroy_process_group()
