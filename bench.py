@@ -59,7 +59,7 @@ def peaks():
 
 
 class ClockSampler:
-    """nvidia-smi clocks and throttle reasons sampled every 200 ms during the timed region."""
+    """nvidia-smi clocks and throttle reasons sampled every 50 ms during the timed region."""
 
     FIELDS = ["clocks.sm", "clocks.max.sm", "power.draw", "clocks_event_reasons.hw_slowdown",
               "clocks_event_reasons.hw_thermal_slowdown", "clocks_event_reasons.sw_thermal_slowdown",
@@ -76,7 +76,7 @@ class ClockSampler:
         try:
             self.proc = subprocess.Popen(
                 ["nvidia-smi", f"--query-gpu={','.join(self.FIELDS)}", "--format=csv,noheader,nounits",
-                 "-lms", "200", "-i", str(self.gpu)], stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+                 "-lms", "50", "-i", str(self.gpu)], stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
         except OSError:
             self.proc = None
         time.sleep(0.3)
@@ -293,7 +293,7 @@ def main():
     achieved = (iters * M / world) * ops_per_nbr / kern_avg_s / 1e12  # per-GPU share of the work
     peak = sms * 128 * mhz * 1e6 / 1e12  # 128 integer lanes issued per SM per clock (4 SMSP x 1 warp-instr)
     traffic = None
-    prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_C4.json")
+    prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_C4.json")  # ncu --set full of the bench step
     if os.path.exists(prof):
         try:
             with open(prof) as fh:
@@ -324,8 +324,8 @@ def main():
             "tabu_iters_per_s": iters_done / (total_ms / 1e3),
             "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
-            # our kernels per timed step: k_fill_i64 + k_init + (1 persistent k_search | 2 per iteration stepped)
-            "gpu_launches": args.steps * (3 if world == 1 else 2 + 2 * iters),
+            # our kernels per timed step: 2 x k_fill_i64 + k_init + (1 persistent k_search | 2 per iteration stepped)
+            "gpu_launches": args.steps * (4 if world == 1 else 2 + 2 * iters),
             "clocks": clocks,
             "roofline": roofline,
             "cpu_baseline": cpu,
