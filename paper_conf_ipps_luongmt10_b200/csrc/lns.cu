@@ -87,7 +87,9 @@ struct SearchArgs {
     int64_t L;              // tenure
     int32_t stop_on_zero;
     int32_t a_in_smem;      // stage A's bit rows in shared memory
-    int32_t until_smem;     // cache the CTA's until[] slice in shared memory (capacity in entries, 0 = no)
+    int32_t until_smem;     // cache the CTA's until[] slice in shared memory (1 = yes)
+    int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
+    int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     uint32_t *vb;           // state: NWn words of V's sign bits
     int32_t *Y;             // state: m
     int64_t *fs;            // FS_N
@@ -119,7 +121,7 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
     s.pofs = o;   o = align16(o + 4 * (n + 2));
     s.rowAt = o;  o = align16(o + 4 * m);
     s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
-    s.pieces = o; o = align16(o + 8 * (n + 1 + W));      // P <= U + W - 1 pieces
+    s.pieces = o; o = align16(o + 8 * (n + 2 + W));      // P <= U + W - 1 pieces (+1 prefetch pad)
     s.pstart = o; o = align16(o + 4 * (W + 1));
     s.T2 = o;     o = align16(o + 4 * n);                // C(y,2), y < n (u32)
     s.T3 = o;     o = align16(o + 4 * n);                // C(z,3), z < n (u32: C(n,3) < 2^32)
@@ -298,7 +300,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             int inc = v;
             for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, inc, o); if (lane >= o) inc += t; }
             const int st = runr + inc - v, en = runr + inc;
-            const int np = v > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : 1;  // empty point: one zero piece
+            const int np = v_ < U ? (v > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : 1) : 0;  // empty point: one zero piece
             int incp = np;
             for (int o = 1; o < 32; o <<= 1) { int t = __shfl_up_sync(FULL, incp, o); if (lane >= o) incp += t; }
             if (v_ < U) { seg[v_] = st; cur[u] = st; pofs[v_] = runp + incp - np; }
@@ -369,16 +371,20 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
 // counts N_t land in bins beta + 2t and bin beta is complete. Registers Ra.. hold bins
 // beta .. beta+2K-1; the caller rotates the names (Ra becomes bin beta+2K), so no moves are needed.
 template <int K>
-__device__ __forceinline__ void seg_step(const uint2 *__restrict__ &pp, const int2 *__restrict__ &bp,
+__device__ __forceinline__ void seg_step(const uint2 *__restrict__ &pp, uint2 &rec, const int2 *__restrict__ &bp,
                                          const uint32_t *__restrict__ X, int n, int a, int b, int c, int &curw,
                                          uint32_t &lo, uint32_t &hi, uint32_t &lh, int &f, int &smin,
                                          int &Ra, int &Rc, int &Re)
 {
     int c1 = 0, c2 = 0, c3 = 0;
-    uint2 rec;
+    const int2 bn = *bp++;  // this segment's bin constants, loaded early
+    uint2 cur;
     do {
-        rec = *pp++;
-        const int w = (int)((rec.y >> 1) & 0x7fffu);
+        // rec holds the current piece (prefetched); fetch the next one before using it (the piece
+        // list is padded, so reading one past the last piece is safe)
+        cur = rec;
+        rec = *++pp;
+        const int w = (int)((cur.y >> 1) & 0x7fffu);
         if (w != curw) {
             curw = w;
             const uint32_t *xr = X + w * n;
@@ -394,11 +400,11 @@ __device__ __forceinline__ void seg_step(const uint2 *__restrict__ &pp, const in
                 lh = lo & hi;
             }
         }
-        c1 += __popc(lo & rec.x);
-        if (K >= 2) c2 += __popc(hi & rec.x);
-        if (K == 3) c3 += __popc(lh & rec.x);
-    } while (!(rec.y & 1u));
-    const int len = (int)(rec.y >> 16);
+        c1 += __popc(lo & cur.x);
+        if (K >= 2) c2 += __popc(hi & cur.x);
+        if (K == 3) c3 += __popc(lh & cur.x);
+    } while (!(cur.y & 1u));
+    const int len = (int)(cur.y >> 16);
     int h;
     if (K == 1) {         // N1 = c1 -> bin beta+2 (reuses Ra)
         h = Ra + len - c1;
@@ -410,7 +416,6 @@ __device__ __forceinline__ void seg_step(const uint2 *__restrict__ &pp, const in
         h = Ra + len - c1 - c2 + c3;
         Rc += c1 - c3; Re += c2 - c3; Ra = c3;
     }
-    const int2 bn = *bp++;
     f += bn.y * h;
     smin += min(h, bn.x);
 }
@@ -433,9 +438,10 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
     int curw = -1;
     uint32_t lo = 0, hi = 0, lh = 0;
     const uint2 *pp = pieces;
+    uint2 rec = *pp;
     const int2 *bp = bins;
     int u = 0;
-#define SEG(Ra, Rc, Re) seg_step<K>(pp, bp, X, n, a, b, c, curw, lo, hi, lh, f, smin, Ra, Rc, Re)
+#define SEG(Ra, Rc, Re) seg_step<K>(pp, rec, bp, X, n, a, b, c, curw, lo, hi, lh, f, smin, Ra, Rc, Re)
 #define TRAIL2(A, B) { bin_cost(A, bp[0], f, smin); bin_cost(B, bp[1], f, smin); }
 #define TRAIL4(A, B, C, D) { TRAIL2(A, B) bin_cost(C, bp[2], f, smin); bin_cost(D, bp[3], f, smin); }
 #define TRAIL6(A, B, C, D, E, F) { TRAIL4(A, B, C, D) bin_cost(E, bp[4], f, smin); bin_cost(F, bp[5], f, smin); }
@@ -473,7 +479,7 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
 template <int K, bool WRITE_ALL>
 __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L, int U,
                                          uint32_t M, uint32_t blo, uint32_t bhi, const uint32_t *until,
-                                         uint32_t ubase, uint32_t t, int32_t *fit_out)
+                                         uint32_t ubase, uint32_t t, int32_t *fit_out, const uint2 *tri = nullptr)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
@@ -487,7 +493,12 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const bool is_tabu = until && until[r - ubase] >= t;
             if (!is_tabu || WRITE_ALL) {
                 int a, b, c;
-                unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
+                if (tri) {  // flip sets of this CTA's fixed slice, precomputed at launch
+                    const uint2 q = tri[r - blo];
+                    a = (int)(q.x & 0xffffu); b = (int)(q.x >> 16); c = (int)q.y;
+                } else {
+                    unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
+                }
                 const int f = eval_fit<K>(X, pieces, bins, I.n, U, 2 * I.m, a, b, c);
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
@@ -635,6 +646,18 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         ubase = blo;
     }
     const uint32_t *Ar = load_state<K>(A, sm, L, ps);
+    const uint2 *tri = nullptr;
+    if (A.tri_smem) {
+        uint2 *ts = (uint2 *)(sm + L.a_end + 4 * A.slice_cap);
+        const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
+        for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) {
+            int a, b, c;
+            unrank_tab<K>(r, A.I.n, A.M, T2, T3, a, b, c);
+            ts[r - blo] = make_uint2((uint32_t)(a & 0xffff) | ((uint32_t)(b & 0xffff) << 16), (uint32_t)c);
+        }
+        __syncthreads();
+        tri = ts;
+    }
 #ifdef LNS_PHASE_TIMING
     if (threadIdx.x == 0) { for (int i = 0; i < NPH; i++) s_ph[i] = 0; s_last = clock64(); }
 #endif
@@ -646,7 +669,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     for (; t <= t0 + A.iters; t++) {
         if (A.stop_on_zero && f == 0) break;
         build_plan<K>(A.I, Ar, sm, L, ps);
-        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps.U, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr);
+        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps.U, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr, tri);
         mine = warp_min_k(mine);
         if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
         __syncthreads();
@@ -660,14 +683,23 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             // CTA 0 resets it here for iteration t+2.
             if (threadIdx.x == 0) {
                 unsigned long long *slot = (unsigned long long *)A.slots + 16 * (t % 3);
-                if (key != (unsigned long long)KEY_NONE) atomicMin(slot, key);
-                __threadfence();
-                atomicAdd((unsigned long long *)A.slots + 48, 1ull);
+                unsigned long long *ctr = (unsigned long long *)A.slots + 48;
+                if (key != (unsigned long long)KEY_NONE)
+                    asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
+                // the release orders the MIN above before the arrival; the acquire below orders
+                // the slot read after every CTA's arrival (and hence its MIN)
+                asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
                 const unsigned long long target = (unsigned long long)nb * (unsigned long long)(t - t0);
-                volatile unsigned long long *ctr = (volatile unsigned long long *)A.slots + 48;
-                while (*ctr < target) { }
-                ps.gkey = *(volatile unsigned long long *)slot;
-                if (bid == 0) *((volatile unsigned long long *)A.slots + 16 * ((t + 2) % 3)) = (unsigned long long)KEY_NONE;
+                unsigned long long seen;
+                do {
+                    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+                } while (seen < target);
+                unsigned long long g;
+                asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(g) : "l"(slot) : "memory");
+                ps.gkey = g;
+                if (bid == 0)
+                    asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"((unsigned long long *)A.slots + 16 * ((t + 2) % 3)),
+                                 "l"((unsigned long long)KEY_NONE) : "memory");
             }
             __syncthreads();
             key = ps.gkey;
@@ -979,7 +1011,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.a_in_smem = g.a_in_smem;
-    A.until_smem = 0;
+    A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     return A;
@@ -1047,9 +1079,13 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
     const int nb = search_blocks(c, A.hi - A.lo, 1);
-    const uint64_t slice = ((uint64_t)(A.hi - A.lo) + nb - 1) / nb + 64;
+    const uint64_t slice = ((((uint64_t)(A.hi - A.lo) + nb - 1) / nb + 64) + 3) & ~3ull;  // 16-B aligned caches
     size_t smem = g.smem_eval;
-    if (g.smem_eval + 4 * slice <= (size_t)budget) {
+    A.slice_cap = (int32_t)std::min<uint64_t>(slice, 1u << 30);
+    if (g.smem_eval + 12 * slice <= (size_t)budget) {  // until[] slice + flip-set table
+        A.until_smem = 1; A.tri_smem = 1;
+        smem = g.smem_eval + 12 * slice;
+    } else if (g.smem_eval + 4 * slice <= (size_t)budget) {
         A.until_smem = 1;
         smem = g.smem_eval + 4 * slice;
     }
