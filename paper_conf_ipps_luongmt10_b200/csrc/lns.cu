@@ -28,6 +28,7 @@
 
 #include <algorithm>
 #include <climits>
+#include <cstdlib>
 #include <cmath>
 #include <cstdio>
 #include <cstring>
@@ -74,6 +75,7 @@ struct DevInst {
     int32_t m, n, W, NWn;  // W = ceil(m/32) row words, NWn = ceil(n/32) column words
     const uint32_t *Arow;  // m x NWn, bit (i%32) of word i/32 = 1 <=> A[j][i] = -1
     const int32_t *H;      // n+1 bins of S
+    int32_t maxS;          // largest b with H_b > 0
 };
 
 // fstate layout (int64): current f, iterations done, best f, best iter, first zero iter, done, error
@@ -90,6 +92,7 @@ struct SearchArgs {
     int32_t until_smem;     // cache the CTA's until[] slice in shared memory (1 = yes)
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
+    int32_t no_split;       // 1: evaluate every lattice point (disable the linear-region shortcuts)
     uint32_t *vb;           // state: NWn words of V's sign bits
     int32_t *Y;             // state: m
     int64_t *fs;            // FS_N
@@ -134,6 +137,10 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
 
 struct PlanScalars {
     int vmin, U, NB, P, ufirst;
+    // linear regions: lattice points u < uneg are "deep negative" (all k+1
+    // destinations negative: cost linear, aggregated as cneg - 240 sum t over the first rneg sorted
+    // rows); points u >= utop land only above max(S) (zero cost) and are skipped
+    int uneg, utop, rneg, cneg;
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
     unsigned long long key, gkey;
     int red[2 * NWARP + 2];
@@ -307,10 +314,17 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             runr += __shfl_sync(FULL, inc, 31);
             runp += __shfl_sync(FULL, incp, 31);
         }
+        // deep-negative prefix: points with value v < -2K (v = vlo + 2(uf + u))
+        const int vmin_ = vlo + 2 * uf;
+        int uneg = (-2 * K - vmin_ + 1) >> 1;  // least u with vmin + 2u >= -2K
+        uneg = min(max(uneg, 0), U);
+        int utop = ((I.maxS + 2 * K - vmin_) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
+        utop = min(max(utop, uneg), U);
         if (lane == 0) {
-            const int vmin = vlo + 2 * uf;
-            seg[U] = runr; ps.P = runp; pstart[W] = runp;
+            const int vmin = vmin_;
+            seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[W] = runp;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
+            ps.uneg = uneg; ps.utop = utop; ps.cneg = 0;
             ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
             ps.key = (unsigned long long)KEY_NONE;
             ps.gkey = (unsigned long long)KEY_NONE;
@@ -320,13 +334,19 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     PH(1);
     // C. place rows; emit pieces (one thread per segment); bin constants
     const int vmin = ps.vmin, U = ps.U, NB = ps.NB, uf = ps.ufirst;
+    if (tid == 0) ps.rneg = seg[ps.uneg];
     for (int j = tid; j < m; j += NT) {
         const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
         rowAt[p] = j;
     }
+    const int uneg = ps.uneg;
     for (int v = tid; v < U; v += NT) {
         const int st = seg[v], en = seg[v + 1];
         int p = pofs[v];
+        // deep-negative constant sum_rows 60(2K - Y_j) - 1 (unsigned: the constant may exceed
+        // 2^31 on its own; the fitness it enters does not)
+        if (v < uneg && en > st)
+            atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - 1));
         if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
             pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
             continue;
@@ -429,17 +449,46 @@ __device__ __forceinline__ void bin_cost(int h, int2 bn, int &f, int &smin)
 // Fitness of neighbour (a, b, c) from the plan, segment-major over the U lattice points:
 //   f = 2m + sum_beta ( w_beta h_beta - 2 min(h_beta, H_beta) )
 // (|h - H| = h + H - 2 min(h, H) summed over b = 0..n; every row lands in exactly one bin.)
-template <int K>
+struct EvalRange {
+    int u0, u1;       // lattice points [u0, u1) go through the segment loop (u0 = uneg, u1 = utop)
+    int rneg, cneg;   // deep-negative rows [0, rneg) and their constant part
+    int p0;           // first piece of point u0
+};
+
+template <int K, bool DEEP>
 __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
-                                        const int2 *__restrict__ bins, int n, int U, int m2, int a, int b, int c)
+                                        const int2 *__restrict__ bins, int n, const EvalRange &er, int m2,
+                                        int a, int b, int c)
 {
     int f = m2, smin = 0;
+    // deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
+    //   = cneg - 240 sum_j t_j, with sum t = popc(lo) + 2 popc(hi) over their (sorted) row words
+    if (DEEP) {
+        int st = 0;
+        const int nw = (er.rneg + 31) >> 5;
+        for (int w = 0; w < nw; w++) {
+            const uint32_t mask = (w == nw - 1 && (er.rneg & 31)) ? ((1u << (er.rneg & 31)) - 1u) : FULL;
+            const uint32_t *xr = X + w * n;
+            if (K == 1) {
+                st += __popc(xr[a] & mask);
+            } else if (K == 2) {
+                const uint32_t xa = xr[a], xb = xr[b];
+                st += __popc((xa ^ xb) & mask) + 2 * __popc(xa & xb & mask);
+            } else {
+                const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+                st += __popc((xa ^ xb ^ xc) & mask) + 2 * __popc(((xa & xb) | (xc & (xa ^ xb))) & mask);
+            }
+        }
+        f = (int)((unsigned)f + (unsigned)er.cneg - 240u * (unsigned)st);
+    }
+    const int U = er.u1 - er.u0;
+    if (U <= 0) return f;
     int R0 = 0, R1 = 0, R2 = 0, R3 = 0, R4 = 0, R5 = 0;
     int curw = -1;
     uint32_t lo = 0, hi = 0, lh = 0;
-    const uint2 *pp = pieces;
+    const uint2 *pp = pieces + er.p0;
     uint2 rec = *pp;
-    const int2 *bp = bins;
+    const int2 *bp = bins + er.u0;
     int u = 0;
 #define SEG(Ra, Rc, Re) seg_step<K>(pp, rec, bp, X, n, a, b, c, curw, lo, hi, lh, f, smin, Ra, Rc, Re)
 #define TRAIL2(A, B) { bin_cost(A, bp[0], f, smin); bin_cost(B, bp[1], f, smin); }
@@ -477,15 +526,21 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
 // key. until (nullable) is indexed by r - ubase: rank r is tabu iff until[r - ubase] >= t.
 template <int K, bool WRITE_ALL>
-__device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L, int U,
-                                         uint32_t M, uint32_t blo, uint32_t bhi, const uint32_t *until,
-                                         uint32_t ubase, uint32_t t, int32_t *fit_out, const uint2 *tri = nullptr)
+__device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
+                                         const PlanScalars &ps, uint32_t M, uint32_t blo, uint32_t bhi,
+                                         const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
+                                         const uint2 *tri = nullptr, int no_split = 0)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
     const uint2 *pieces = (const uint2 *)(sm + L.pieces);
     const int2 *bins = (const int2 *)(sm + L.bins);
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
+    EvalRange er;
+    er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
+    er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
+    if (no_split & 1) { er.u0 = 0; er.u1 = ps.U; er.rneg = 0; er.cneg = 0; er.p0 = 0; }
+    if (no_split & 2) er.u1 = ps.U;
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
@@ -499,7 +554,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 } else {
                     unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
                 }
-                const int f = eval_fit<K>(X, pieces, bins, I.n, U, 2 * I.m, a, b, c);
+                const int f = er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
+                                          : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c);
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 if (!is_tabu && key < best) best = key;
@@ -669,7 +725,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     for (; t <= t0 + A.iters; t++) {
         if (A.stop_on_zero && f == 0) break;
         build_plan<K>(A.I, Ar, sm, L, ps);
-        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps.U, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr, tri);
+        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr, tri, A.no_split);
         mine = warp_min_k(mine);
         if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
         __syncthreads();
@@ -755,7 +811,7 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
     cta_slice(A.lo, A.hi, blockIdx.x, gridDim.x, blo, bhi);
     build_plan<K>(A.I, Ar, sm, L, ps);
     const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
-    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps.U, A.M, blo, bhi, A.until, 0, t, fit_out);
+    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps, A.M, blo, bhi, A.until, 0, t, fit_out);
     mine = warp_min_k(mine);
     if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
     __syncthreads();
@@ -875,7 +931,7 @@ typedef int (*nccl_allreduce_fn)(const void *, void *, size_t, int, int, void *,
 
 struct lns_ctx {
     int device = 0;
-    int m = 0, n = 0, W = 0, NWn = 0;
+    int m = 0, n = 0, W = 0, NWn = 0, maxS = 0;
     uint32_t *d_Arow = nullptr;
     int32_t *d_H = nullptr;
     int numSMs = 0, smemOptin = 0;
@@ -930,7 +986,7 @@ int64_t comb_k(int64_t n, int k)
     return -1;
 }
 
-DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->d_Arow, c->d_H}; }
+DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->d_Arow, c->d_H, c->maxS}; }
 
 template <typename T>
 lns_status grow(T *&p, size_t &cap, size_t need)
@@ -1012,6 +1068,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
+    A.no_split = getenv("LNS_NO_SPLIT") ? atoi(getenv("LNS_NO_SPLIT")) : 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     return A;
@@ -1222,6 +1279,8 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     }
     lns_ctx *c = new lns_ctx();
     c->device = device; c->m = m; c->n = n; c->W = W; c->NWn = NWn;
+    for (int b = 0; b <= n; b++)
+        if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };
     if (cudaDeviceGetAttribute(&c->numSMs, cudaDevAttrMultiProcessorCount, device) != cudaSuccess ||
         cudaDeviceGetAttribute(&c->smemOptin, cudaDevAttrMaxSharedMemoryPerBlockOptin, device) != cudaSuccess)

@@ -2,7 +2,7 @@
 import os, sys, ctypes
 sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 from paper_conf_ipps_luongmt10_b200 import _build
-os.environ["LNS_LIB"] = _build.LIB_PROF
+os.environ["LNS_LIB"] = os.environ.get("LNS_PROF_LIB") or _build.LIB_PROF
 import numpy as np
 import paper_conf_ipps_luongmt10_b200 as L, ppp_inputs as pi
 names = ["A count+bins", "B scans", "C place+pieces", "D X build", "eval+reduce", "exchange", "apply", "-"]
