@@ -93,6 +93,13 @@ struct SearchArgs {
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     int32_t no_split;       // 1: evaluate every lattice point (disable the linear-region shortcuts)
+    // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
+    // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
+    // search from the state in (vb, Y, fs).
+    int32_t groups, R;
+    const int8_t *V0s;      // R x n
+    int64_t *res;           // R x FS_N
+    uint32_t *vouts;        // R x NWn
     uint32_t *vb;           // state: NWn words of V's sign bits
     int32_t *Y;             // state: m
     int64_t *fs;            // FS_N
@@ -137,6 +144,7 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
 
 struct PlanScalars {
     int vmin, U, NB, P, ufirst;
+    int fpen, fhd;  // block_fitness accumulators
     // linear regions: lattice points u < uneg are "deep negative" (all k+1
     // destinations negative: cost linear, aggregated as cneg - 240 sum t over the first rneg sorted
     // rows); points u >= utop land only above max(S) (zero cost) and are skipped
@@ -594,24 +602,16 @@ __device__ __forceinline__ void cta_slice(uint32_t lo, uint32_t hi, unsigned b, 
     bhi = (b + 1 == nb) ? hi : lo + 32u * (uint32_t)((span * (b + 1) / nb) / 32);
 }
 
-// Stage the state (and A's bits when A.a_in_smem) into shared memory, zero cnt[] and publish the
-// range of Y; returns A's bit rows.
+// Stage the instance parts (H, A's bits when A.a_in_smem, unranking tables) into shared memory and
+// zero cnt[]; returns A's bit rows. No barrier: callers follow with one.
 template <int K>
-__device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, const Smem &L, PlanScalars &ps)
+__device__ const uint32_t *load_common(const SearchArgs &A, unsigned char *sm, const Smem &L)
 {
-    int *Ys = (int *)(sm + L.Y);
-    uint32_t *vbs = (uint32_t *)(sm + L.vb);
     int *Hs = (int *)(sm + L.H);
     int *cnt = (int *)(sm + L.cnt);
-    int mn = INT_MAX, mx = INT_MIN;
-    for (int j = threadIdx.x; j < A.I.m; j += NT) {
-        const int y = A.Y[j];
-        Ys[j] = y;
-        mn = min(mn, y); mx = max(mx, y);
-    }
-    for (int w = threadIdx.x; w < A.I.NWn; w += NT) vbs[w] = A.vb[w];
+    int *cur = (int *)(sm + L.cur);
     for (int b = threadIdx.x; b <= A.I.n; b += NT) Hs[b] = A.I.H[b];
-    for (int u = threadIdx.x; u < A.I.n + 2 + 2 * K; u += NT) cnt[u] = 0;
+    for (int u = threadIdx.x; u < A.I.n + 2 + 2 * K; u += NT) { cnt[u] = 0; cur[u] = 0; }
     fill_tables((uint32_t *)(sm + L.T2), (uint32_t *)(sm + L.T3), A.I.n);
     const uint32_t *Ar = A.I.Arow;
     if (A.a_in_smem) {
@@ -620,6 +620,60 @@ __device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, co
         for (int q = threadIdx.x; q < nw; q += NT) As[q] = __ldg(A.I.Arow + q);
         Ar = As;
     }
+    return Ar;
+}
+
+// Start a restart inside the CTA: V bits from the int8 vector V0, Y = A V0 (<a_j, v> = n - 2
+// popcount(a xor v)), the range of Y, and f from scratch into ps.fpen/fhd:
+// f = 30 fpen + fhd. Uses cur[] (n+1 zeroed entries) as the histogram and leaves it zeroed.
+template <int K>
+__device__ void init_restart(const SearchArgs &A, const uint32_t *Ar, const int8_t *V0, unsigned char *sm,
+                             const Smem &L, PlanScalars &ps)
+{
+    int *Ys = (int *)(sm + L.Y);
+    uint32_t *vbs = (uint32_t *)(sm + L.vb);
+    const int *Hs = (const int *)(sm + L.H);
+    int *hist = (int *)(sm + L.cur);
+    for (int w = threadIdx.x; w < A.I.NWn; w += NT) vbs[w] = 0u;
+    for (int b = threadIdx.x; b <= A.I.n; b += NT) hist[b] = 0;  // cur[] holds the last plan's cursors
+    if (threadIdx.x == 0) { ps.fpen = 0; ps.fhd = 0; }
+    __syncthreads();
+    for (int i = threadIdx.x; i < A.I.n; i += NT)
+        if (V0[i] < 0) atomicOr(&vbs[i >> 5], 1u << (i & 31));
+    __syncthreads();
+    int mn = INT_MAX, mx = INT_MIN, pen = 0;
+    for (int j = threadIdx.x; j < A.I.m; j += NT) {
+        const uint32_t *ar = Ar + (size_t)j * A.I.NWn;
+        int d = 0;
+        for (int w = 0; w < A.I.NWn; w++) d += __popc(ar[w] ^ vbs[w]);
+        const int y = A.I.n - 2 * d;
+        Ys[j] = y;
+        mn = min(mn, y); mx = max(mx, y);
+        if (y < 0) pen += -2 * y;
+        else atomicAdd(&hist[y], 1);
+    }
+    atomicAdd(&ps.fpen, pen);
+    range_publish<K>(mn, mx, ps);  // includes a __syncthreads: the histogram is complete
+    int hd = 0;
+    for (int b = threadIdx.x; b <= A.I.n; b += NT) { hd += abs(Hs[b] - hist[b]); hist[b] = 0; }
+    atomicAdd(&ps.fhd, hd);
+    __syncthreads();
+}
+
+// Stage the state (vb, Y) of a single search into shared memory and publish the range of Y.
+template <int K>
+__device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, const Smem &L, PlanScalars &ps)
+{
+    int *Ys = (int *)(sm + L.Y);
+    uint32_t *vbs = (uint32_t *)(sm + L.vb);
+    const uint32_t *Ar = load_common<K>(A, sm, L);
+    int mn = INT_MAX, mx = INT_MIN;
+    for (int j = threadIdx.x; j < A.I.m; j += NT) {
+        const int y = A.Y[j];
+        Ys[j] = y;
+        mn = min(mn, y); mx = max(mx, y);
+    }
+    for (int w = threadIdx.x; w < A.I.NWn; w += NT) vbs[w] = A.vb[w];
     range_publish<K>(mn, mx, ps);
     __syncthreads();
     return Ar;
@@ -678,7 +732,8 @@ __global__ void __launch_bounds__(NT) k_init(DevInst I, const int8_t *V0, uint32
     }
 }
 
-// The persistent tabu search: all iterations in one cooperative launch.
+// The persistent tabu search: all iterations in one cooperative launch. With A.R > 0 the grid is
+// split into A.groups groups; each group runs its restarts one after another (batched restarts).
 template <int K>
 __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
@@ -687,21 +742,28 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
-    const int nb = (int)gridDim.x, bid = (int)blockIdx.x;
+    const int G = A.groups > 0 ? A.groups : 1;
+    const int nb = (int)gridDim.x / G;
+    const int g = (int)blockIdx.x / nb, bid = (int)blockIdx.x - g * nb;
+    if (g >= G) return;
+    const bool batch = A.R > 0;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const bool leader = (bid == 0 && threadIdx.x == 0);
+    unsigned long long *gslots = (unsigned long long *)A.slots + 64 * (size_t)g;
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, bid, nb, blo, bhi);
-    // the CTA's until[] slice: shared-memory copy when it fits, else the global array
-    uint32_t *until = A.until;
+    // the CTA's until[] slice: shared-memory copy when it fits, else the group's global array
+    uint32_t *until = A.until + (batch ? (size_t)g * A.M : 0);
     uint32_t ubase = 0;
     if (A.until_smem) {
         uint32_t *us = (uint32_t *)(sm + L.a_end);
-        for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) us[r - blo] = A.until[r];
+        if (!batch)
+            for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) us[r - blo] = A.until[r];
         until = us;
         ubase = blo;
     }
-    const uint32_t *Ar = load_state<K>(A, sm, L, ps);
+    const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
+    __syncthreads();
     const uint2 *tri = nullptr;
     if (A.tri_smem) {
         uint2 *ts = (uint2 *)(sm + L.a_end + 4 * A.slice_cap);
@@ -717,80 +779,107 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 #ifdef LNS_PHASE_TIMING
     if (threadIdx.x == 0) { for (int i = 0; i < NPH; i++) s_ph[i] = 0; s_last = clock64(); }
 #endif
-    int64_t f = A.fs[FS_F];
-    int64_t best_f = A.fs[FS_BEST], best_it = A.fs[FS_BESTIT], zero_it = A.fs[FS_ZERO];
-    const int64_t t0 = A.fs[FS_T];
-    int64_t t = t0 + 1;
-    bool failed = false;
-    for (; t <= t0 + A.iters; t++) {
-        if (A.stop_on_zero && f == 0) break;
-        build_plan<K>(A.I, Ar, sm, L, ps);
-        unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, until, ubase, (uint32_t)t, nullptr, tri, A.no_split);
-        mine = warp_min_k(mine);
-        if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
-        __syncthreads();
-        PH(4);
-        unsigned long long key = ps.key;
-        if (nb > 1) {
-            // exchange: u64 MIN of this CTA's key into slot t%3 (each slot on its own 128-B line),
-            // then one arrival on a monotonic 64-bit counter; when the counter reaches
-            // nb * (t - t0) every CTA's MIN has landed and the slot holds the global minimum.
-            // Slot (t+2)%3 was last read in iteration t-1 by CTAs that have all arrived at t, so
-            // CTA 0 resets it here for iteration t+2.
-            if (threadIdx.x == 0) {
-                unsigned long long *slot = (unsigned long long *)A.slots + 16 * (t % 3);
-                unsigned long long *ctr = (unsigned long long *)A.slots + 48;
-                if (key != (unsigned long long)KEY_NONE)
-                    asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
-                // the release orders the MIN above before the arrival; the acquire below orders
-                // the slot read after every CTA's arrival (and hence its MIN)
-                asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
-                const unsigned long long target = (unsigned long long)nb * (unsigned long long)(t - t0);
-                unsigned long long seen;
-                do {
-                    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
-                } while (seen < target);
-                unsigned long long g;
-                asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(g) : "l"(slot) : "memory");
-                ps.gkey = g;
-                if (bid == 0)
-                    asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"((unsigned long long *)A.slots + 16 * ((t + 2) % 3)),
-                                 "l"((unsigned long long)KEY_NONE) : "memory");
-            }
+    unsigned long long tg = 0;  // iterations run by this group in this launch (exchange clock)
+    for (int rs = batch ? g : 0; rs < (batch ? A.R : 1); rs += G) {
+        int64_t f, best_f, best_it, zero_it, t0;
+        if (batch) {
+            init_restart<K>(A, Ar, A.V0s + (size_t)rs * A.I.n, sm, L, ps);
+            for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) until[r - ubase] = 0u;
             __syncthreads();
-            key = ps.gkey;
+            f = 30 * (int64_t)ps.fpen + ps.fhd;
+            best_f = f; best_it = 0; zero_it = (f == 0) ? 0 : -1; t0 = 0;
+        } else {
+            f = A.fs[FS_F];
+            best_f = A.fs[FS_BEST]; best_it = A.fs[FS_BESTIT]; zero_it = A.fs[FS_ZERO];
+            t0 = A.fs[FS_T];
         }
-        PH(5);
-        if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
-        const uint32_t r = (uint32_t)(key & 0xffffffffu);
-        f = (int64_t)(key >> 32);
-        if (threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
-        if (leader) {
-            if (A.trace_r) A.trace_r[t - 1] = r;
-            if (A.trace_f) A.trace_f[t - 1] = f;
-            if (f < best_f) { best_f = f; best_it = t; }
-            if (f == 0 && zero_it < 0) zero_it = t;
+        int64_t t = t0 + 1;
+        bool failed = false;
+        for (; t <= t0 + A.iters; t++) {
+            if (A.stop_on_zero && f == 0) break;
+            build_plan<K>(A.I, Ar, sm, L, ps);
+            unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, until, ubase, (uint32_t)t,
+                                                           nullptr, tri, A.no_split);
+            mine = warp_min_k(mine);
+            if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
+            __syncthreads();
+            PH(4);
+            unsigned long long key = ps.key;
+            tg++;
+            if (nb > 1) {
+                // exchange: u64 MIN of this CTA's key into slot tg%3 (each slot on its own 128-B
+                // line), then one arrival on the group's monotonic 64-bit counter; when it reaches
+                // nb * tg every CTA's MIN has landed and the slot holds the group minimum. Slot
+                // (tg+2)%3 was last read one exchange earlier by CTAs that have all arrived now,
+                // so CTA 0 resets it here for exchange tg+2.
+                if (threadIdx.x == 0) {
+                    unsigned long long *slot = gslots + 16 * (tg % 3);
+                    unsigned long long *ctr = gslots + 48;
+                    if (key != (unsigned long long)KEY_NONE)
+                        asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
+                    // the release orders the MIN above before the arrival; the acquire below orders
+                    // the slot read after every CTA's arrival (and hence its MIN)
+                    asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
+                    const unsigned long long target = (unsigned long long)nb * tg;
+                    unsigned long long seen;
+                    do {
+                        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+                    } while (seen < target);
+                    unsigned long long gk;
+                    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
+                    ps.gkey = gk;
+                    if (bid == 0)
+                        asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(gslots + 16 * ((tg + 2) % 3)),
+                                     "l"((unsigned long long)KEY_NONE) : "memory");
+                }
+                __syncthreads();
+                key = ps.gkey;
+            }
+            PH(5);
+            if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
+            const uint32_t r = (uint32_t)(key & 0xffffffffu);
+            f = (int64_t)(key >> 32);
+            if (threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
+            if (leader) {
+                if (A.trace_r) A.trace_r[t - 1] = r;
+                if (A.trace_f) A.trace_f[t - 1] = f;
+                if (f < best_f) { best_f = f; best_it = t; }
+                if (f == 0 && zero_it < 0) zero_it = t;
+            }
+            int a, b, c;
+            unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), a, b, c);
+            apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
+            PH(6);
         }
-        int a, b, c;
-        unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), a, b, c);
-        apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
-        PH(6);
+        __syncthreads();  // the last move's V flip (thread 0) before V is written out / reused
+        if (batch) {
+            if (bid == 0) {
+                for (int w = threadIdx.x; w < A.I.NWn; w += NT) A.vouts[(size_t)rs * A.I.NWn + w] = vbs[w];
+                if (threadIdx.x == 0) {
+                    int64_t *o = A.res + (size_t)rs * FS_N;
+                    o[FS_F] = f; o[FS_T] = t - 1; o[FS_BEST] = best_f; o[FS_BESTIT] = best_it;
+                    o[FS_ZERO] = zero_it; o[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
+                    o[FS_ERR] = failed ? 2 : 0;
+                }
+            }
+        } else {
+            if (A.until_smem)
+                for (uint32_t q = blo + threadIdx.x; q < bhi; q += NT) A.until[q] = until[q - ubase];
+            if (bid == 0) {
+                for (int j = threadIdx.x; j < A.I.m; j += NT) A.Y[j] = Ys[j];
+                for (int w = threadIdx.x; w < A.I.NWn; w += NT) A.vb[w] = vbs[w];
+                if (threadIdx.x == 0) {
+                    A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
+                    A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
+                    if (failed) A.fs[FS_ERR] = 2;
+                }
+            }
+        }
     }
 #ifdef LNS_PHASE_TIMING
     if (threadIdx.x == 0)
         for (int i = 0; i < NPH; i++) atomicAdd(&g_ph[i], (unsigned long long)s_ph[i]);
 #endif
-    if (A.until_smem)
-        for (uint32_t q = blo + threadIdx.x; q < bhi; q += NT) A.until[q] = until[q - ubase];
-    if (bid == 0) {
-        for (int j = threadIdx.x; j < A.I.m; j += NT) A.Y[j] = Ys[j];
-        for (int w = threadIdx.x; w < A.I.NWn; w += NT) A.vb[w] = vbs[w];
-        if (threadIdx.x == 0) {
-            A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
-            A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
-            if (failed) A.fs[FS_ERR] = 2;
-        }
-    }
 }
 
 // Stepped mode, evaluation of iteration t = fs[FS_T] + 1: partial best key of this device's slice
@@ -951,6 +1040,10 @@ struct lns_ctx {
     uint32_t *d_until = nullptr; size_t until_cap = 0;
     int64_t *d_tr = nullptr, *d_tf = nullptr; size_t trace_cap = 0, trace_cap_f = 0;
     int32_t *d_fit = nullptr; size_t fit_cap = 0;
+    int8_t *d_V0s = nullptr; size_t v0s_cap = 0;       // batched restarts
+    int64_t *d_res = nullptr; size_t res_cap = 0;
+    uint32_t *d_vouts = nullptr; size_t vouts_cap = 0;
+    int64_t *d_gslots = nullptr; size_t gslots_cap = 0;
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
     double last_ms = 0.0;
     // stepped search
@@ -1068,6 +1161,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
+    A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
     A.no_split = getenv("LNS_NO_SPLIT") ? atoi(getenv("LNS_NO_SPLIT")) : 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
@@ -1125,6 +1219,24 @@ lns_status search_finish(lns_ctx *c, int8_t *V_out, int64_t *trace_rank, int64_t
     return LNS_OK;
 }
 
+// Shared-memory caches of a search with nb CTAs over [A.lo, A.hi): the until[] slice and the
+// flip-set table when they fit next to the plan. Returns the dynamic shared-memory bytes.
+size_t cache_geometry(SearchArgs &A, const Geometry &g, int nb, int budget)
+{
+    const uint64_t slice = ((((uint64_t)(A.hi - A.lo) + nb - 1) / nb + 64) + 3) & ~3ull;  // 16-B aligned caches
+    size_t smem = g.smem_eval;
+    A.slice_cap = (int32_t)std::min<uint64_t>(slice, 1u << 30);
+    A.until_smem = 0; A.tri_smem = 0;
+    if (g.smem_eval + 12 * slice <= (size_t)budget) {  // until[] slice + flip-set table
+        A.until_smem = 1; A.tri_smem = 1;
+        smem = g.smem_eval + 12 * slice;
+    } else if (g.smem_eval + 4 * slice <= (size_t)budget) {
+        A.until_smem = 1;
+        smem = g.smem_eval + 4 * slice;
+    }
+    return smem;
+}
+
 template <int K>
 lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st)
 {
@@ -1136,22 +1248,38 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
     const int nb = search_blocks(c, A.hi - A.lo, 1);
-    const uint64_t slice = ((((uint64_t)(A.hi - A.lo) + nb - 1) / nb + 64) + 3) & ~3ull;  // 16-B aligned caches
-    size_t smem = g.smem_eval;
-    A.slice_cap = (int32_t)std::min<uint64_t>(slice, 1u << 30);
-    if (g.smem_eval + 12 * slice <= (size_t)budget) {  // until[] slice + flip-set table
-        A.until_smem = 1; A.tri_smem = 1;
-        smem = g.smem_eval + 12 * slice;
-    } else if (g.smem_eval + 4 * slice <= (size_t)budget) {
-        A.until_smem = 1;
-        smem = g.smem_eval + 4 * slice;
-    }
+    const size_t smem = cache_geometry(A, g, nb, budget);
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
     k_fill_i64<<<1, 64, 0, st>>>(c->d_slots, KEY_NONE, 48);
     CK(cudaMemsetAsync(c->d_slots + 48, 0, 8, st));
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
     CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
+    CK(cudaEventRecord(c->ev1, st));
+    return LNS_OK;
+}
+
+// Batched restarts: G groups of nb CTAs (cooperative grid G * nb); A carries V0s / res / vouts.
+template <int K>
+lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int G, int nb, int64_t *gslots, cudaStream_t st)
+{
+    const int budget = c->smemOptin - 1024;
+    CK(cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, budget));
+    const size_t smem = cache_geometry(A, g, nb, budget);
+    if (!A.until_smem) {  // one global until[] per concurrent group
+        lns_status s = grow(c->d_until, c->until_cap, (size_t)G * g.M);
+        if (s != LNS_OK) return s;
+        A.until = c->d_until;
+    }
+    for (int q = 0; q < G; q++) {
+        k_fill_i64<<<1, 64, 0, st>>>(gslots + 64 * (size_t)q, KEY_NONE, 48);
+        CK(cudaMemsetAsync(gslots + 64 * (size_t)q + 48, 0, 8, st));
+    }
+    A.slots = gslots;
+    A.groups = G;
+    void *args[] = {&A};
+    CK(cudaEventRecord(c->ev0, st));
+    CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(G * nb), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     return LNS_OK;
 }
@@ -1309,6 +1437,7 @@ void lns_destroy(lns_ctx *c)
     cudaFree(c->d_Arow); cudaFree(c->d_H); cudaFree(c->d_vb); cudaFree(c->d_Y); cudaFree(c->d_fs);
     cudaFree(c->d_slots); cudaFree(c->d_counter); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_bits);
     cudaFree(c->d_until); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
+    cudaFree(c->d_V0s); cudaFree(c->d_res); cudaFree(c->d_vouts); cudaFree(c->d_gslots);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
     delete c;
@@ -1506,35 +1635,85 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
 lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, int64_t tenure, uint64_t seed,
                               const int8_t *V0, int32_t flags, int8_t *V_out, lns_result *res, void *stream)
 {
-    if (!c || !res || R < 0) return fail(LNS_EINVAL, "bad argument");
-    const int savep = c->part, saven = c->nparts;
-    void *savec = c->comm;
-    c->part = 0; c->nparts = 1; c->comm = nullptr;
-    lns_status s = LNS_OK;
-    double total_ms = 0;
-    for (int r = 0; r < R && s == LNS_OK; r++) {
-        uint64_t st = seed + (uint64_t)r;
-        const uint64_t seed_r = splitmix64_next(st);
-        const int8_t *v0 = V0 ? V0 + (size_t)r * c->n : nullptr;
-        int8_t *vo = V_out ? V_out + (size_t)r * c->n : nullptr;
-        s = lns_tabu_run(c, k, iters, tenure, seed_r, v0, flags & ~LNS_FORCE_STEPPED, vo, nullptr, nullptr, &res[r], stream);
-        total_ms += c->last_ms;
+    Geometry g;
+    lns_status s = check_k(c, k, g);
+    if (s != LNS_OK) return s;
+    if (!res || R < 0) return fail(LNS_EINVAL, "bad argument");
+    if (iters < 0 || iters >= (int64_t)INT32_MAX) return fail(LNS_EINVAL, "iters must be in [0, 2^31)");
+    int64_t L;
+    if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
+    if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    if (R == 0) return LNS_OK;
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    // start vectors: given (validated) or drawn from seed_r = splitmix64(seed + r) (reading R12)
+    const int n = c->n;
+    std::vector<int8_t> hv((size_t)R * n);
+    if (V0) {
+        CK(cudaMemcpy(hv.data(), V0, hv.size(), cudaMemcpyDefault));
+        for (int8_t v : hv)
+            if (v != 1 && v != -1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
+    } else {
+        for (int r = 0; r < R; r++) {
+            uint64_t sr = seed + (uint64_t)r;
+            vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
+        }
     }
-    c->last_ms = total_ms;
-    c->part = savep; c->nparts = saven; c->comm = savec;
-    return s;
-}
-
-#ifdef LNS_PHASE_TIMING
-// Profiling build only: read (and reset) the per-phase cycle sums over CTAs and iterations.
-lns_status lns_debug_phases(unsigned long long *out8)
-{
-    CK(cudaMemcpyFromSymbol(out8, g_ph, sizeof(unsigned long long) * NPH));
-    unsigned long long z[NPH] = {0};
-    CK(cudaMemcpyToSymbol(g_ph, z, sizeof(z)));
+    // groups: as many concurrent searches as SMs allow; CTAs per group = SMs / groups; a global
+    // until[] per group (when it is not cached in shared memory) is capped at 8 GiB
+    int G = std::min<int>(R, c->numSMs);
+    if (c->blocks_override > 0) G = std::min(G, std::max(1, c->numSMs / c->blocks_override));
+    const int budget = c->smemOptin - 1024;
+    const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / (4LL * g.M));
+    for (;;) {
+        const int nb = c->numSMs / G;
+        const uint64_t slice = ((uint64_t)g.M + nb - 1) / nb + 64;
+        const bool cached = g.smem_eval + 4 * slice <= (size_t)budget;
+        if (cached || G <= cap_groups) break;
+        G = (int)cap_groups;
+    }
+    const int nb = c->numSMs / G;
+    if ((s = grow(c->d_V0s, c->v0s_cap, hv.size())) != LNS_OK) return s;
+    if ((s = grow(c->d_res, c->res_cap, (size_t)R * FS_N)) != LNS_OK) return s;
+    if ((s = grow(c->d_vouts, c->vouts_cap, (size_t)R * c->NWn)) != LNS_OK) return s;
+    if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)G * 64)) != LNS_OK) return s;
+    if ((s = grow(c->d_until, c->until_cap, std::max<size_t>(g.M, 1))) != LNS_OK) return s;
+    CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
+    const int savep = c->part, saven = c->nparts;
+    c->part = 0; c->nparts = 1;
+    SearchArgs A = make_args(c, g, iters, L, flags);
+    c->part = savep; c->nparts = saven;
+    A.R = R; A.V0s = c->d_V0s; A.res = c->d_res; A.vouts = c->d_vouts;
+    A.trace_r = nullptr; A.trace_f = nullptr;
+    switch (k) {
+    case 1: s = launch_batch<1>(c, A, g, G, nb, c->d_gslots, st); break;
+    case 2: s = launch_batch<2>(c, A, g, G, nb, c->d_gslots, st); break;
+    default: s = launch_batch<3>(c, A, g, G, nb, c->d_gslots, st); break;
+    }
+    if (s != LNS_OK) return s;
+    std::vector<int64_t> hres((size_t)R * FS_N);
+    std::vector<uint32_t> hvo((size_t)R * c->NWn);
+    CK(cudaMemcpyAsync(hres.data(), c->d_res, hres.size() * 8, cudaMemcpyDeviceToHost, st));
+    CK(cudaMemcpyAsync(hvo.data(), c->d_vouts, hvo.size() * 4, cudaMemcpyDeviceToHost, st));
+    CK(cudaStreamSynchronize(st));
+    float ms = 0;
+    if (cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
+    for (int r = 0; r < R; r++) {
+        const int64_t *o = hres.data() + (size_t)r * FS_N;
+        if (o[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
+        res[r].iters_done = o[FS_T]; res[r].final_f = o[FS_F]; res[r].best_f = o[FS_BEST];
+        res[r].best_iter = o[FS_BESTIT]; res[r].first_zero_iter = o[FS_ZERO];
+        res[r].solved = o[FS_BEST] == 0; res[r].reserved = 0;
+    }
+    if (V_out) {
+        std::vector<int8_t> ho((size_t)R * n);
+        for (int r = 0; r < R; r++)
+            for (int i = 0; i < n; i++)
+                ho[(size_t)r * n + i] = ((hvo[(size_t)r * c->NWn + i / 32] >> (i % 32)) & 1) ? -1 : 1;
+        CK(cudaMemcpy(V_out, ho.data(), ho.size(), cudaMemcpyDefault));
+    }
     return LNS_OK;
 }
-#endif
 
 // Undocumented debug export (tests/tools only): plan of V for neighbourhood k, see k_debug_plan.
 lns_status lns_debug_plan(lns_ctx *c, int32_t k, const int8_t *V, int32_t *out_host, int64_t cap)

@@ -326,3 +326,37 @@ def test_python_partitioned_driver_with_nccl_world1(L, orc):
         assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
     finally:
         dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("cfg,R,iters,stop", [("C1", 300, 200, True), ("C2", 20, 150, False), ("C3", 6, 40, False),
+                                              ("C4", 3, 25, False)])
+def test_batched_restarts_grouped_kernel(L, orc, cfg, R, iters, stop):
+    """lns_tabu_run_batch splits the grid into groups, each running whole searches (C1 with 300
+    restarts: more restarts than SMs, so groups run several in turn). Every restart must equal the
+    oracle's search from splitmix64(seed + r) (reading R12)."""
+    c = pi.CONFIGS[cfg]
+    inst = pi.config_instance(cfg)
+    seed = 1234
+    ten = pi.default_tenure(inst.n, c["k"])
+    with L.Instance(inst.A, inst.S) as I:
+        Vo = np.empty((R, inst.n), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, c["k"], R, iters, -1, seed, None,
+                                     L.LNS_STOP_ON_ZERO if stop else 0, Vo)
+    check = range(R) if R <= 20 else list(range(0, R, 7)) + [R - 1]
+    for r in check:
+        V0 = pi.start_vector(inst.n, pi.restart_seed(seed, r))
+        _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, c["k"], V0, iters, ten, stop_on_zero=stop)
+        assert batch[r] == ores, r
+        assert np.array_equal(Vo[r], oVo), r
+
+
+def test_batched_restarts_given_start_vectors(L, orc):
+    inst = pi.planted_instance(45, 37, 31)
+    rng = np.random.default_rng(3)
+    V0 = np.where(rng.random((9, 37)) < 0.5, -1, 1).astype(np.int8)
+    with L.Instance(inst.A, inst.S) as I:
+        Vo = np.empty((9, 37), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, 3, 9, 60, 11, 0, V0, 0, Vo)
+    for r in range(9):
+        _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0[r], 60, 11, stop_on_zero=False)
+        assert batch[r] == ores and np.array_equal(Vo[r], oVo)
