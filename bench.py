@@ -2,20 +2,26 @@
 """Benchmark of the B200 k-Hamming tabu search.
 
 Contract: ``python bench.py --gpus N --steps K --warmup W [--impl reference]`` prints ONE JSON
-line on rank 0. Workload (BASELINE.json ``metric``: "PPP 3-Hamming neighbors evaluated/sec and
-tabu iters/sec at 1/2/4/8 B200", quoted at 1/2/4/8 GPUs on configs[3]): the planted PPP instance
-m = 101, n = 117 (seed 1004), 3-Hamming neighbourhood (C(117,3) = 260,130 neighbours), tabu
-tenure floor(M/6) = 43,355, no early stop. One STEP = one tabu search of 2,000 iterations
-(every iteration evaluates all 260,130 neighbours, selects, moves) from the start vector of seed
-5 + step. With N > 1 the rank space is partitioned across the GPUs and one NCCL u64-MIN
-all-reduce per iteration picks the global move (strong scaling: the total work is fixed).
+line on rank 0.
 
-``value`` = neighbours evaluated per second over the whole job (device time, CUDA events, max
-over ranks), inputs already resident in HBM. ``e2e`` = the same metric through the C ABI with
-HOST buffers (instance upload, start vector, trace and final vector copies inside the timed
-region). ``roofline`` = the persistent search kernel's integer throughput against the issue-rate
-peak derived in DESIGN.md §6. ``cpu_baseline`` = the CPU oracle timed on this host on a bounded
-sample. ``--impl reference`` times that oracle alone as the reference arm.
+Workload (BASELINE.json ``metric`` "PPP 3-Hamming neighbors evaluated/sec and tabu iters/sec at
+1/2/4/8 B200", quoted at 1/2/4/8 GPUs on configs[3]): the planted PPP instance m = 101, n = 117
+(seed 1004), 3-Hamming neighbourhood (C(117,3) = 260,130 neighbours per iteration), tabu tenure
+floor(M/6) = 43,355, run the way the paper runs it: "A tabu search was executed 50 times"
+(Table III). One STEP = the 50 independent searches of 400 iterations each (the
+paper's cap C(n,3) = 260,130 iterations is scaled down; no early stop), run r of step s starting
+from splitmix64(seed_s + r). Every iteration of every search evaluates all 260,130 neighbours,
+selects the best admissible one and moves. On each GPU the searches run batched in one
+persistent kernel (the grid split into groups, ``lns_tabu_run_batch``); with N GPUs run r goes
+to rank r mod N (no per-iteration collective; the total job is fixed -> strong scaling).
+
+``value`` = neighbours evaluated per second over the whole job (device time by CUDA events, max
+over ranks), inputs resident in HBM. ``e2e`` = the same job through the C ABI with HOST buffers
+(instance upload, start vectors, final vectors and results back inside the timed region).
+``single_search`` = one search at a time (latency view: all SMs on one search, 2,000 iterations).
+``roofline`` = the search kernel's integer throughput against the issue-rate peak.
+``cpu_baseline`` = the CPU oracle on this host on a bounded sample. ``--impl reference`` times
+that oracle alone as the reference arm (this paper has no code).
 """
 from __future__ import annotations
 
@@ -39,7 +45,9 @@ import ppp_inputs as pi  # noqa: E402
 METRIC = "PPP 3-Hamming neighbors evaluated/sec and tabu iters/sec at 1/2/4/8 B200"
 UNIT = "neighbors/s"
 CFG = "C4"
-ITERS = 2000
+RUNS = 50        # independent searches per step
+ITERS = 400      # iterations per search per step
+SINGLE_ITERS = 2000
 L2_FLUSH_BYTES = 512 << 20  # > 126 MB L2
 
 
@@ -56,6 +64,10 @@ def peaks():
             return json.load(fh), "measured"
     except OSError:
         return {"sm_max_mhz": 1965.0, "hbm_gbs": 6650.0}, "fallback"
+
+
+def run_seed(step: int) -> int:
+    return 5 + step
 
 
 class ClockSampler:
@@ -116,30 +128,40 @@ class ClockSampler:
                 "reasons": reasons, "samples": len(rows)}
 
 
+def start_vectors(n: int, step: int, runs) -> np.ndarray:
+    runs = list(runs)
+    if not runs:
+        return np.zeros((0, n), np.int8)
+    return np.stack([pi.start_vector(n, pi.restart_seed(run_seed(step), r)) for r in runs]).astype(np.int8)
+
+
 # --------------------------------------------------------------------------------- oracle arm
 def oracle_sample(budget_s: float, nthreads: int = 0):
-    """Time the CPU oracle (as it stands) on the same instance / tenure, a bounded number of
-    iterations sized to ~budget_s. Returns (neighbors/s, iters/s, iterations, cores, seconds)."""
+    """The CPU oracle (as it stands) on the same job: whole runs (400 iterations each) of step 0,
+    as many as fit ~budget_s. Returns (neighbors/s, iters/s, iterations, cores, seconds)."""
     import oracle
 
     c = pi.CONFIGS[CFG]
     inst = pi.config_instance(CFG)
     M = comb(inst.n, c["k"])
-    V0 = pi.start_vector(inst.n, pi.config_seed(CFG))
     ten = pi.default_tenure(inst.n, c["k"])
-    t = time.perf_counter()
-    oracle.tabu_run(inst.A, inst.S, c["k"], V0, 3, ten, stop_on_zero=False, nthreads=nthreads)
-    per_iter = (time.perf_counter() - t) / 3
-    iters = int(max(3, min(ITERS, budget_s / max(per_iter, 1e-6))))
-    t = time.perf_counter()
-    oracle.tabu_run(inst.A, inst.S, c["k"], V0, iters, ten, stop_on_zero=False, nthreads=nthreads)
+    # whole runs of the job (run 0, 1, ... of step 0) until ~budget_s of CPU work
+    iters, runs, t = 0, 0, time.perf_counter()
+    while True:
+        V0 = start_vectors(inst.n, 0, [runs])[0]
+        oracle.tabu_run(inst.A, inst.S, c["k"], V0, ITERS, ten, stop_on_zero=False, nthreads=nthreads)
+        iters += ITERS
+        runs += 1
+        if time.perf_counter() - t >= budget_s or runs >= RUNS:
+            break
     dt = time.perf_counter() - t
     cores = nthreads or oracle.max_threads()
     return iters * M / dt, iters / dt, iters, cores, dt
 
 
 def run_reference(args, rank, world):
-    """--impl reference: the CPU oracle (the only reference this paper has)."""
+    """--impl reference: the CPU oracle (this paper has no code). Each step = the
+    first 2 runs of the job, 4 iterations each (a bounded sample of the same workload)."""
     if rank != 0:
         return
     import oracle
@@ -149,27 +171,29 @@ def run_reference(args, rank, world):
     inst = pi.config_instance(CFG)
     M = comb(inst.n, c["k"])
     ten = pi.default_tenure(inst.n, c["k"])
-    per_step = 8  # iterations of the search per step (bounded sample of the 2,000-iteration step)
+    runs, per_run = 2, 4
     times = []
     for s in range(args.warmup + args.steps):
-        V0 = pi.start_vector(inst.n, 5 + s)
+        V0 = start_vectors(inst.n, s, range(runs))
         t = time.perf_counter()
-        oracle.tabu_run(inst.A, inst.S, c["k"], V0, per_step, ten, stop_on_zero=False)
+        for r in range(runs):
+            oracle.tabu_run(inst.A, inst.S, c["k"], V0[r], per_run, ten, stop_on_zero=False)
         if s >= args.warmup:
             times.append(time.perf_counter() - t)
     total = sum(times)
-    value = args.steps * per_step * M / total
+    value = args.steps * runs * per_run * M / total
     cores = oracle.max_threads()
+    sample = f"{runs} runs x {per_run} tabu iterations of {CFG} per step, from-scratch fitness ({cores} OpenMP threads)"
     line = {
         "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * total / args.steps,
         "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "int32",
         "data": "synthetic planted PPP instance (seeded splitmix64)",
-        "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming, tenure {ten}", "iters_per_step": per_step,
-                   "parallelism": "cpu-openmp", "l2": "n/a (CPU)"},
-        "tabu_iters_per_s": args.steps * per_step / total,
-        "cpu_baseline": {"value": value, "unit": UNIT, "cores": cores, "kind": "oracle",
-                         "sample": f"{per_step} tabu iterations of {CFG} per step from scratch (oracle, {cores} OpenMP threads)"},
+        "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming, tenure {ten}, independent tabu searches",
+                   "runs_per_step": runs, "iters_per_run": per_run, "parallelism": "cpu-openmp",
+                   "l2": "n/a (CPU)"},
+        "tabu_iters_per_s": args.steps * runs * per_run / total,
+        "cpu_baseline": {"value": value, "unit": UNIT, "cores": cores, "kind": "oracle", "sample": sample},
         "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -183,8 +207,10 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="lns", choices=["lns", "reference"])
     ap.add_argument("--iters", type=int, default=ITERS)
+    ap.add_argument("--runs", type=int, default=RUNS)
     ap.add_argument("--no-cpu-baseline", action="store_true")
-    ap.add_argument("--cpu-budget", type=float, default=12.0)
+    ap.add_argument("--no-single", action="store_true")
+    ap.add_argument("--cpu-budget", type=float, default=10.0)
     args = ap.parse_args()
     rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
     if args.impl == "reference":
@@ -196,6 +222,7 @@ def main():
     import torch.distributed as dist
 
     import paper_conf_ipps_luongmt10_b200 as L
+    from paper_conf_ipps_luongmt10_b200.parallel import restart_shard
 
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
@@ -207,21 +234,19 @@ def main():
     M = comb(inst.n, k)
     ten = pi.default_tenure(inst.n, k)
     iters = args.iters
+    mine = restart_shard(args.runs, rank, world)  # runs of this rank: r = rank, rank + world, ...
+    R = len(mine)
     ctx = L.lns_create(inst.A, inst.S, local)
-    if world > 1:
-        pg = dist.distributed_c10d._get_default_group()
-        comm = pg._get_backend(dev)._comm_ptr()
-        L.lns_attach_comm(ctx, comm, rank, world)
     stream = torch.cuda.current_stream(dev)
     nsteps = args.warmup + args.steps
-    V0s = torch.stack([torch.from_numpy(pi.start_vector(inst.n, 5 + s)) for s in range(nsteps)]).to(dev)
-    tr = torch.empty(iters, dtype=torch.int64, device=dev)
-    tf = torch.empty(iters, dtype=torch.int64, device=dev)
-    Vo = torch.empty(inst.n, dtype=torch.int8, device=dev)
+    V0s = [torch.from_numpy(start_vectors(inst.n, s, mine)).to(dev) for s in range(nsteps)]
+    Vo = torch.empty((max(R, 1), inst.n), dtype=torch.int8, device=dev)
     flush = torch.empty(L2_FLUSH_BYTES // 4, dtype=torch.int32, device=dev)
 
     def step(s):
-        return L.lns_tabu_run(ctx, k, iters, ten, 0, V0s[s], 0, Vo, tr, tf, stream)
+        if R == 0:
+            return []
+        return L.lns_tabu_run_batch(ctx, k, R, iters, ten, 0, V0s[s], 0, Vo, stream)
 
     for s in range(args.warmup):
         step(s)
@@ -239,27 +264,27 @@ def main():
             res = step(args.warmup + i)
             ev1[i].record(stream)
             torch.cuda.synchronize()
-            kernel_ms.append(L.lns_last_kernel_ms(ctx))
-            iters_done += res["iters_done"]
+            kernel_ms.append(L.lns_last_kernel_ms(ctx) if R else 0.0)
+            iters_done += sum(r["iters_done"] for r in res)
     clocks = clk.summary()
     step_ms = [a.elapsed_time(b) for a, b in zip(ev0, ev1)]
-    total_ms = sum(step_ms)
-    kern_ms = sum(kernel_ms)
+    total_ms, kern_ms = sum(step_ms), sum(kernel_ms)
+    my_iters = iters_done
     if world > 1:
         t = torch.tensor([total_ms, kern_ms], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         total_ms, kern_ms = float(t[0]), float(t[1])
+        n_it = torch.tensor([iters_done], dtype=torch.int64, device=dev)
+        dist.all_reduce(n_it, op=dist.ReduceOp.SUM)
+        iters_done = int(n_it[0])
     value = iters_done * M / (total_ms / 1e3)
 
-    # ---- end to end through the C ABI with host buffers (pinned), same metric
+    # ---- end to end through the C ABI with host buffers (pinned), same job
     A_h = torch.from_numpy(inst.A).pin_memory()
     S_h = torch.from_numpy(inst.S).pin_memory()
-    V0_h = torch.from_numpy(pi.start_vector(inst.n, 5)).pin_memory()
-    tr_h = torch.empty(iters, dtype=torch.int64).pin_memory()
-    tf_h = torch.empty(iters, dtype=torch.int64).pin_memory()
-    Vo_h = torch.empty(inst.n, dtype=torch.int8).pin_memory()
-    e2e_ms = 0.0
-    e2e_iters = 0
+    V0_h = [torch.from_numpy(start_vectors(inst.n, s, mine)).pin_memory() for s in range(args.steps)]
+    Vo_h = torch.empty((max(R, 1), inst.n), dtype=torch.int8).pin_memory()
+    e2e_ms, e2e_iters = 0.0, 0
     for i in range(args.steps):
         flush.fill_(i)
         if world > 1:
@@ -268,32 +293,56 @@ def main():
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record(stream)
         c2 = L.lns_create(A_h, S_h, local)
-        if world > 1:
-            L.lns_attach_comm(c2, comm, rank, world)
-        r2 = L.lns_tabu_run(c2, k, iters, ten, 0, V0_h, 0, Vo_h, tr_h, tf_h, stream)
+        r2 = L.lns_tabu_run_batch(c2, k, R, iters, ten, 0, V0_h[i], 0, Vo_h, stream) if R else []
         L.lns_destroy(c2)
         e1.record(stream)
         torch.cuda.synchronize()
         e2e_ms += e0.elapsed_time(e1)
-        e2e_iters += r2["iters_done"]
+        e2e_iters += sum(r["iters_done"] for r in r2)
     if world > 1:
         t = torch.tensor([e2e_ms], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         e2e_ms = float(t[0])
+        n_it = torch.tensor([e2e_iters], dtype=torch.int64, device=dev)
+        dist.all_reduce(n_it, op=dist.ReduceOp.SUM)
+        e2e_iters = int(n_it[0])
     e2e_value = e2e_iters * M / (e2e_ms / 1e3)
-    h2d = A_h.numel() + 4 * S_h.numel() + V0_h.numel()
-    d2h = 8 * tr_h.numel() + 8 * tf_h.numel() + Vo_h.numel()
+    h2d = A_h.numel() + 4 * S_h.numel() + V0_h[0].numel()
+    d2h = Vo_h.numel() + 48 * R  # final vectors + lns_result records
 
-    # ---- roofline: the persistent search kernel (one launch per step)
+    # ---- single search (latency view), N = 1 only
+    single = None
+    if world == 1 and not args.no_single:
+        tr = torch.empty(SINGLE_ITERS, dtype=torch.int64, device=dev)
+        tf = torch.empty(SINGLE_ITERS, dtype=torch.int64, device=dev)
+        v1 = torch.empty(inst.n, dtype=torch.int8, device=dev)
+        v0 = V0s[0][0].contiguous()
+        L.lns_tabu_run(ctx, k, SINGLE_ITERS, ten, 0, v0, 0, v1, tr, tf, stream)
+        ms = []
+        for _ in range(3):
+            flush.fill_(0)
+            torch.cuda.synchronize()
+            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            a.record(stream)
+            L.lns_tabu_run(ctx, k, SINGLE_ITERS, ten, 0, v0, 0, v1, tr, tf, stream)
+            b.record(stream)
+            torch.cuda.synchronize()
+            ms.append(a.elapsed_time(b))
+        best = min(ms)
+        single = {"neighbors_per_s": SINGLE_ITERS * M / (best / 1e3), "tabu_iters_per_s": SINGLE_ITERS / (best / 1e3),
+                  "us_per_iteration": 1e3 * best / SINGLE_ITERS, "iters": SINGLE_ITERS,
+                  "note": "one search on all SMs (persistent kernel, one exchange per iteration)"}
+
+    # ---- roofline: the search kernel (one launch per step)
     pk, src = peaks()
     mhz = float(pk.get("sm_max_mhz", 1965.0))
     sms = torch.cuda.get_device_properties(dev).multi_processor_count
     ops_per_nbr = inst.m * (k + 4)  # SURVEY.md §8(d) model: k sign reads + Y' add + penalty + 2 histogram moves per row
     kern_avg_s = kern_ms / 1e3 / args.steps
-    achieved = (iters * M / world) * ops_per_nbr / kern_avg_s / 1e12  # per-GPU share of the work
+    achieved = (my_iters / args.steps) * M * ops_per_nbr / kern_avg_s / 1e12 if kern_avg_s > 0 else 0.0
     peak = sms * 128 * mhz * 1e6 / 1e12  # 128 integer lanes issued per SM per clock (4 SMSP x 1 warp-instr)
     traffic = None
-    prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_C4.json")  # ncu --set full of the bench step
+    prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_bench.json")  # ncu --set full of one bench step
     if os.path.exists(prof):
         try:
             with open(prof) as fh:
@@ -301,7 +350,7 @@ def main():
         except (OSError, ValueError):
             traffic = None
     roofline = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tops/s", "frac": achieved / peak,
-                "traffic": traffic, "kernel": "k_search<3> (persistent tabu search)",
+                "traffic": traffic, "kernel": "k_search<3> (persistent, batched searches)",
                 "peak_source": f"{sms} SMs x 128 int lanes/clk x {mhz:.0f} MHz ({src} sm_max_mhz)",
                 "ops_per_neighbor": ops_per_nbr}
 
@@ -309,7 +358,7 @@ def main():
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
         v, ips, it, cores, dt = oracle_sample(args.cpu_budget)
         cpu = {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
-               "sample": f"{it} tabu iterations of {CFG} (same instance, tenure, start vector of seed 5), "
+               "sample": f"{it // ITERS} runs x {ITERS} tabu iterations of step 0 of the {CFG} job (same instance, tenure, start vectors), "
                          f"{dt:.1f} s, from-scratch fitness per neighbour", "tabu_iters_per_s": ips}
     if rank == 0:
         line = {
@@ -317,15 +366,19 @@ def main():
             "warmup": args.warmup, "ms_per_step": total_ms / args.steps, "higher_is_better": True,
             "scaling": "strong", "vs_baseline": None, "dtype": "int32",
             "data": "synthetic planted PPP instance (seeded splitmix64, DESIGN.md §3)",
-            "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming (260,130 neighbours), tabu tenure {ten}, "
-                                   f"{iters} iterations per step, no early stop",
-                       "iters_per_step": iters, "parallelism": f"rank-space partition x{world}" if world > 1 else "1 GPU",
+            "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming (260,130 neighbours/iteration), tenure {ten}; "
+                                   f"{args.runs} independent tabu searches x {iters} iterations per step "
+                                   "(PAPER.md:250 protocol), no early stop",
+                       "runs_per_step": args.runs, "iters_per_run": iters,
+                       "parallelism": f"runs sharded over {world} GPUs (r mod N), batched per GPU" if world > 1
+                       else "1 GPU, runs batched in one persistent kernel",
                        "l2": "flushed (512 MiB write) between timed steps"},
             "tabu_iters_per_s": iters_done / (total_ms / 1e3),
             "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
-            # our kernels per timed step: 2 x k_fill_i64 + k_init + (1 persistent k_search | 2 per iteration stepped)
-            "gpu_launches": args.steps * (4 if world == 1 else 2 + 2 * iters),
+            "single_search": single,
+            # our kernels per timed step: k_init_slots + the persistent k_search
+            "gpu_launches": args.steps * 2,
             "clocks": clocks,
             "roofline": roofline,
             "cpu_baseline": cpu,

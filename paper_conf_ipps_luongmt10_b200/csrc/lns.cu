@@ -1004,6 +1004,15 @@ __global__ void k_fill_i64(int64_t *p, int64_t v, int64_t cnt)
     for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < cnt; i += (int64_t)gridDim.x * blockDim.x) p[i] = v;
 }
 
+// Exchange slots of G groups: 3 keys (one per 128-B line) = KEY_NONE, arrival counter = 0.
+__global__ void k_init_slots(int64_t *slots, int G)
+{
+    for (int i = blockIdx.x * blockDim.x + threadIdx.x; i < 64 * G; i += gridDim.x * blockDim.x) {
+        const int q = i & 63;
+        slots[i] = q < 48 ? KEY_NONE : 0;
+    }
+}
+
 // until[r] = bit r of the caller's tabu bitmap (tabu at t = 1 <=> until >= 1).
 __global__ void k_bits_to_until(const uint32_t *bits, uint32_t *until, uint32_t M)
 {
@@ -1250,8 +1259,7 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     const int nb = search_blocks(c, A.hi - A.lo, 1);
     const size_t smem = cache_geometry(A, g, nb, budget);
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
-    k_fill_i64<<<1, 64, 0, st>>>(c->d_slots, KEY_NONE, 48);
-    CK(cudaMemsetAsync(c->d_slots + 48, 0, 8, st));
+    k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
     CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
@@ -1271,10 +1279,7 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int G, int 
         if (s != LNS_OK) return s;
         A.until = c->d_until;
     }
-    for (int q = 0; q < G; q++) {
-        k_fill_i64<<<1, 64, 0, st>>>(gslots + 64 * (size_t)q, KEY_NONE, 48);
-        CK(cudaMemsetAsync(gslots + 64 * (size_t)q + 48, 0, 8, st));
-    }
+    k_init_slots<<<(64 * G + 255) / 256, 256, 0, st>>>(gslots, G);
     A.slots = gslots;
     A.groups = G;
     void *args[] = {&A};
@@ -1661,8 +1666,20 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     }
     // groups: as many concurrent searches as SMs allow; CTAs per group = SMs / groups; a global
     // until[] per group (when it is not cached in shared memory) is capped at 8 GiB
-    int G = std::min<int>(R, c->numSMs);
-    if (c->blocks_override > 0) G = std::min(G, std::max(1, c->numSMs / c->blocks_override));
+    // choose G to minimise the makespan ceil(R/G) * T(SMs/G) with the iteration-time model
+    // T(nb) = 5 us + 3e-5 us * M (m + 32) / nb (fixed plan/exchange cost + evaluation spread over
+    // nb SMs; calibrated on C2-C4)
+    int G = 1;
+    {
+        double best = 1e300;
+        const double work = 3e-5 * (double)g.M * (double)(c->m + 32);
+        for (int q = 1; q <= std::min<int>(R, c->numSMs); q++) {
+            const int nbq = c->numSMs / q;
+            const double mk = (double)((R + q - 1) / q) * (5.0 + work / nbq);
+            if (mk < best * 0.999) { best = mk; G = q; }
+        }
+    }
+    if (c->blocks_override > 0) G = std::min(R, std::max(1, c->numSMs / c->blocks_override));
     const int budget = c->smemOptin - 1024;
     const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / (4LL * g.M));
     for (;;) {
