@@ -51,6 +51,8 @@ typedef int32_t lns_status;
 
 #define LNS_STOP_ON_ZERO 1      /* stop the search when f = 0 */
 #define LNS_FORCE_STEPPED 2     /* run one launch sequence per iteration instead of the persistent kernel */
+#define LNS_ASPIRATION 4        /* variant (not the default, reading R4'): a tabu move is admissible when its
+                                   fitness is below the best fitness found so far (Taillard [11]) */
 
 typedef struct lns_ctx lns_ctx;
 

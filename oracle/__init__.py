@@ -57,7 +57,7 @@ def _load():
             "oracle_eval_ranks": (i32, [_i8p, i32, i32, _i32p, _i8p, i32, _i64p, i64, _i64p, i32]),
             "oracle_eval_best": (i32, [_i8p, i32, i32, _i32p, _i8p, i32, _u8p, _i64p, _i64p, i32]),
             "oracle_tabu_run": (i32, [_i8p, i32, i32, _i32p, i32, _i8p, i64, i64, i32, _i64p, _i64p,
-                                      _i8p, _i64p, i32]),
+                                      _i8p, _i64p, i32, i32]),
             "oracle_max_threads": (i32, []),
         }
         for name, (res, args) in sig.items():
@@ -170,8 +170,10 @@ def eval_best(A, S, V, k: int, tabu=None, nthreads: int = 0) -> tuple[int, int]:
 RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_iter", "solved")
 
 
-def tabu_run(A, S, k: int, V0, iters: int, tenure: int, stop_on_zero: bool = True, nthreads: int = 0):
-    """Tabu search of PAPER.md:241-258. Returns (trace_rank, trace_fit, V_out, result dict)."""
+def tabu_run(A, S, k: int, V0, iters: int, tenure: int, stop_on_zero: bool = True, nthreads: int = 0,
+             aspiration: bool = False):
+    """Tabu search of PAPER.md:241-258. Returns (trace_rank, trace_fit, V_out, result dict).
+    aspiration: a tabu move is admissible when it beats the best fitness so far (variant R4')."""
     A, S, m, n = _prep(A, S)
     V0 = np.ascontiguousarray(V0, dtype=np.int8)
     tr = np.full(max(iters, 1), -1, dtype=np.int64)
@@ -180,7 +182,7 @@ def tabu_run(A, S, k: int, V0, iters: int, tenure: int, stop_on_zero: bool = Tru
     res = np.zeros(6, dtype=np.int64)
     rc = _load().oracle_tabu_run(_p(A, _i8p), m, n, _p(S, _i32p), k, _p(V0, _i8p), iters,
                                  tenure, int(bool(stop_on_zero)), _p(tr, _i64p),
-                                 _p(tf, _i64p), _p(Vo, _i8p), _p(res, _i64p), nthreads)
+                                 _p(tf, _i64p), _p(Vo, _i8p), _p(res, _i64p), nthreads, int(bool(aspiration)))
     if rc == -2:
         raise ValueError("tenure >= C(n,k): no admissible move would remain")
     if rc != 0:

@@ -227,7 +227,7 @@ static void flip(uint64_t *vb, int32_t i) { vb[i / 64] ^= 1ULL << (i % 64); }
 
 static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k, int mode,
                                int64_t *f_all, const int32_t *until, int64_t t,
-                               const int64_t *sample, int64_t nsample, int nthreads)
+                               const int64_t *sample, int64_t nsample, int nthreads, int64_t aspire_below)
 {
     int32_t n = P->n;
     int64_t *base = malloc(sizeof(int64_t) * (size_t)(n + 1));
@@ -260,12 +260,16 @@ static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k
                     if (mode == 2) {
                         if (q >= nsample || sample[q] != r) continue;
                     }
-                    if (mode == 1 && until && !(until[r] < t)) continue; /* tabu */
+                    const int tabu = (mode == 1 && until && !(until[r] < t));
+                    if (tabu && aspire_below < 0) continue; /* tabu, no aspiration */
                     memcpy(vb, vb0, sizeof(uint64_t) * (size_t)P->nw);
                     flip(vb, i1);
                     if (k >= 2) flip(vb, i2);
                     if (k == 3) flip(vb, i3);
                     int64_t f = fitness_packed(P, vb, Y, Hp);
+                    /* aspiration (reading R4'): a tabu move is admissible if it beats the best
+                     * fitness found so far */
+                    if (tabu && !(f < aspire_below)) continue;
                     if (mode == 0) f_all[r] = f;
                     else if (mode == 2) { while (q < nsample && sample[q] == r) { f_all[q] = f; q++; } }
                     else if (f < mine.f || (f == mine.f && r < mine.r)) { mine.f = f; mine.r = r; }
@@ -290,7 +294,7 @@ int32_t oracle_eval_all(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    scan_neighbourhood(&P, vb, k, 0, f_all, NULL, 0, NULL, 0, nthreads);
+    scan_neighbourhood(&P, vb, k, 0, f_all, NULL, 0, NULL, 0, nthreads, -1);
     free(vb); free_packed(&P);
     return 0;
 }
@@ -304,7 +308,7 @@ int32_t oracle_eval_ranks(const int8_t *A, int32_t m, int32_t n, const int32_t *
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    scan_neighbourhood(&P, vb, k, 2, f_out, NULL, 0, ranks, cnt, nthreads);
+    scan_neighbourhood(&P, vb, k, 2, f_out, NULL, 0, ranks, cnt, nthreads, -1);
     free(vb); free_packed(&P);
     return 0;
 }
@@ -324,7 +328,7 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, 1, NULL, 0, nthreads);
+    fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, 1, NULL, 0, nthreads, -1);
     *best_f = b.f == INT64_MAX ? -1 : b.f;
     *best_r = b.r;
     free(vb); free_packed(&P); free(until);
@@ -337,7 +341,9 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
  * replaces the current solution.
  *   - tabu list: FIFO of the last L accepted move ranks (reading R3), implemented literally as
  *     until[r]: a rank accepted at iteration t is tabu for t+1 .. t+L;
- *   - no aspiration (reading R4); lowest rank wins ties (reading R5);
+ *   - no aspiration by default (reading R4); with aspiration != 0 a tabu move is admissible when
+ *     it is better than the best fitness seen so far (Taillard's criterion, variant R4');
+ *     lowest rank wins ties (reading R5);
  *   - stop when f = 0 if stop_on_zero (checked before every iteration, also before t = 1),
  *     otherwise after `iters` iterations (reading R11).
  * res[0..5] = iters_done, final_f, best_f, best_iter, first_zero_iter (-1: never), solved.
@@ -345,7 +351,7 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
 int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S, int32_t k,
                         const int8_t *V0, int64_t iters, int64_t L, int32_t stop_on_zero,
                         int64_t *trace_r, int64_t *trace_f, int8_t *V_out, int64_t *res,
-                        int32_t nthreads)
+                        int32_t nthreads, int32_t aspiration)
 {
     if (k < 1 || k > 3 || n < k || m < 1 || iters < 0 || L < 0) return -1;
     int64_t M = oracle_neighborhood_size(n, k);
@@ -361,7 +367,7 @@ int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
     int64_t best_f = f, best_iter = 0, first_zero = (f == 0) ? 0 : -1, t;
     for (t = 1; t <= iters; t++) {
         if (stop_on_zero && f == 0) break;
-        fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, t, NULL, 0, nthreads);
+        fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, t, NULL, 0, nthreads, aspiration ? best_f : -1);
         if (b.r < 0) break; /* unreachable for L < M */
         /* apply: V <- V xor F_{r*}; flip set of r* found by walking the same nested loops */
         int32_t F[3];

@@ -28,6 +28,7 @@ LNS_ENCCL = -5
 LNS_ENOADMISSIBLE = -6
 LNS_STOP_ON_ZERO = 1
 LNS_FORCE_STEPPED = 2
+LNS_ASPIRATION = 4
 KEY_NONE = (1 << 63) - 1
 
 RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_iter", "solved")

@@ -93,6 +93,7 @@ struct SearchArgs {
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     int32_t no_split;       // 1: evaluate every lattice point (disable the linear-region shortcuts)
+    int32_t aspiration;     // a tabu move is admissible when it beats the best fitness so far
     // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
     // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
     // search from the state in (vb, Y, fs).
@@ -537,7 +538,8 @@ template <int K, bool WRITE_ALL>
 __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
                                          const PlanScalars &ps, uint32_t M, uint32_t blo, uint32_t bhi,
                                          const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
-                                         const uint2 *tri = nullptr, int no_split = 0)
+                                         const uint2 *tri = nullptr, int no_split = 0, int aspire = 0,
+                                         int best_f = 0)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
@@ -554,7 +556,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
         const uint32_t r = r0 + lane;
         if (r < bhi) {
             const bool is_tabu = until && until[r - ubase] >= t;
-            if (!is_tabu || WRITE_ALL) {
+            if (!is_tabu || WRITE_ALL || aspire) {
                 int a, b, c;
                 if (tri) {  // flip sets of this CTA's fixed slice, precomputed at launch
                     const uint2 q = tri[r - blo];
@@ -566,7 +568,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                                           : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c);
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
-                if (!is_tabu && key < best) best = key;
+                // admissible: not tabu, or (aspiration) better than the best fitness so far
+                if ((!is_tabu || (aspire && f < best_f)) && key < best) best = key;
             }
         }
     }
@@ -799,7 +802,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (A.stop_on_zero && f == 0) break;
             build_plan<K>(A.I, Ar, sm, L, ps);
             unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                           nullptr, tri, A.no_split);
+                                                           nullptr, tri, A.no_split, A.aspiration, (int)best_f);
             mine = warp_min_k(mine);
             if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
             __syncthreads();
@@ -843,9 +846,9 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (leader) {
                 if (A.trace_r) A.trace_r[t - 1] = r;
                 if (A.trace_f) A.trace_f[t - 1] = f;
-                if (f < best_f) { best_f = f; best_it = t; }
-                if (f == 0 && zero_it < 0) zero_it = t;
             }
+            if (f < best_f) { best_f = f; best_it = t; }  // every thread (aspiration needs it)
+            if (f == 0 && zero_it < 0) zero_it = t;
             int a, b, c;
             unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), a, b, c);
             apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
@@ -900,7 +903,8 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
     cta_slice(A.lo, A.hi, blockIdx.x, gridDim.x, blo, bhi);
     build_plan<K>(A.I, Ar, sm, L, ps);
     const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
-    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps, A.M, blo, bhi, A.until, 0, t, fit_out);
+    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps, A.M, blo, bhi, A.until, 0, t, fit_out,
+                                                       nullptr, 0, A.aspiration, (int)A.fs[FS_BEST]);
     mine = warp_min_k(mine);
     if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
     __syncthreads();
@@ -1168,6 +1172,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.M = g.M;
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
+    A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;

@@ -360,3 +360,18 @@ def test_batched_restarts_given_start_vectors(L, orc):
     for r in range(9):
         _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0[r], 60, 11, stop_on_zero=False)
         assert batch[r] == ores and np.array_equal(Vo[r], oVo)
+
+
+@pytest.mark.parametrize("k,L_ten,iters", [(1, 5, 200), (2, 100, 150), (3, 2000, 80)])
+def test_aspiration_variant_bit_exact(L, orc, k, L_ten, iters):
+    """LNS_ASPIRATION (variant R4'): persistent, stepped and batched paths against the oracle."""
+    inst = pi.planted_instance(41, 35, 800 + k)
+    V0 = pi.start_vector(35, 60 + k)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0, iters, L_ten, stop_on_zero=False, aspiration=True)
+    with L.Instance(inst.A, inst.S) as I:
+        for flags in (L.LNS_ASPIRATION, L.LNS_ASPIRATION | L.LNS_FORCE_STEPPED):
+            tr, tf, Vo, res = I.tabu_run(k, iters, L_ten, V0=V0, stop_on_zero=False, flags=flags)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+        Vb = np.empty((1, 35), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, k, 1, iters, L_ten, 0, V0[None, :], L.LNS_ASPIRATION, Vb)
+        assert batch[0] == ores and np.array_equal(Vb[0], oVo)

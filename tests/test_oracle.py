@@ -265,9 +265,10 @@ def test_eval_best_is_lowest_rank_argmin_over_admissible(orc, k):
 
 
 # ----------------------------------------------------------------------------- tabu search
-def _check_tabu_trace(orc, A, S, k, V0, L, tr, tf, res, stop_on_zero):
+def _check_tabu_trace(orc, A, S, k, V0, L, tr, tf, res, stop_on_zero, aspiration=False):
     """Each iteration: the accepted rank is the lowest-rank argmin over ranks not accepted in the
-    previous L iterations (FIFO tabu list, reading R3, no aspiration R4)."""
+    previous L iterations (FIFO tabu list, reading R3, no aspiration R4) -- or, with aspiration,
+    over those plus the tabu ranks whose fitness beats the best seen so far (variant R4')."""
     V = V0.copy()
     f = orc.fitness(A, S, V)
     best = f
@@ -277,6 +278,8 @@ def _check_tabu_trace(orc, A, S, k, V0, L, tr, tf, res, stop_on_zero):
         fa = orc.eval_all(A, S, V, k)
         tabu = np.zeros(len(fa), bool)
         tabu[tr[max(0, t - L):t]] = True
+        if aspiration:
+            tabu &= ~(fa < best)
         masked = np.where(tabu, np.iinfo(np.int64).max, fa)
         assert tr[t] == int(np.argmin(masked)), t
         assert tf[t] == fa[tr[t]]
@@ -326,3 +329,14 @@ def test_tabu_rejects_tenure_that_exhausts_neighbourhood(orc):
     I = pi.planted_instance(5, 6, 1)
     with pytest.raises(ValueError):
         orc.tabu_run(I.A, I.S, 1, np.ones(6, np.int8), 5, 6)
+
+
+@pytest.mark.parametrize("k,L", [(1, 5), (2, 60), (3, 300)])
+def test_tabu_aspiration_variant(orc, k, L):
+    """Aspiration (Taillard [11], variant R4'): a tabu move is allowed when it is better than the
+    best fitness found so far; the check re-derives every step by brute force."""
+    I = pi.planted_instance(17, 19, 900 + k)
+    V0 = pi.start_vector(19, 40 + k)
+    tr, tf, Vo, res = orc.tabu_run(I.A, I.S, k, V0, 50, L, stop_on_zero=False, aspiration=True)
+    V = _check_tabu_trace(orc, I.A, I.S, k, V0, L, tr, tf, res, False, aspiration=True)
+    assert np.array_equal(V, Vo)
