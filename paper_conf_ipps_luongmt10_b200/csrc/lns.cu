@@ -94,6 +94,7 @@ struct SearchArgs {
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     int32_t no_split;       // 1: evaluate every lattice point (disable the linear-region shortcuts)
     int32_t aspiration;     // a tabu move is admissible when it beats the best fitness so far
+    uint32_t *Xg;           // non-null: X lives in global memory, W * n words per CTA (large m x n)
     // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
     // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
     // search from the state in (vb, Y, fs).
@@ -110,6 +111,9 @@ struct SearchArgs {
     int64_t *trace_r, *trace_f;
 };
 
+// The CTA's X (sorted sign bits): shared memory, or its own slot of the global fallback buffer.
+#define X_OF(A, sm, L) ((A).Xg ? (A).Xg + (size_t)blockIdx.x * (A).I.W * (A).I.n : (uint32_t *)((sm) + (L).X))
+
 // Shared-memory carve-up (identical on host and device). The bit-packed A (Ar) and the until[]
 // slice are staged only when they fit.
 struct Smem {
@@ -118,11 +122,11 @@ struct Smem {
 
 __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
 
-__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem)
+__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0)
 {
     Smem s;
     int o = 0;
-    s.X = o;      o = align16(o + 4 * W * n);
+    s.X = o;      o = align16(o + (x_global ? 0 : 4 * W * n));  // X in global memory when it cannot fit
     s.Y = o;      o = align16(o + 4 * m);
     s.vb = o;     o = align16(o + 4 * NWn);
     s.H = o;      o = align16(o + 4 * (n + 1));
@@ -273,9 +277,11 @@ __device__ __forceinline__ void range_publish(int mn, int mx, PlanScalars &ps)
 //   X[w][c]   sign bits x_jc = [A_jc V_c = -1] of sorted rows 32w..32w+31, column c
 // Leaves cnt[] zeroed, ps.key / gkey = KEY_NONE and ps.vlo / Uc set for the next plan.
 // ------------------------------------------------------------------------------------------
-template <int K>
-__device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps)
+template <int K, bool XG = false>
+__device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                           uint32_t *Xarg)
 {
+    uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int m = I.m, n = I.n, W = I.W, NWn = I.NWn;
     const int *Ys = (const int *)(sm + L.Y);
@@ -289,7 +295,6 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     int2 *bins = (int2 *)(sm + L.bins);
     uint2 *pieces = (uint2 *)(sm + L.pieces);
     int *pstart = (int *)(sm + L.pstart);
-    uint32_t *X = (uint32_t *)(sm + L.X);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
     // A. counting sort over the conservative lattice
@@ -534,15 +539,16 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
 
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
 // key. until (nullable) is indexed by r - ubase: rank r is tabu iff until[r - ubase] >= t.
-template <int K, bool WRITE_ALL>
+template <int K, bool WRITE_ALL, bool XG = false>
 __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
-                                         const PlanScalars &ps, uint32_t M, uint32_t blo, uint32_t bhi,
+                                         const PlanScalars &ps, const uint32_t *Xarg, uint32_t M, uint32_t blo, uint32_t bhi,
                                          const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
                                          const uint2 *tri = nullptr, int no_split = 0, int aspire = 0,
                                          int best_f = 0)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const uint32_t *X = (const uint32_t *)(sm + L.X);
+    // X from the shared window when it lives there, so the compiler emits LDS (not generic loads)
+    const uint32_t *X = XG ? Xarg : (const uint32_t *)(sm + L.X);
     const uint2 *pieces = (const uint2 *)(sm + L.pieces);
     const int2 *bins = (const int2 *)(sm + L.bins);
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
@@ -742,7 +748,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
     const int G = A.groups > 0 ? A.groups : 1;
@@ -800,9 +806,13 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         bool failed = false;
         for (; t <= t0 + A.iters; t++) {
             if (A.stop_on_zero && f == 0) break;
-            build_plan<K>(A.I, Ar, sm, L, ps);
-            unsigned long long mine = eval_range<K, false>(A.I, sm, L, ps, A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                           nullptr, tri, A.no_split, A.aspiration, (int)best_f);
+            if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
+            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr);
+            unsigned long long mine =
+                A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
+                                                  nullptr, tri, A.no_split, A.aspiration, (int)best_f)
+                     : eval_range<K, false, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, until, ubase, (uint32_t)t,
+                                                   nullptr, tri, A.no_split, A.aspiration, (int)best_f);
             mine = warp_min_k(mine);
             if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
             __syncthreads();
@@ -892,7 +902,7 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     const int lane = threadIdx.x & 31;
     if (!WRITE_ALL && A.fs[FS_DONE]) {
         if (blockIdx.x == 0 && threadIdx.x == 0) *key_out = KEY_NONE;
@@ -901,10 +911,14 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
     const uint32_t *Ar = load_state<K>(A, sm, L, ps);
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, blockIdx.x, gridDim.x, blo, bhi);
-    build_plan<K>(A.I, Ar, sm, L, ps);
+    if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
+            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr);
     const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
-    unsigned long long mine = eval_range<K, WRITE_ALL>(A.I, sm, L, ps, A.M, blo, bhi, A.until, 0, t, fit_out,
-                                                       nullptr, 0, A.aspiration, (int)A.fs[FS_BEST]);
+    unsigned long long mine =
+        A.Xg ? eval_range<K, WRITE_ALL, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, A.until, 0, t, fit_out,
+                                              nullptr, 0, A.aspiration, (int)A.fs[FS_BEST])
+             : eval_range<K, WRITE_ALL, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, A.until, 0, t, fit_out,
+                                               nullptr, 0, A.aspiration, (int)A.fs[FS_BEST]);
     mine = warp_min_k(mine);
     if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
     __syncthreads();
@@ -967,10 +981,11 @@ __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     const uint32_t *Ar = load_state<K>(A, sm, L, ps);
     const int *segp = (const int *)(sm + L.seg);
-    build_plan<K>(A.I, Ar, sm, L, ps);
+    if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
+            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr);
     const int U = ps.U;
     if (threadIdx.x == 0) {
         const int2 *bins = (const int2 *)(sm + L.bins);
@@ -1057,6 +1072,7 @@ struct lns_ctx {
     int64_t *d_res = nullptr; size_t res_cap = 0;
     uint32_t *d_vouts = nullptr; size_t vouts_cap = 0;
     int64_t *d_gslots = nullptr; size_t gslots_cap = 0;
+    uint32_t *d_X = nullptr; size_t X_cap = 0;                // global X fallback (per CTA)
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
     double last_ms = 0.0;
     // stepped search
@@ -1137,10 +1153,11 @@ void slice_of(uint32_t M, int part, int nparts, uint32_t &lo, uint32_t &hi)
 struct Geometry {
     uint32_t M = 0;
     int a_in_smem = 0;
+    int x_global = 0;      // X does not fit in shared memory: per-CTA slots in global memory
     size_t smem_eval = 0;  // bytes for the stepped / eval kernels
 };
 
-lns_status check_k(const lns_ctx *c, int k, Geometry &g)
+lns_status check_k(lns_ctx *c, int k, Geometry &g)
 {
     if (!c) return fail(LNS_EINVAL, "null context");
     if (k < 1 || k > 3) return fail(LNS_EINVAL, "k must be 1, 2 or 3");
@@ -1149,19 +1166,29 @@ lns_status check_k(const lns_ctx *c, int k, Geometry &g)
     if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
     g.M = (uint32_t)Mk;
     const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
+    // preference: X and A in shared memory; X only; neither (X in global memory)
     const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1);
     const Smem without = smem_layout(c->m, c->n, c->W, c->NWn, k, 0);
+    const Smem xg = smem_layout(c->m, c->n, c->W, c->NWn, k, 0, 1);
     if (with.a_end <= budget) { g.a_in_smem = 1; g.smem_eval = (size_t)with.a_end; }
     else if (without.a_end <= budget) { g.a_in_smem = 0; g.smem_eval = (size_t)without.a_end; }
-    else return fail(LNS_ERANGE, "bit-packed A does not fit in shared memory");
+    else if (xg.a_end <= budget) { g.a_in_smem = 0; g.x_global = 1; g.smem_eval = (size_t)xg.a_end; }
+    else return fail(LNS_ERANGE, "plan does not fit in shared memory (n or m too large)");
+    if (g.x_global) {  // one X slot per CTA of the largest grid any launch uses (eval_all: 8 x SMs)
+        lns_status s = grow(c->d_X, c->X_cap, (size_t)8 * c->numSMs * c->W * c->n);
+        if (s != LNS_OK) return s;
+    }
     return LNS_OK;
 }
 
+// CTAs for one search over `span` ranks: about one CTA per 2,048 neighbour x (row words + 2) of
+// evaluation work (per-neighbour cost grows with the row words), capped by the SMs.
 int search_blocks(const lns_ctx *c, uint32_t span, int occ)
 {
     const int cap = std::min(c->numSMs * occ, MAX_SLOTS);
     if (c->blocks_override > 0) return std::min(c->blocks_override, cap);
-    const int nb = (int)std::min<int64_t>((int64_t)cap, std::max<int64_t>(1, span / 1024));
+    const int64_t work = (int64_t)span * (c->W + 2);
+    const int nb = (int)std::min<int64_t>((int64_t)cap, std::max<int64_t>(1, (work + 2047) / 2048));
     return std::max(1, nb);
 }
 
@@ -1173,6 +1200,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
+    A.Xg = g.x_global ? c->d_X : nullptr;
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
@@ -1447,7 +1475,7 @@ void lns_destroy(lns_ctx *c)
     cudaFree(c->d_Arow); cudaFree(c->d_H); cudaFree(c->d_vb); cudaFree(c->d_Y); cudaFree(c->d_fs);
     cudaFree(c->d_slots); cudaFree(c->d_counter); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_bits);
     cudaFree(c->d_until); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
-    cudaFree(c->d_V0s); cudaFree(c->d_res); cudaFree(c->d_vouts); cudaFree(c->d_gslots);
+    cudaFree(c->d_V0s); cudaFree(c->d_res); cudaFree(c->d_vouts); cudaFree(c->d_gslots); cudaFree(c->d_X);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
     delete c;

@@ -375,3 +375,23 @@ def test_aspiration_variant_bit_exact(L, orc, k, L_ten, iters):
         Vb = np.empty((1, 35), np.int8)
         batch = L.lns_tabu_run_batch(I.ctx, k, 1, iters, L_ten, 0, V0[None, :], L.LNS_ASPIRATION, Vb)
         assert batch[0] == ores and np.array_equal(Vb[0], oVo)
+
+
+@pytest.mark.parametrize("k", [1, 2])
+def test_large_instance_global_X_fallback(L, orc, k):
+    """1201 x 1217 (the Fig. 8 ladder): the sorted sign bits X no longer fit in
+    shared memory, so each CTA keeps them in global memory. All fitnesses (k = 1) or a sample
+    (k = 2) and a short k = 1 trajectory against the oracle."""
+    inst = pi.planted_instance(1201, 1217, 4321)
+    V = pi.start_vector(1217, 77)
+    M = comb(1217, k)
+    with L.Instance(inst.A, inst.S) as I:
+        got = L.lns_eval_all(I.ctx, k, V).astype(np.int64)
+        if k == 1:
+            assert np.array_equal(got, orc.eval_all(inst.A, inst.S, V, 1))
+            tr, tf, Vo, res = I.tabu_run(1, 40, -1, V0=V, stop_on_zero=False)
+            otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, 1, V, 40, pi.default_tenure(1217, 1), stop_on_zero=False)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(Vo, oVo)
+        else:
+            ranks = np.unique(np.random.default_rng(2).integers(0, M, 4000))
+            assert np.array_equal(got[ranks], orc.eval_ranks(inst.A, inst.S, V, 2, ranks))
