@@ -555,8 +555,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     EvalRange er;
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
-    if (no_split & 1) { er.u0 = 0; er.u1 = ps.U; er.rneg = 0; er.cneg = 0; er.p0 = 0; }
-    if (no_split & 2) er.u1 = ps.U;
+    if (no_split) { er.u0 = 0; er.u1 = ps.U; er.rneg = 0; er.cneg = 0; er.p0 = 0; }
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
@@ -1204,7 +1203,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
-    A.no_split = getenv("LNS_NO_SPLIT") ? atoi(getenv("LNS_NO_SPLIT")) : 0;
+    A.no_split = 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     return A;
