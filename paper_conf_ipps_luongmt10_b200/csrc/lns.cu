@@ -467,7 +467,33 @@ struct EvalRange {
     int u0, u1;       // lattice points [u0, u1) go through the segment loop (u0 = uneg, u1 = utop)
     int rneg, cneg;   // deep-negative rows [0, rneg) and their constant part
     int p0;           // first piece of point u0
+    int p1;           // first piece of point u1 (packed path)
+    int w0;           // row word of piece p0 (packed path)
 };
+
+// Deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
+//   = cneg - 240 sum_j t_j, with sum t = popc(lo) + 2 popc(hi) over their (sorted) row words.
+template <int K>
+__device__ __forceinline__ int deep_negative(const uint32_t *__restrict__ X, int n, const EvalRange &er, int f,
+                                             int a, int b, int c)
+{
+    int st = 0;
+    const int nw = (er.rneg + 31) >> 5;
+    for (int w = 0; w < nw; w++) {
+        const uint32_t mask = (w == nw - 1 && (er.rneg & 31)) ? ((1u << (er.rneg & 31)) - 1u) : FULL;
+        const uint32_t *xr = X + w * n;
+        if (K == 1) {
+            st += __popc(xr[a] & mask);
+        } else if (K == 2) {
+            const uint32_t xa = xr[a], xb = xr[b];
+            st += __popc((xa ^ xb) & mask) + 2 * __popc(xa & xb & mask);
+        } else {
+            const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+            st += __popc((xa ^ xb ^ xc) & mask) + 2 * __popc(((xa & xb) | (xc & (xa ^ xb))) & mask);
+        }
+    }
+    return (int)((unsigned)f + (unsigned)er.cneg - 240u * (unsigned)st);
+}
 
 template <int K, bool DEEP>
 __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
@@ -475,26 +501,7 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
                                         int a, int b, int c)
 {
     int f = m2, smin = 0;
-    // deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
-    //   = cneg - 240 sum_j t_j, with sum t = popc(lo) + 2 popc(hi) over their (sorted) row words
-    if (DEEP) {
-        int st = 0;
-        const int nw = (er.rneg + 31) >> 5;
-        for (int w = 0; w < nw; w++) {
-            const uint32_t mask = (w == nw - 1 && (er.rneg & 31)) ? ((1u << (er.rneg & 31)) - 1u) : FULL;
-            const uint32_t *xr = X + w * n;
-            if (K == 1) {
-                st += __popc(xr[a] & mask);
-            } else if (K == 2) {
-                const uint32_t xa = xr[a], xb = xr[b];
-                st += __popc((xa ^ xb) & mask) + 2 * __popc(xa & xb & mask);
-            } else {
-                const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
-                st += __popc((xa ^ xb ^ xc) & mask) + 2 * __popc(((xa & xb) | (xc & (xa ^ xb))) & mask);
-            }
-        }
-        f = (int)((unsigned)f + (unsigned)er.cneg - 240u * (unsigned)st);
-    }
+    if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
     const int U = er.u1 - er.u0;
     if (U <= 0) return f;
     int R0 = 0, R1 = 0, R2 = 0, R3 = 0, R4 = 0, R5 = 0;
@@ -537,6 +544,94 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
     return f - 2 * smin;
 }
 
+// eval_fit for m <= 255 (every bin count fits a byte): the 2K+1 open bins beta .. beta+2K live as
+// bytes of the 64-bit window (whi:wlo), byte i = bin beta+i. A piece adds its row counts straight
+// into the window (N0 -> byte 0, N1 -> byte 2, N2 -> byte 4, N3 -> byte 6, with N0 = len - sum_t N_t
+// added as -sum_t N_t now and len at the segment's end); byte 0 may go transiently negative, which
+// is harmless because each half is exact modulo 2^32 and its final bytes all lie in [0, 255].
+// Completing bin beta = adding len, reading byte 0, shifting the window down 8 bits. The walk is
+// word-major (the lane's three column words are loaded once per row word) and inside a word every
+// piece but the last finalises its bin, so the inner loop has no branch.
+template <int K>
+__device__ __forceinline__ void packed_add(uint32_t m, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &wlo, uint32_t &whi)
+{
+    const int p1 = __popc(lo & m);
+    if (K == 1) {               // N1 = p1 -> byte 2; -p1 -> byte 0
+        wlo += (uint32_t)p1 * 65535u;
+    } else if (K == 2) {        // N1 = p1 -> byte 2, N2 = p2 -> byte 4
+        const int p2 = __popc(hi & m);
+        wlo += ((uint32_t)p1 << 16) - (uint32_t)p1 - (uint32_t)p2;
+        whi += (uint32_t)p2;
+    } else {                    // N1 = p1 - p3 -> byte 2, N2 = p2 - p3 -> byte 4, N3 = p3 -> byte 6
+        const int p2 = __popc(hi & m), p3 = __popc(lh & m);
+        const uint32_t d1 = (uint32_t)(p1 - p3);
+        wlo += (d1 << 16) - d1 - (uint32_t)p2;
+        whi += (uint32_t)p2 + (uint32_t)p3 * 65535u;
+    }
+}
+
+__device__ __forceinline__ void packed_fin(uint32_t len, const int2 *__restrict__ &bp, uint32_t &wlo, uint32_t &whi,
+                                           int &f, int &smin)
+{
+    wlo += len;
+    const int h = (int)(wlo & 0xffu);
+    const int2 bn = *bp++;
+    f += bn.y * h;
+    smin += min(h, bn.x);
+    wlo = __funnelshift_r(wlo, whi, 8);
+    whi >>= 8;
+}
+
+template <int K, bool DEEP>
+__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
+                                               const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
+                                               const EvalRange &er, int m2, int a, int b, int c)
+{
+    int f = m2, smin = 0;
+    if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
+    if (er.u1 <= er.u0) return f;
+    uint32_t wlo = 0, whi = 0;
+    const uint2 *pp = pieces + er.p0;
+    const int2 *bp = bins + er.u0;
+    const uint32_t *xr = X + er.w0 * n;
+    const int *pw = pstart + er.w0 + 1;
+    for (;;) {
+        uint32_t lo, hi = 0, lh = 0;
+        if (K == 1) {
+            lo = xr[a];
+        } else if (K == 2) {
+            const uint32_t xa = xr[a], xb = xr[b];
+            lo = xa ^ xb; hi = xa & xb;
+        } else {
+            const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+            lo = xa ^ xb ^ xc;
+            hi = (xa & xb) | (xc & (xa ^ xb));
+            lh = lo & hi;
+        }
+        xr += n;
+        const int pend = min(*pw++, er.p1);
+        const uint2 *plast = pieces + pend - 1;
+        for (; pp < plast; ++pp) {  // all of these finalise their bin
+            const uint2 rec = *pp;
+            packed_add<K>(rec.x, lo, hi, lh, wlo, whi);
+            packed_fin(rec.y >> 16, bp, wlo, whi, f, smin);
+        }
+        const uint2 rec = *pp++;
+        packed_add<K>(rec.x, lo, hi, lh, wlo, whi);
+        if (rec.y & 1u) packed_fin(rec.y >> 16, bp, wlo, whi, f, smin);
+        if (pend == er.p1) break;
+    }
+    // bins beta .. beta+2K-1 past the last point hold only carried counts
+#pragma unroll
+    for (int i = 0; i < 2 * K; i++) {
+        const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
+        const int2 bn = bp[i];
+        f += bn.y * h;
+        smin += min(h, bn.x);
+    }
+    return f - 2 * smin;
+}
+
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
 // key. until (nullable) is indexed by r - ubase: rank r is tabu iff until[r - ubase] >= t.
 template <int K, bool WRITE_ALL, bool XG = false>
@@ -556,6 +651,10 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
     if (no_split) { er.u0 = 0; er.u1 = ps.U; er.rneg = 0; er.cneg = 0; er.p0 = 0; }
+    er.p1 = ((const int *)(sm + L.pofs))[er.u1];
+    er.w0 = (int)((pieces[er.p0].y >> 1) & 0x7fffu);
+    const int *pstart = (const int *)(sm + L.pstart);
+    const bool packed = I.m <= 255;
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
@@ -569,8 +668,10 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 } else {
                     unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
                 }
-                const int f = er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
-                                          : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c);
+                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pieces, pstart, bins, I.n, er, 2 * I.m, a, b, c)
+                                                    : eval_fit_packed<K, false>(X, pieces, pstart, bins, I.n, er, 2 * I.m, a, b, c))
+                                     : (er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
+                                                    : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c));
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 // admissible: not tabu, or (aspiration) better than the best fitness so far
