@@ -50,5 +50,15 @@ def build(force: bool = False, verbose: bool = False, profiling: bool = False) -
     return lib
 
 
+def build_variant(name: str, defines: list[str]) -> str:
+    """Experimental build with extra -D flags into build/variants/liblns_<name>.so (LNS_LIB=... selects it)."""
+    out_dir = os.path.join(ROOT, "build", "variants")
+    os.makedirs(out_dir, exist_ok=True)
+    lib = os.path.join(out_dir, f"liblns_{name}.so")
+    cmd = [nvcc(), *NVCC_FLAGS, *[f"-D{d}" for d in defines], "-I", os.path.join(ROOT, "include"), "-o", lib, *SRC, "-ldl"]
+    subprocess.check_call(cmd)
+    return lib
+
+
 if __name__ == "__main__":
     print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, profiling="--profiling" in sys.argv))

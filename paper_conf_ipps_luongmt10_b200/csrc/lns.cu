@@ -117,10 +117,17 @@ struct SearchArgs {
 // Shared-memory carve-up (identical on host and device). The bit-packed A (Ar) and the until[]
 // slice are staged only when they fit.
 struct Smem {
-    int X, Y, vb, H, cnt, seg, cur, pofs, rowAt, bins, pieces, pstart, T2, T3, base_end, Ar, a_end;
+    int X, Y, vb, H, cnt, seg, cur, pofs, rowAt, bins, pieces, pk, pstart, T2, T3, base_end, Ar, a_end;
 };
 
 __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
+
+// Bin counts fit a byte (the packed evaluation path, eval_fit_packed) when m <= 255.
+#define PACKED_MAX_M 255
+#ifndef PK_UNROLL
+#define PK_UNROLL 1
+#endif
+constexpr int kPkUnroll = PK_UNROLL;  // unroll of the packed piece loop
 
 __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0)
 {
@@ -137,6 +144,7 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
     s.rowAt = o;  o = align16(o + 4 * m);
     s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
     s.pieces = o; o = align16(o + 8 * (n + 2 + W));      // P <= U + W - 1 pieces (+1 prefetch pad)
+    s.pk = o;     o = align16(o + (m <= PACKED_MAX_M ? 16 * (n + 2 + W) : 0));  // packed-path pieces
     s.pstart = o; o = align16(o + 4 * (W + 1));
     s.T2 = o;     o = align16(o + 4 * n);                // C(y,2), y < n (u32)
     s.T3 = o;     o = align16(o + 4 * n);                // C(z,3), z < n (u32: C(n,3) < 2^32)
@@ -354,15 +362,23 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         rowAt[p] = j;
     }
     const int uneg = ps.uneg;
+    uint4 *pk = (uint4 *)(sm + L.pk);
+    const bool packed = m <= PACKED_MAX_M;
     for (int v = tid; v < U; v += NT) {
         const int st = seg[v], en = seg[v + 1];
         int p = pofs[v];
+        // packed-path record of this point's last piece: (mask, 8 | len << 24, H_b, w_b) of its bin
+        // beta = v (b = vmin + 2(v - K)); earlier pieces carry (mask, 0, 0, 0) and finalise nothing
+        const int bfin = vmin + 2 * (v - K);
+        const uint32_t Hfin = (bfin >= 0 && bfin <= n) ? (uint32_t)Hs[bfin] : 0u;
+        const uint32_t wfin = bfin < 0 ? (uint32_t)(60 * (-bfin) - 1) : 0u;
         // deep-negative constant sum_rows 60(2K - Y_j) - 1 (unsigned: the constant may exceed
         // 2^31 on its own; the fitness it enters does not)
         if (v < uneg && en > st)
             atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - 1));
         if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
             pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
+            if (packed) pk[p] = make_uint4(0u, 8u, Hfin, wfin);
             continue;
         }
         const int w0 = st >> 5, w1 = (en - 1) >> 5;
@@ -370,6 +386,8 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
             const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
             pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? 1 : 0) | ((uint32_t)w << 1) | ((uint32_t)(en - st) << 16));
+            if (packed)
+                pk[p] = w == w1 ? make_uint4(mask, 8u | ((uint32_t)(en - st) << 24), Hfin, wfin) : make_uint4(mask, 0u, 0u, 0u);
             if (w > w0 || (st & 31) == 0) pstart[w] = p;
         }
     }
@@ -570,20 +588,8 @@ __device__ __forceinline__ void packed_add(uint32_t m, uint32_t lo, uint32_t hi,
     }
 }
 
-__device__ __forceinline__ void packed_fin(uint32_t len, const int2 *__restrict__ &bp, uint32_t &wlo, uint32_t &whi,
-                                           int &f, int &smin)
-{
-    wlo += len;
-    const int h = (int)(wlo & 0xffu);
-    const int2 bn = *bp++;
-    f += bn.y * h;
-    smin += min(h, bn.x);
-    wlo = __funnelshift_r(wlo, whi, 8);
-    whi >>= 8;
-}
-
 template <int K, bool DEEP>
-__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint2 *__restrict__ pieces,
+__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
                                                const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
                                                const EvalRange &er, int m2, int a, int b, int c)
 {
@@ -591,8 +597,7 @@ __device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, c
     if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
     if (er.u1 <= er.u0) return f;
     uint32_t wlo = 0, whi = 0;
-    const uint2 *pp = pieces + er.p0;
-    const int2 *bp = bins + er.u0;
+    const uint4 *pp = pk + er.p0;
     const uint32_t *xr = X + er.w0 * n;
     const int *pw = pstart + er.w0 + 1;
     for (;;) {
@@ -610,18 +615,24 @@ __device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, c
         }
         xr += n;
         const int pend = min(*pw++, er.p1);
-        const uint2 *plast = pieces + pend - 1;
-        for (; pp < plast; ++pp) {  // all of these finalise their bin
-            const uint2 rec = *pp;
-            packed_add<K>(rec.x, lo, hi, lh, wlo, whi);
-            packed_fin(rec.y >> 16, bp, wlo, whi, f, smin);
+        const uint4 *pe = pk + pend;
+        // every record is applied the same way: a non-final piece has len = shift = H = w = 0,
+        // so its "bin" costs 0 and the window does not move
+#pragma unroll kPkUnroll
+        for (; pp < pe; ++pp) {
+            const uint4 r = *pp;
+            packed_add<K>(r.x, lo, hi, lh, wlo, whi);
+            wlo += r.y >> 24;
+            const int h = (int)(wlo & 0xffu);
+            f += (int)r.w * h;
+            smin += min(h, (int)r.z);
+            wlo = __funnelshift_r(wlo, whi, r.y);  // shift = r.y & 31 (8 or 0)
+            whi = __funnelshift_r(whi, 0u, r.y);
         }
-        const uint2 rec = *pp++;
-        packed_add<K>(rec.x, lo, hi, lh, wlo, whi);
-        if (rec.y & 1u) packed_fin(rec.y >> 16, bp, wlo, whi, f, smin);
         if (pend == er.p1) break;
     }
     // bins beta .. beta+2K-1 past the last point hold only carried counts
+    const int2 *bp = bins + er.u1;
 #pragma unroll
     for (int i = 0; i < 2 * K; i++) {
         const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
@@ -654,7 +665,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     er.p1 = ((const int *)(sm + L.pofs))[er.u1];
     er.w0 = (int)((pieces[er.p0].y >> 1) & 0x7fffu);
     const int *pstart = (const int *)(sm + L.pstart);
-    const bool packed = I.m <= 255;
+    const bool packed = I.m <= PACKED_MAX_M;
+    const uint4 *pk = (const uint4 *)(sm + L.pk);
     unsigned long long best = (unsigned long long)KEY_NONE;
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
@@ -668,8 +680,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 } else {
                     unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
                 }
-                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pieces, pstart, bins, I.n, er, 2 * I.m, a, b, c)
-                                                    : eval_fit_packed<K, false>(X, pieces, pstart, bins, I.n, er, 2 * I.m, a, b, c))
+                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a, b, c)
+                                                    : eval_fit_packed<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a, b, c))
                                      : (er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
                                                     : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c));
                 if (WRITE_ALL) fit_out[r] = f;
