@@ -128,6 +128,9 @@ __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
 #define PK_UNROLL 1
 #endif
 constexpr int kPkUnroll = PK_UNROLL;  // unroll of the packed piece loop
+#ifndef PK_PAIR
+#define PK_PAIR 1
+#endif
 
 __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0)
 {
@@ -588,6 +591,87 @@ __device__ __forceinline__ void packed_add(uint32_t m, uint32_t lo, uint32_t hi,
     }
 }
 
+// One packed record applied to one neighbour's window (see eval_fit_packed).
+template <int K>
+__device__ __forceinline__ void packed_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &wlo,
+                                            uint32_t &whi, int &f, int &smin)
+{
+    packed_add<K>(r.x, lo, hi, lh, wlo, whi);
+    wlo += r.y >> 24;
+    const int h = (int)(wlo & 0xffu);
+    f += (int)r.w * h;
+    smin += min(h, (int)r.z);
+    wlo = __funnelshift_r(wlo, whi, r.y);  // shift = r.y & 31 (8 or 0)
+    whi = __funnelshift_r(whi, 0u, r.y);
+}
+
+template <int K>
+__device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int a, int b, int c, uint32_t &lo,
+                                            uint32_t &hi, uint32_t &lh)
+{
+    if (K == 1) {
+        lo = xr[a]; hi = 0; lh = 0;
+    } else if (K == 2) {
+        const uint32_t xa = xr[a], xb = xr[b];
+        lo = xa ^ xb; hi = xa & xb; lh = 0;
+    } else {
+        const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
+        lo = xa ^ xb ^ xc;
+        hi = (xa & xb) | (xc & (xa ^ xb));
+        lh = lo & hi;
+    }
+}
+
+__device__ __forceinline__ void packed_trail(int K2, const int2 *__restrict__ bp, uint32_t wlo, uint32_t whi, int &f,
+                                             int &smin)
+{
+#pragma unroll
+    for (int i = 0; i < 6; i++) {
+        if (i < K2) {
+            const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
+            const int2 bn = bp[i];
+            f += bn.y * h;
+            smin += min(h, bn.x);
+        }
+    }
+}
+
+// Two neighbours per thread: the record stream, loop control and word bookkeeping are shared.
+template <int K, bool DEEP>
+__device__ __forceinline__ void eval_fit_packed2(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
+                                                 const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
+                                                 const EvalRange &er, int m2, int a0, int b0, int c0, int a1, int b1,
+                                                 int c1, int &f0, int &f1)
+{
+    f0 = m2; f1 = m2;
+    if (DEEP) { f0 = deep_negative<K>(X, n, er, f0, a0, b0, c0); f1 = deep_negative<K>(X, n, er, f1, a1, b1, c1); }
+    if (er.u1 <= er.u0) return;
+    int s0 = 0, s1 = 0;
+    uint32_t wl0 = 0, wh0 = 0, wl1 = 0, wh1 = 0;
+    const uint4 *pp = pk + er.p0;
+    const uint32_t *xr = X + er.w0 * n;
+    const int *pw = pstart + er.w0 + 1;
+    for (;;) {
+        uint32_t lo0, hi0, lh0, lo1, hi1, lh1;
+        load_planes<K>(xr, a0, b0, c0, lo0, hi0, lh0);
+        load_planes<K>(xr, a1, b1, c1, lo1, hi1, lh1);
+        xr += n;
+        const int pend = min(*pw++, er.p1);
+        const uint4 *pe = pk + pend;
+#pragma unroll 1
+        for (; pp < pe; ++pp) {
+            const uint4 r = *pp;
+            packed_step<K>(r, lo0, hi0, lh0, wl0, wh0, f0, s0);
+            packed_step<K>(r, lo1, hi1, lh1, wl1, wh1, f1, s1);
+        }
+        if (pend == er.p1) break;
+    }
+    const int2 *bp = bins + er.u1;
+    packed_trail(2 * K, bp, wl0, wh0, f0, s0);
+    packed_trail(2 * K, bp, wl1, wh1, f1, s1);
+    f0 -= 2 * s0; f1 -= 2 * s1;
+}
+
 template <int K, bool DEEP>
 __device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
                                                const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
@@ -668,6 +752,36 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     const bool packed = I.m <= PACKED_MAX_M;
     const uint4 *pk = (const uint4 *)(sm + L.pk);
     unsigned long long best = (unsigned long long)KEY_NONE;
+    if (packed && PK_PAIR && bhi - blo > (uint32_t)NT) {
+        // two neighbours per thread: ranks r and r + 32 (a warp covers 64 consecutive ranks); only
+        // when the slice needs more than one pass of the block, else half the warps would idle
+        for (uint32_t r0 = blo + 64u * warp; r0 < bhi; r0 += 2 * NT) {
+            const uint32_t rA = r0 + lane, rB = rA + 32u;
+            if (rA >= bhi) continue;
+            const bool vB = rB < bhi;
+            const uint32_t rb = vB ? rB : rA;  // a ragged tail re-evaluates rA in the B slot
+            int a0, b0, c0, a1, b1, c1;
+            if (tri) {
+                const uint2 q0 = tri[rA - blo], q1 = tri[rb - blo];
+                a0 = (int)(q0.x & 0xffffu); b0 = (int)(q0.x >> 16); c0 = (int)q0.y;
+                a1 = (int)(q1.x & 0xffffu); b1 = (int)(q1.x >> 16); c1 = (int)q1.y;
+            } else {
+                unrank_tab<K>(rA, I.n, M, T2, T3, a0, b0, c0);
+                unrank_tab<K>(rb, I.n, M, T2, T3, a1, b1, c1);
+            }
+            int fA, fB;
+            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            const bool tA = until && until[rA - ubase] >= t;
+            const bool tB = until && until[rb - ubase] >= t;
+            if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
+            const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
+            const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
+            if ((!tA || (aspire && fA < best_f)) && kA < best) best = kA;
+            if ((!tB || (aspire && fB < best_f)) && kB < best) best = kB;
+        }
+        return best;
+    }
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
         if (r < bhi) {
