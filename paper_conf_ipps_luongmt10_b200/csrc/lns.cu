@@ -228,6 +228,23 @@ __device__ __forceinline__ void unrank_tab(uint32_t r, int n, uint32_t M, const 
     else { b = n - 1 - y; c = n - 1 - (int)R; }
 }
 
+// Lexicographic successor of a sorted flip set (the last index varies fastest). Undefined past
+// the last rank (never used there).
+template <int K>
+__device__ __forceinline__ void succ_flip(int n, int &a, int &b, int &c)
+{
+    if (K == 1) {
+        ++a;
+    } else if (K == 2) {
+        if (++b == n) { ++a; b = a + 1; }
+    } else {
+        if (++c == n) {
+            if (++b == n - 1) { ++a; b = a + 1; }
+            c = b + 1;
+        }
+    }
+}
+
 __device__ __forceinline__ void fill_tables(uint32_t *T2, uint32_t *T3, int n)
 {
     for (int i = threadIdx.x; i < n; i += blockDim.x) {
@@ -752,6 +769,37 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     const bool packed = I.m <= PACKED_MAX_M;
     const uint4 *pk = (const uint4 *)(sm + L.pk);
     unsigned long long best = (unsigned long long)KEY_NONE;
+    if (packed && PK_PAIR && !tri && bhi - blo >= 4u * NT) {
+        // large slices (batched searches): each thread owns a contiguous run of ranks, split into
+        // halves A and B evaluated as a pair; flip sets advance by lexicographic successor, so
+        // only the two run starts are unranked
+        const uint32_t span = bhi - blo, tid = threadIdx.x;
+        const uint32_t lo = blo + (uint32_t)(((uint64_t)span * tid) / NT);
+        const uint32_t hi = blo + (uint32_t)(((uint64_t)span * (tid + 1)) / NT);
+        const uint32_t mid = lo + (hi - lo + 1) / 2;
+        int a0, b0, c0, a1, b1, c1;
+        unrank_tab<K>(lo, I.n, M, T2, T3, a0, b0, c0);
+        if (mid < hi) unrank_tab<K>(mid, I.n, M, T2, T3, a1, b1, c1);
+        else { a1 = a0; b1 = b0; c1 = c0; }
+        for (uint32_t rA = lo, rB = mid; rA < mid; ++rA, ++rB) {
+            const bool vB = rB < hi;
+            const uint32_t rb = vB ? rB : rA;
+            if (!vB) { a1 = a0; b1 = b0; c1 = c0; }
+            int fA, fB;
+            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            const bool tA = until && until[rA - ubase] >= t;
+            const bool tB = until && until[rb - ubase] >= t;
+            if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
+            const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
+            const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
+            if ((!tA || (aspire && fA < best_f)) && kA < best) best = kA;
+            if ((!tB || (aspire && fB < best_f)) && kB < best) best = kB;
+            succ_flip<K>(I.n, a0, b0, c0);
+            succ_flip<K>(I.n, a1, b1, c1);
+        }
+        return best;
+    }
     if (packed && PK_PAIR && bhi - blo > (uint32_t)NT) {
         // two neighbours per thread: ranks r and r + 32 (a warp covers 64 consecutive ranks); only
         // when the slice needs more than one pass of the block, else half the warps would idle
