@@ -92,7 +92,6 @@ struct SearchArgs {
     int32_t until_smem;     // cache the CTA's until[] slice in shared memory (1 = yes)
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
-    int32_t no_split;       // 1: evaluate every lattice point (disable the linear-region shortcuts)
     int32_t aspiration;     // a tabu move is admissible when it beats the best fitness so far
     uint32_t *Xg;           // non-null: X lives in global memory, W * n words per CTA (large m x n)
     // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
@@ -128,6 +127,10 @@ __host__ __device__ inline int align16(int x) { return (x + 15) & ~15; }
 #define PK_UNROLL 1
 #endif
 constexpr int kPkUnroll = PK_UNROLL;  // unroll of the packed piece loop
+// byte_perm selectors of the packed records: h = window byte 0 moved to byte 1 (a final piece), or
+// an always-zero byte (byte 7 of the window, unused for K <= 3) for a piece that completes no bin
+#define PK_SEL_FIN 0x7707u
+#define PK_SEL_NONE 0x7777u
 #ifndef PK_PAIR
 #define PK_PAIR 1
 #endif
@@ -165,6 +168,10 @@ struct PlanScalars {
     // destinations negative: cost linear, aggregated as cneg - 240 sum t over the first rneg sorted
     // rows); points u >= utop land only above max(S) (zero cost) and are skipped
     int uneg, utop, rneg, cneg;
+    // packed path (abs form): sum of H_b over the walked bins [uneg, utop + 2K),
+    // H of the 2K trailing bins as bytes, and whether any trailing bin is negative (w != 0)
+    int hwalk, trlin;
+    uint32_t htr_lo, htr_hi;
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
     unsigned long long key, gkey;
     int red[2 * NWARP + 2];
@@ -367,6 +374,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[W] = runp;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
             ps.uneg = uneg; ps.utop = utop; ps.cneg = 0;
+            ps.hwalk = 0; ps.trlin = 0; ps.htr_lo = 0; ps.htr_hi = 0;
             ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
             ps.key = (unsigned long long)KEY_NONE;
             ps.gkey = (unsigned long long)KEY_NONE;
@@ -387,18 +395,21 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     for (int v = tid; v < U; v += NT) {
         const int st = seg[v], en = seg[v + 1];
         int p = pofs[v];
-        // packed-path record of this point's last piece: (mask, 8 | len << 24, H_b, w_b) of its bin
-        // beta = v (b = vmin + 2(v - K)); earlier pieces carry (mask, 0, 0, 0) and finalise nothing
+        // packed-path record of this point's last piece (it completes bin beta = v, b = vmin + 2(v - K)):
+        //   (mask, len, H_b << 8 | 8, PK_SEL_FIN | w_b << 16)
+        // earlier pieces: (mask, 0, 0, PK_SEL_NONE) -- no shift, and h reads an always-zero byte.
+        // The low byte of z is the window shift; the SAD of hb (byte 0 = 0) against z adds it to f,
+        // 8 per final piece, which the constant C takes back
         const int bfin = vmin + 2 * (v - K);
-        const uint32_t Hfin = (bfin >= 0 && bfin <= n) ? (uint32_t)Hs[bfin] : 0u;
-        const uint32_t wfin = bfin < 0 ? (uint32_t)(60 * (-bfin) - 1) : 0u;
+        const uint32_t Hfin = ((bfin >= 0 && bfin <= n) ? (uint32_t)Hs[bfin] << 8 : 0u) | 8u;
+        const uint32_t wfin = PK_SEL_FIN | ((bfin < 0 ? (uint32_t)(60 * (-bfin) - 1) : 0u) << 16);
         // deep-negative constant sum_rows 60(2K - Y_j) - 1 (unsigned: the constant may exceed
         // 2^31 on its own; the fitness it enters does not)
         if (v < uneg && en > st)
             atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - 1));
         if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
             pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
-            if (packed) pk[p] = make_uint4(0u, 8u, Hfin, wfin);
+            if (packed) pk[p] = make_uint4(0u, 0u, Hfin, wfin);
             continue;
         }
         const int w0 = st >> 5, w1 = (en - 1) >> 5;
@@ -407,13 +418,24 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
             pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? 1 : 0) | ((uint32_t)w << 1) | ((uint32_t)(en - st) << 16));
             if (packed)
-                pk[p] = w == w1 ? make_uint4(mask, 8u | ((uint32_t)(en - st) << 24), Hfin, wfin) : make_uint4(mask, 0u, 0u, 0u);
+                pk[p] = w == w1 ? make_uint4(mask, (uint32_t)(en - st), Hfin, wfin)
+                                : make_uint4(mask, 0u, 0u, PK_SEL_NONE);
             if (w > w0 || (st & 31) == 0) pstart[w] = p;
         }
     }
+    const int utop = ps.utop;
     for (int beta = tid; beta < NB; beta += NT) {
         const int b = vmin + 2 * (beta - K);
-        bins[beta] = make_int2((b >= 0 && b <= n) ? Hs[b] : 0, b < 0 ? 60 * (-b) - 1 : 0);
+        const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
+        bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
+        if (packed && beta >= uneg && beta < utop + 2 * K) {
+            if (Hb) atomicAdd(&ps.hwalk, Hb);
+            if (beta >= utop) {
+                const int i = beta - utop;
+                if (Hb) atomicOr(i < 4 ? &ps.htr_lo : &ps.htr_hi, (uint32_t)Hb << (8 * (i & 3)));
+                if (b < 0) atomicOr(&ps.trlin, 1);
+            }
+        }
     }
     __syncthreads();
     PH(2);
@@ -507,6 +529,9 @@ struct EvalRange {
     int p0;           // first piece of point u0
     int p1;           // first piece of point u1 (packed path)
     int w0;           // row word of piece p0 (packed path)
+    int cabs;         // packed path: the fitness constant C
+    int trlin;        // packed path: some trailing bin is negative (scalar trailing)
+    uint32_t htr_lo, htr_hi;
 };
 
 // Deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
@@ -611,15 +636,19 @@ __device__ __forceinline__ void packed_add(uint32_t m, uint32_t lo, uint32_t hi,
 // One packed record applied to one neighbour's window (see eval_fit_packed).
 template <int K>
 __device__ __forceinline__ void packed_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &wlo,
-                                            uint32_t &whi, int &f, int &smin)
+                                            uint32_t &whi, int &f)
 {
     packed_add<K>(r.x, lo, hi, lh, wlo, whi);
-    wlo += r.y >> 24;
-    const int h = (int)(wlo & 0xffu);
-    f += (int)r.w * h;
-    smin += min(h, (int)r.z);
-    wlo = __funnelshift_r(wlo, whi, r.y);  // shift = r.y & 31 (8 or 0)
-    whi = __funnelshift_r(whi, 0u, r.y);
+    wlo += r.y;  // len
+    // hb = h << 8 (h = byte 0 of the window, or 0 for a piece that completes no bin); prmt reads
+    // only the low 16 bits of its selector
+    uint32_t hb, fu = (uint32_t)f;
+    asm("prmt.b32 %0, %1, %2, %3;" : "=r"(hb) : "r"(wlo), "r"(whi), "r"(r.w));
+    fu = __dp2a_lo(r.w, hb, fu);  // + w_b h (w_b in the high half of r.w)
+    asm("vabsdiff4.u32.u32.u32.add %0, %1, %2, %3;" : "=r"(fu) : "r"(hb), "r"(r.z), "r"(fu));  // + |h - H_b| (+ shift)
+    f = (int)fu;
+    wlo = __funnelshift_r(wlo, whi, r.z);  // shift = r.z & 31 (8 or 0)
+    whi = __funnelshift_r(whi, 0u, r.z);
 }
 
 template <int K>
@@ -639,109 +668,90 @@ __device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int
     }
 }
 
-__device__ __forceinline__ void packed_trail(int K2, const int2 *__restrict__ bp, uint32_t wlo, uint32_t whi, int &f,
-                                             int &smin)
+// The 2K bins past the last walked point hold only carried counts (bytes 0 .. 2K-1 of the window;
+// the higher bytes are zero). When none of them is negative their cost is sum |h - H| over the
+// bytes, two SAD instructions against the plan's packed H; otherwise per bin.
+template <int K>
+__device__ __forceinline__ void packed_trail(const EvalRange &er, const int2 *__restrict__ bins, uint32_t wlo,
+                                             uint32_t whi, int &f)
 {
-#pragma unroll
-    for (int i = 0; i < 6; i++) {
-        if (i < K2) {
-            const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
-            const int2 bn = bp[i];
-            f += bn.y * h;
-            smin += min(h, bn.x);
-        }
+    if (!er.trlin) {
+        f += (int)__vsadu4(wlo, er.htr_lo);
+        if (K >= 2) f += (int)__vsadu4(whi, er.htr_hi);
+        return;
     }
-}
-
-// Two neighbours per thread: the record stream, loop control and word bookkeeping are shared.
-template <int K, bool DEEP>
-__device__ __forceinline__ void eval_fit_packed2(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
-                                                 const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
-                                                 const EvalRange &er, int m2, int a0, int b0, int c0, int a1, int b1,
-                                                 int c1, int &f0, int &f1)
-{
-    f0 = m2; f1 = m2;
-    if (DEEP) { f0 = deep_negative<K>(X, n, er, f0, a0, b0, c0); f1 = deep_negative<K>(X, n, er, f1, a1, b1, c1); }
-    if (er.u1 <= er.u0) return;
-    int s0 = 0, s1 = 0;
-    uint32_t wl0 = 0, wh0 = 0, wl1 = 0, wh1 = 0;
-    const uint4 *pp = pk + er.p0;
-    const uint32_t *xr = X + er.w0 * n;
-    const int *pw = pstart + er.w0 + 1;
-    for (;;) {
-        uint32_t lo0, hi0, lh0, lo1, hi1, lh1;
-        load_planes<K>(xr, a0, b0, c0, lo0, hi0, lh0);
-        load_planes<K>(xr, a1, b1, c1, lo1, hi1, lh1);
-        xr += n;
-        const int pend = min(*pw++, er.p1);
-        const uint4 *pe = pk + pend;
-#pragma unroll 1
-        for (; pp < pe; ++pp) {
-            const uint4 r = *pp;
-            packed_step<K>(r, lo0, hi0, lh0, wl0, wh0, f0, s0);
-            packed_step<K>(r, lo1, hi1, lh1, wl1, wh1, f1, s1);
-        }
-        if (pend == er.p1) break;
-    }
-    const int2 *bp = bins + er.u1;
-    packed_trail(2 * K, bp, wl0, wh0, f0, s0);
-    packed_trail(2 * K, bp, wl1, wh1, f1, s1);
-    f0 -= 2 * s0; f1 -= 2 * s1;
-}
-
-template <int K, bool DEEP>
-__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
-                                               const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
-                                               const EvalRange &er, int m2, int a, int b, int c)
-{
-    int f = m2, smin = 0;
-    if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
-    if (er.u1 <= er.u0) return f;
-    uint32_t wlo = 0, whi = 0;
-    const uint4 *pp = pk + er.p0;
-    const uint32_t *xr = X + er.w0 * n;
-    const int *pw = pstart + er.w0 + 1;
-    for (;;) {
-        uint32_t lo, hi = 0, lh = 0;
-        if (K == 1) {
-            lo = xr[a];
-        } else if (K == 2) {
-            const uint32_t xa = xr[a], xb = xr[b];
-            lo = xa ^ xb; hi = xa & xb;
-        } else {
-            const uint32_t xa = xr[a], xb = xr[b], xc = xr[c];
-            lo = xa ^ xb ^ xc;
-            hi = (xa & xb) | (xc & (xa ^ xb));
-            lh = lo & hi;
-        }
-        xr += n;
-        const int pend = min(*pw++, er.p1);
-        const uint4 *pe = pk + pend;
-        // every record is applied the same way: a non-final piece has len = shift = H = w = 0,
-        // so its "bin" costs 0 and the window does not move
-#pragma unroll kPkUnroll
-        for (; pp < pe; ++pp) {
-            const uint4 r = *pp;
-            packed_add<K>(r.x, lo, hi, lh, wlo, whi);
-            wlo += r.y >> 24;
-            const int h = (int)(wlo & 0xffu);
-            f += (int)r.w * h;
-            smin += min(h, (int)r.z);
-            wlo = __funnelshift_r(wlo, whi, r.y);  // shift = r.y & 31 (8 or 0)
-            whi = __funnelshift_r(whi, 0u, r.y);
-        }
-        if (pend == er.p1) break;
-    }
-    // bins beta .. beta+2K-1 past the last point hold only carried counts
     const int2 *bp = bins + er.u1;
 #pragma unroll
     for (int i = 0; i < 2 * K; i++) {
         const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
         const int2 bn = bp[i];
-        f += bn.y * h;
-        smin += min(h, bn.x);
+        f += bn.y * h + abs(h - bn.x);
     }
-    return f - 2 * smin;
+}
+
+// eval_fit for m <= 255, abs form:
+//   f = C + [deep rows] + sum over walked bins beta of ( w_beta h_beta + |h_beta - H_beta| )
+// with C = m - sum_{walked b in [0,n]} H_b + (rows above the top cut). Two neighbours per thread:
+// the record stream, loop control and word bookkeeping are shared.
+template <int K, bool DEEP>
+__device__ __forceinline__ void eval_fit_packed2(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
+                                                 const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
+                                                 const EvalRange &er, int a0, int b0, int c0, int a1, int b1,
+                                                 int c1, int &f0, int &f1)
+{
+    f0 = er.cabs; f1 = er.cabs;
+    if (DEEP) { f0 = deep_negative<K>(X, n, er, f0, a0, b0, c0); f1 = deep_negative<K>(X, n, er, f1, a1, b1, c1); }
+    uint32_t wl0 = 0, wh0 = 0, wl1 = 0, wh1 = 0;
+    if (er.u1 > er.u0) {
+        const uint4 *pp = pk + er.p0;
+        const uint32_t *xr = X + er.w0 * n;
+        const int *pw = pstart + er.w0 + 1;
+        for (;;) {
+            uint32_t lo0, hi0, lh0, lo1, hi1, lh1;
+            load_planes<K>(xr, a0, b0, c0, lo0, hi0, lh0);
+            load_planes<K>(xr, a1, b1, c1, lo1, hi1, lh1);
+            xr += n;
+            const int pend = min(*pw++, er.p1);
+            const uint4 *pe = pk + pend;
+#pragma unroll kPkUnroll
+            for (; pp < pe; ++pp) {
+                const uint4 r = *pp;
+                packed_step<K>(r, lo0, hi0, lh0, wl0, wh0, f0);
+                packed_step<K>(r, lo1, hi1, lh1, wl1, wh1, f1);
+            }
+            if (pend == er.p1) break;
+        }
+    }
+    packed_trail<K>(er, bins, wl0, wh0, f0);
+    packed_trail<K>(er, bins, wl1, wh1, f1);
+}
+
+// One neighbour per thread (slices of at most one block pass).
+template <int K, bool DEEP>
+__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
+                                               const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
+                                               const EvalRange &er, int a, int b, int c)
+{
+    int f = er.cabs;
+    if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
+    uint32_t wlo = 0, whi = 0;
+    if (er.u1 > er.u0) {
+        const uint4 *pp = pk + er.p0;
+        const uint32_t *xr = X + er.w0 * n;
+        const int *pw = pstart + er.w0 + 1;
+        for (;;) {
+            uint32_t lo, hi, lh;
+            load_planes<K>(xr, a, b, c, lo, hi, lh);
+            xr += n;
+            const int pend = min(*pw++, er.p1);
+            const uint4 *pe = pk + pend;
+#pragma unroll kPkUnroll
+            for (; pp < pe; ++pp) packed_step<K>(*pp, lo, hi, lh, wlo, whi, f);
+            if (pend == er.p1) break;
+        }
+    }
+    packed_trail<K>(er, bins, wlo, whi, f);
+    return f;
 }
 
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
@@ -750,7 +760,7 @@ template <int K, bool WRITE_ALL, bool XG = false>
 __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *sm, const Smem &L,
                                          const PlanScalars &ps, const uint32_t *Xarg, uint32_t M, uint32_t blo, uint32_t bhi,
                                          const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
-                                         const uint2 *tri = nullptr, int no_split = 0, int aspire = 0,
+                                         const uint2 *tri = nullptr, int aspire = 0,
                                          int best_f = 0)
 {
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -759,14 +769,18 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     const uint2 *pieces = (const uint2 *)(sm + L.pieces);
     const int2 *bins = (const int2 *)(sm + L.bins);
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
+    const bool packed = I.m <= PACKED_MAX_M;
     EvalRange er;
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
-    if (no_split) { er.u0 = 0; er.u1 = ps.U; er.rneg = 0; er.cneg = 0; er.p0 = 0; }
     er.p1 = ((const int *)(sm + L.pofs))[er.u1];
+    if (packed) {  // abs form: deep rows cost 60 |b| (no -1), C as in eval_fit_packed2
+        er.cneg = ps.cneg + ps.rneg;
+        er.cabs = 2 * I.m - ps.hwalk - ((const int *)(sm + L.seg))[er.u1] - 8 * (er.u1 - er.u0);
+        er.trlin = ps.trlin; er.htr_lo = ps.htr_lo; er.htr_hi = ps.htr_hi;
+    }
     er.w0 = (int)((pieces[er.p0].y >> 1) & 0x7fffu);
     const int *pstart = (const int *)(sm + L.pstart);
-    const bool packed = I.m <= PACKED_MAX_M;
     const uint4 *pk = (const uint4 *)(sm + L.pk);
     unsigned long long best = (unsigned long long)KEY_NONE;
     if (packed && PK_PAIR && !tri && bhi - blo >= 4u * NT) {
@@ -786,8 +800,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const uint32_t rb = vB ? rB : rA;
             if (!vB) { a1 = a0; b1 = b0; c1 = c0; }
             int fA, fB;
-            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
-            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
             const bool tA = until && until[rA - ubase] >= t;
             const bool tB = until && until[rb - ubase] >= t;
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
@@ -818,8 +832,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 unrank_tab<K>(rb, I.n, M, T2, T3, a1, b1, c1);
             }
             int fA, fB;
-            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
-            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a0, b0, c0, a1, b1, c1, fA, fB);
+            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
             const bool tA = until && until[rA - ubase] >= t;
             const bool tB = until && until[rb - ubase] >= t;
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
@@ -842,8 +856,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 } else {
                     unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
                 }
-                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pk, pstart, bins, I.n, er, 2 * I.m, a, b, c)
-                                                    : eval_fit_packed<K, false>(X, pk, pstart, bins, I.n, er, 2 * I.m, a, b, c))
+                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pk, pstart, bins, I.n, er, a, b, c)
+                                                    : eval_fit_packed<K, false>(X, pk, pstart, bins, I.n, er, a, b, c))
                                      : (er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
                                                     : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c));
                 if (WRITE_ALL) fit_out[r] = f;
@@ -1084,9 +1098,9 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr);
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                  nullptr, tri, A.no_split, A.aspiration, (int)best_f)
+                                                  nullptr, tri, A.aspiration, (int)best_f)
                      : eval_range<K, false, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                   nullptr, tri, A.no_split, A.aspiration, (int)best_f);
+                                                   nullptr, tri, A.aspiration, (int)best_f);
             mine = warp_min_k(mine);
             if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
             __syncthreads();
@@ -1190,9 +1204,9 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
     const uint32_t t = (uint32_t)(A.fs[FS_T] + 1);
     unsigned long long mine =
         A.Xg ? eval_range<K, WRITE_ALL, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, A.until, 0, t, fit_out,
-                                              nullptr, 0, A.aspiration, (int)A.fs[FS_BEST])
+                                              nullptr, A.aspiration, (int)A.fs[FS_BEST])
              : eval_range<K, WRITE_ALL, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, A.until, 0, t, fit_out,
-                                               nullptr, 0, A.aspiration, (int)A.fs[FS_BEST]);
+                                               nullptr, A.aspiration, (int)A.fs[FS_BEST]);
     mine = warp_min_k(mine);
     if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
     __syncthreads();
@@ -1478,7 +1492,6 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
-    A.no_split = 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     return A;
