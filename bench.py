@@ -341,18 +341,30 @@ def main():
     kern_avg_s = kern_ms / 1e3 / args.steps
     achieved = (my_iters / args.steps) * M * ops_per_nbr / kern_avg_s / 1e12 if kern_avg_s > 0 else 0.0
     peak = sms * 128 * mhz * 1e6 / 1e12  # 128 integer lanes issued per SM per clock (4 SMSP x 1 warp-instr)
-    traffic = None
+    traffic, per_nbr = None, None
     prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_bench.json")  # ncu --set full of one bench step
     if os.path.exists(prof):
         try:
             with open(prof) as fh:
-                traffic = json.load(fh).get("dram_bytes_per_launch")
+                pj = json.load(fh)
+            traffic, per_nbr = pj.get("dram_bytes_per_launch"), pj.get("per_neighbor")
         except (OSError, ValueError):
             traffic = None
+    nbr_per_s_kernel = (my_iters / args.steps) * M / kern_avg_s if kern_avg_s > 0 else 0.0
     roofline = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tops/s", "frac": achieved / peak,
                 "traffic": traffic, "kernel": "k_search<3> (persistent, batched searches)",
                 "peak_source": f"{sms} SMs x 128 int lanes/clk x {mhz:.0f} MHz ({src} sm_max_mhz)",
-                "ops_per_neighbor": ops_per_nbr}
+                "ops_per_neighbor": ops_per_nbr,
+                "ops_model": "SURVEY.md §8(d): m(k+4) integer ops per neighbour; the bit-sliced kernel issues fewer"}
+    if per_nbr:
+        # what the kernel actually issues (ncu source page of the committed capture, same kernel and job)
+        ipn, ppn = per_nbr["issued_instructions"], per_nbr["popc"]
+        roofline["issued"] = {"instructions_per_neighbor": ipn, "achieved": nbr_per_s_kernel * ipn / 1e12,
+                              "frac": nbr_per_s_kernel * ipn / 1e12 / peak}
+        # the pipe that binds the piece loop: POPC on XU at 1/8 of the issue rate (16 lanes/clk/SM)
+        xu_ceiling = sms * 16 * mhz * 1e6 / ppn
+        roofline["binding_pipe"] = {"pipe": "xu (POPC, 16 lanes/clk/SM)", "popc_per_neighbor": ppn,
+                                    "ceiling_neighbors_per_s": xu_ceiling, "frac": nbr_per_s_kernel / xu_ceiling}
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:

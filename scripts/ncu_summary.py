@@ -39,6 +39,8 @@ def main():
     ap.add_argument("out")
     ap.add_argument("--kernel", required=True)
     ap.add_argument("--capture", required=True)
+    ap.add_argument("--source", help="`--page source --csv` export of the same capture (per-SASS counts)")
+    ap.add_argument("--units", type=float, default=0.0, help="neighbour evaluations in the profiled launch")
     a = ap.parse_args()
     with open(a.raw) as fh:
         rows = list(csv.reader(fh))
@@ -56,6 +58,23 @@ def main():
     out = {"kernel": a.kernel, "capture": a.capture,
            "dram_bytes_per_launch": nbytes("dram__bytes_read.sum") + nbytes("dram__bytes_write.sum"),
            "metrics": metrics}
+    if a.source and a.units:
+        src = list(csv.reader(open(a.source)))
+        h = src[1]
+        isrc, ie = h.index("Source"), h.index("Instructions Executed")
+        tot = popc = 0
+        for r in src[2:]:
+            if len(r) <= ie:
+                continue
+            e = int(r[ie] or 0)
+            tot += e
+            op = r[isrc].split()
+            op = op[1] if op and op[0].startswith("@") and len(op) > 1 else (op[0] if op else "")
+            if op == "POPC":
+                popc += e
+        # warp-level counts x 32 lanes / neighbours = per-neighbour (per-lane) instruction counts
+        out["per_neighbor"] = {"units": a.units, "issued_instructions": 32 * tot / a.units,
+                               "popc": 32 * popc / a.units}
     with open(a.out, "w") as fh:
         json.dump(out, fh, indent=1)
     print(json.dumps(out, indent=1)[:3000])
