@@ -161,7 +161,8 @@ lns_status lns_step_end(lns_ctx *ctx, int8_t *V_out, int64_t *trace_rank, int64_
 /* lns_last_kernel_ms -- device time (CUDA events) of the hot kernel(s) of the last run or eval. */
 double lns_last_kernel_ms(lns_ctx *ctx);
 
-/* lns_config -- override launch parameters (0 = automatic): blocks per search. */
+/* lns_config -- override launch parameters (0 = automatic): CTAs per search (lns_tabu_run,
+ * the stepped API) and CTAs of lns_eval_all / lns_eval_neighborhood. Results never depend on it. */
 lns_status lns_config(lns_ctx *ctx, int32_t blocks);
 
 int64_t lns_neighborhood_size(int32_t n, int32_t k); /* C(n,k), or -1 if k not in {1,2,3} */

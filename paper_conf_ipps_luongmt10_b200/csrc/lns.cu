@@ -73,6 +73,8 @@ __device__ unsigned long long g_ph[NPH];
 // ------------------------------------------------------------------------------------------
 struct DevInst {
     int32_t m, n, W, NWn;  // W = ceil(m/32) row words, NWn = ceil(n/32) column words
+    int32_t XW;            // row words X has room for: W, or 2W + 1 with padded placement
+    int32_t pad;           // padded placement: no segment of <= 32 rows straddles a row word
     const uint32_t *Arow;  // m x NWn, bit (i%32) of word i/32 = 1 <=> A[j][i] = -1
     const int32_t *H;      // n+1 bins of S
     int32_t maxS;          // largest b with H_b > 0
@@ -93,7 +95,7 @@ struct SearchArgs {
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     int32_t aspiration;     // a tabu move is admissible when it beats the best fitness so far
-    uint32_t *Xg;           // non-null: X lives in global memory, W * n words per CTA (large m x n)
+    uint32_t *Xg;           // non-null: X lives in global memory, XW * n words per CTA (large m x n)
     // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
     // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
     // search from the state in (vb, Y, fs).
@@ -111,7 +113,7 @@ struct SearchArgs {
 };
 
 // The CTA's X (sorted sign bits): shared memory, or its own slot of the global fallback buffer.
-#define X_OF(A, sm, L) ((A).Xg ? (A).Xg + (size_t)blockIdx.x * (A).I.W * (A).I.n : (uint32_t *)((sm) + (L).X))
+#define X_OF(A, sm, L) ((A).Xg ? (A).Xg + (size_t)blockIdx.x * (A).I.XW * (A).I.n : (uint32_t *)((sm) + (L).X))
 
 // Shared-memory carve-up (identical on host and device). The bit-packed A (Ar) and the until[]
 // slice are staged only when they fit.
@@ -135,6 +137,7 @@ constexpr int kPkUnroll = PK_UNROLL;  // unroll of the packed piece loop
 #define PK_PAIR 1
 #endif
 
+// XW = row words of X (I.XW: W, or 2W + 1 with padded placement)
 __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0)
 {
     Smem s;
@@ -147,7 +150,7 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
     s.seg = o;    o = align16(o + 4 * (n + 2));          // seg[0..U], U <= n + 1
     s.cur = o;    o = align16(o + 4 * (n + 2 + 2 * K));
     s.pofs = o;   o = align16(o + 4 * (n + 2));
-    s.rowAt = o;  o = align16(o + 4 * m);
+    s.rowAt = o;  o = align16(o + 4 * (m > 32 * W ? m : 32 * W));  // row slots (holes = -1 when padded)
     s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
     s.pieces = o; o = align16(o + 8 * (n + 2 + W));      // P <= U + W - 1 pieces (+1 prefetch pad)
     s.pk = o;     o = align16(o + (m <= PACKED_MAX_M ? 16 * (n + 2 + W) : 0));  // packed-path pieces
@@ -171,6 +174,8 @@ struct PlanScalars {
     // packed path (abs form): sum of H_b over the walked bins [uneg, utop + 2K),
     // H of the 2K trailing bins as bytes, and whether any trailing bin is negative (w != 0)
     int hwalk, trlin;
+    int Wp;    // row words X holds this plan (ceil(row slots / 32); padded slots are holes)
+    int rtop;  // rows below the top cut (points < utop), unpadded
     uint32_t htr_lo, htr_hi;
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
     unsigned long long key, gkey;
@@ -318,7 +323,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
 {
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
-    const int m = I.m, n = I.n, W = I.W, NWn = I.NWn;
+    const int m = I.m, n = I.n, NWn = I.NWn;
     const int *Ys = (const int *)(sm + L.Y);
     const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
     const int *Hs = (const int *)(sm + L.H);
@@ -332,8 +337,9 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     int *pstart = (int *)(sm + L.pstart);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
-    // A. counting sort over the conservative lattice
+    // A. counting sort over the conservative lattice (and mark every row slot a hole)
     for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
+    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
     __syncthreads();
     PH(0);
     // B. warp 0: exact range (first / last non-empty point), exclusive scans of the row and piece
@@ -369,9 +375,36 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         uneg = min(max(uneg, 0), U);
         int utop = ((I.maxS + 2 * K - vmin_) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
+        int Wp = (m + 31) >> 5;
+        __syncwarp();
+        if (lane == 0) ps.rtop = utop < U ? seg[utop] : runr;  // unpadded rows below the top cut
+        if (I.pad) {
+            // padded placement: segments go in order; one that would straddle a row
+            // word while starting mid-word starts at the next word instead, so it stays one piece.
+            // At most 2W + 1 words (a word is left short only when the next segment does not fit).
+            __syncwarp();
+            int pos = 0;
+            runp = 0;
+            for (int b0 = 0; b0 < U; b0 += 32) {
+                const int v_ = b0 + lane;
+                const int L = v_ < U ? cnt[uf + v_] : 0;
+                int myP = 0, myO = 0;
+                const int nv = min(32, U - b0);
+                for (int i = 0; i < nv; i++) {
+                    const int Li = __shfl_sync(FULL, L, i);
+                    if (Li > 0 && (pos & 31) != 0 && (pos & 31) + Li > 32) pos = (pos + 31) & ~31;
+                    if (lane == i) { myP = pos; myO = runp; }
+                    runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : 1;
+                    pos += Li;
+                }
+                if (v_ < U) { seg[v_] = myP; cur[uf + v_] = myP; pofs[v_] = myO; }
+            }
+            runr = pos;
+            Wp = (pos + 31) >> 5;
+        }
         if (lane == 0) {
             const int vmin = vmin_;
-            seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[W] = runp;
+            seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[Wp] = runp; ps.Wp = Wp;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
             ps.uneg = uneg; ps.utop = utop; ps.cneg = 0;
             ps.hwalk = 0; ps.trlin = 0; ps.htr_lo = 0; ps.htr_hi = 0;
@@ -393,7 +426,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     uint4 *pk = (uint4 *)(sm + L.pk);
     const bool packed = m <= PACKED_MAX_M;
     for (int v = tid; v < U; v += NT) {
-        const int st = seg[v], en = seg[v + 1];
+        const int st = seg[v], en = st + cnt[uf + v];  // padded start, real length
         int p = pofs[v];
         // packed-path record of this point's last piece (it completes bin beta = v, b = vmin + 2(v - K)):
         //   (mask, len, H_b << 8 | 8, PK_SEL_FIN | w_b << 16)
@@ -405,8 +438,9 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         const uint32_t wfin = PK_SEL_FIN | ((bfin < 0 ? (uint32_t)(60 * (-bfin) - 1) : 0u) << 16);
         // deep-negative constant sum_rows 60(2K - Y_j) - 1 (unsigned: the constant may exceed
         // 2^31 on its own; the fitness it enters does not)
+        // (the packed path's abs form counts 60 |b| per deep row, without the -1: DESIGN.md §5.9)
         if (v < uneg && en > st)
-            atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - 1));
+            atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - (packed ? 0 : 1)));
         if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
             pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
             if (packed) pk[p] = make_uint4(0u, 0u, Hfin, wfin);
@@ -442,10 +476,12 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     // D. X[w][c]: per (row word, column word) pair, lane l loads sorted row 32w+l's sign bits of
     //    columns 32cw..32cw+31 and a 5-round shuffle transpose turns rows into columns; zero cnt[]
     for (int u = tid; u < Uc; u += NT) cnt[u] = 0;
-    for (int pr = warp; pr < W * NWn; pr += NWARP) {
+    const int Wp = ps.Wp;
+    for (int pr = warp; pr < Wp * NWn; pr += NWARP) {
         const int w = pr / NWn, cw = pr - w * NWn;
         const int p = 32 * w + lane;
-        uint32_t x = p < m ? (Ar[(size_t)rowAt[p] * NWn + cw] ^ vbs[cw]) : 0u;
+        const int j = I.pad ? rowAt[p] : (p < m ? rowAt[p] : -1);
+        uint32_t x = j >= 0 ? (Ar[(size_t)j * NWn + cw] ^ vbs[cw]) : 0u;
 #pragma unroll
         for (int j = 16; j >= 1; j >>= 1) {
             const uint32_t mk = j == 16 ? 0x0000FFFFu : j == 8 ? 0x00FF00FFu : j == 4 ? 0x0F0F0F0Fu
@@ -774,9 +810,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
     er.p1 = ((const int *)(sm + L.pofs))[er.u1];
-    if (packed) {  // abs form: deep rows cost 60 |b| (no -1), C as in eval_fit_packed2
-        er.cneg = ps.cneg + ps.rneg;
-        er.cabs = 2 * I.m - ps.hwalk - ((const int *)(sm + L.seg))[er.u1] - 8 * (er.u1 - er.u0);
+    if (packed) {  // abs form (deep rows: 60 |b| each, accumulated so by build_plan); C as in eval_fit_packed2
+        er.cabs = 2 * I.m - ps.hwalk - ps.rtop - 8 * (er.u1 - er.u0);
         er.trlin = ps.trlin; er.htr_lo = ps.htr_lo; er.htr_hi = ps.htr_hi;
     }
     er.w0 = (int)((pieces[er.p0].y >> 1) & 0x7fffu);
@@ -1036,7 +1071,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
     const int G = A.groups > 0 ? A.groups : 1;
@@ -1190,7 +1225,7 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     const int lane = threadIdx.x & 31;
     if (!WRITE_ALL && A.fs[FS_DONE]) {
         if (blockIdx.x == 0 && threadIdx.x == 0) *key_out = KEY_NONE;
@@ -1269,7 +1304,7 @@ __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.W, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     const uint32_t *Ar = load_state<K>(A, sm, L, ps);
     const int *segp = (const int *)(sm + L.seg);
     if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
@@ -1284,7 +1319,7 @@ __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out
         for (int u = 0; u <= U; u++) out[o++] = segp[u];
         for (int q = 0; q < ps.NB; q++) { out[o++] = bins[q].x; out[o++] = bins[q].y; }
         for (int q = 0; q < ps.P; q++) { out[o++] = (int)pieces[q].x; out[o++] = (int)pieces[q].y; }
-        for (int w = 0; w <= A.I.W; w++) out[o++] = pstart[w];
+        for (int w = 0; w <= ps.Wp; w++) out[o++] = pstart[w];
     }
 }
 
@@ -1344,6 +1379,7 @@ struct lns_ctx {
     void *comm = nullptr;
     nccl_allreduce_fn nccl_allreduce = nullptr;
     int blocks_override = 0;
+    int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
     // run state
     uint32_t *d_vb = nullptr;
     int32_t *d_Y = nullptr;
@@ -1396,7 +1432,7 @@ int64_t comb_k(int64_t n, int k)
     return -1;
 }
 
-DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->d_Arow, c->d_H, c->maxS}; }
+DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->W, 0, c->d_Arow, c->d_H, c->maxS}; }
 
 template <typename T>
 lns_status grow(T *&p, size_t &cap, size_t need)
@@ -1442,6 +1478,7 @@ struct Geometry {
     uint32_t M = 0;
     int a_in_smem = 0;
     int x_global = 0;      // X does not fit in shared memory: per-CTA slots in global memory
+    int pad = 0, XW = 0;   // padded placement (packed path, when X of 2W + 1 words fits)
     size_t smem_eval = 0;  // bytes for the stepped / eval kernels
 };
 
@@ -1455,6 +1492,16 @@ lns_status check_k(lns_ctx *c, int k, Geometry &g)
     g.M = (uint32_t)Mk;
     const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
     // preference: X and A in shared memory; X only; neither (X in global memory)
+    // padded placement first (packed path only): X of 2W + 1 words, with or without A staged
+    g.pad = 0; g.XW = c->W;
+    if (c->m <= PACKED_MAX_M && !c->no_pad) {
+        const int XWp = 2 * c->W + 1;
+        const Smem pw = smem_layout(c->m, c->n, XWp, c->NWn, k, 1);
+        const Smem pwo = smem_layout(c->m, c->n, XWp, c->NWn, k, 0);
+        if (pw.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 1; g.smem_eval = (size_t)pw.a_end; }
+        else if (pwo.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 0; g.smem_eval = (size_t)pwo.a_end; }
+        if (g.pad) return LNS_OK;
+    }
     const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1);
     const Smem without = smem_layout(c->m, c->n, c->W, c->NWn, k, 0);
     const Smem xg = smem_layout(c->m, c->n, c->W, c->NWn, k, 0, 1);
@@ -1484,6 +1531,8 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
 {
     SearchArgs A;
     A.I = dev_inst(c);
+    A.I.XW = g.XW > 0 ? g.XW : c->W;
+    A.I.pad = 0;  // per launch: pad_for()
     A.M = g.M;
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
@@ -1566,6 +1615,13 @@ size_t cache_geometry(SearchArgs &A, const Geometry &g, int nb, int budget)
     return smem;
 }
 
+// Padded placement pays off when a CTA evaluates many neighbours per plan (it adds a serial warp
+// pass to every plan build): the same slice test as the contiguous-run evaluation path.
+inline int pad_for(const Geometry &g, uint32_t span, int nb)
+{
+    return (g.pad && span / (uint32_t)std::max(nb, 1) >= 4u * NT) ? 1 : 0;
+}
+
 template <int K>
 lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st)
 {
@@ -1577,6 +1633,7 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
     const int nb = search_blocks(c, A.hi - A.lo, 1);
+    A.I.pad = pad_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
     k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
@@ -1593,6 +1650,7 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int G, int 
 {
     const int budget = c->smemOptin - 1024;
     CK(cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, budget));
+    A.I.pad = pad_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
     if (!A.until_smem) {  // one global until[] per concurrent group
         lns_status s = grow(c->d_until, c->until_cap, (size_t)G * g.M);
@@ -1623,8 +1681,11 @@ lns_status launch_step_eval(lns_ctx *c, const SearchArgs &A, const Geometry &g, 
     int nb = search_blocks(c, A.hi - A.lo, occ);
     if (all) {
         nb = (int)std::min<int64_t>(std::max<int64_t>(1, (A.hi - A.lo) / 1024), 4LL * c->numSMs * occ);
+        if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs * occ);
+        a.I.pad = pad_for(g, A.hi - A.lo, nb);
         k_step_eval<K, true><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     } else {
+        a.I.pad = pad_for(g, A.hi - A.lo, nb);
         k_step_eval<K, false><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     }
     CK(cudaGetLastError());
@@ -1732,6 +1793,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     }
     lns_ctx *c = new lns_ctx();
     c->device = device; c->m = m; c->n = n; c->W = W; c->NWn = NWn;
+    { const char *e = getenv("LNS_NO_PAD"); c->no_pad = (e && e[0] == '1') ? 1 : 0; }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };
@@ -2051,6 +2113,17 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     }
     return LNS_OK;
 }
+
+#ifdef LNS_PHASE_TIMING
+// Profiling build only: per-phase cycle sums of thread 0 of every CTA since the last call (PH()).
+lns_status lns_debug_phases(unsigned long long *out8)
+{
+    CK(cudaMemcpyFromSymbol(out8, g_ph, sizeof(unsigned long long) * NPH));
+    unsigned long long z[NPH] = {0};
+    CK(cudaMemcpyToSymbol(g_ph, z, sizeof(z)));
+    return LNS_OK;
+}
+#endif
 
 // Undocumented debug export (tests/tools only): plan of V for neighbourhood k, see k_debug_plan.
 lns_status lns_debug_plan(lns_ctx *c, int32_t k, const int8_t *V, int32_t *out_host, int64_t cap)

@@ -395,3 +395,21 @@ def test_large_instance_global_X_fallback(L, orc, k):
         else:
             ranks = np.unique(np.random.default_rng(2).integers(0, M, 4000))
             assert np.array_equal(got[ranks], orc.eval_ranks(inst.A, inst.S, V, 2, ranks))
+
+
+@pytest.mark.parametrize("m,n,k", [(m, n, k) for (m, n, k) in SHAPES if comb(n, k) >= 4096])
+def test_eval_all_large_slices(L, orc, m, n, k):
+    """One CTA for the whole neighbourhood: slices of >= 4 block passes take the batched-search
+    evaluation path (two neighbours per thread over contiguous rank runs, lexicographic successor)
+    and, for m <= 255, the padded row placement -- every fitness vs the oracle."""
+    inst = pi.planted_instance(m, n, 7000 + m * 31 + n)
+    rng = np.random.default_rng(m * n + k + 1)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        L.lns_config(ctx, 1)
+        for V in _states(inst, rng, count=2):
+            got = L.lns_eval_all(ctx, k, V)
+            want = orc.eval_all(inst.A, inst.S, V, k)
+            assert np.array_equal(got.astype(np.int64), want)
+    finally:
+        L.lns_destroy(ctx)
