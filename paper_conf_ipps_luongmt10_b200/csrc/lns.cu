@@ -2049,15 +2049,17 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     // groups: as many concurrent searches as SMs allow; CTAs per group = SMs / groups; a global
     // until[] per group (when it is not cached in shared memory) is capped at 8 GiB
     // choose G to minimise the makespan ceil(R/G) * T(SMs/G) with the iteration-time model
-    // T(nb) = 5 us + 3e-5 us * M (m + 32) / nb (fixed plan/exchange cost + evaluation spread over
-    // nb SMs; calibrated on C2-C4)
+    // T(nb) = (2 + 7.5e-4 m n) us + 1.63e-5 us * M (m + 32) / nb: a per-iteration cost of every
+    // CTA (plan build, exchange, move, per-thread run start-up; grows with m n) plus evaluation
+    // spread over nb SMs. Fitted on C2-C4 batches of 50 (nb = 2..14).
     int G = 1;
     {
         double best = 1e300;
-        const double work = 3e-5 * (double)g.M * (double)(c->m + 32);
+        const double work = 1.63e-5 * (double)g.M * (double)(c->m + 32);
+        const double fixed = 2.0 + 7.5e-4 * (double)c->m * (double)c->n;
         for (int q = 1; q <= std::min<int>(R, c->numSMs); q++) {
             const int nbq = c->numSMs / q;
-            const double mk = (double)((R + q - 1) / q) * (5.0 + work / nbq);
+            const double mk = (double)((R + q - 1) / q) * (fixed + work / nbq);
             if (mk < best * 0.999) { best = mk; G = q; }
         }
     }
