@@ -48,11 +48,19 @@ typedef int32_t lns_status;
 #define LNS_ECUDA (-4)          /* CUDA runtime error (message in lns_last_error) */
 #define LNS_ENCCL (-5)          /* NCCL missing or failed */
 #define LNS_ENOADMISSIBLE (-6)  /* every neighbour is tabu (best_rank = -1) */
+#define LNS_EPEER (-7)          /* device-side peer exchange: a partition did not arrive in time */
+
+#define LNS_IPC_HANDLE_BYTES 64 /* size of a cudaIpcMemHandle_t (lns_exchange_ipc_handle) */
 
 #define LNS_STOP_ON_ZERO 1      /* stop the search when f = 0 */
 #define LNS_FORCE_STEPPED 2     /* run one launch sequence per iteration instead of the persistent kernel */
 #define LNS_ASPIRATION 4        /* variant (not the default, reading R4'): a tabu move is admissible when its
                                    fitness is below the best fitness found so far (Taillard [11]) */
+#define LNS_PLAIN_LAUNCH 8      /* lns_tabu_run: launch the persistent kernel with a plain launch instead of
+                                   a cooperative one. The driver serialises cooperative launches, so several
+                                   peer partitions on ONE device (tests, emulation) need this; co-residency
+                                   is then not guaranteed (an idle device with room for all CTAs gives it;
+                                   the peer exchange times out otherwise). */
 
 typedef struct lns_ctx lns_ctx;
 
@@ -140,6 +148,38 @@ lns_status lns_set_partition(lns_ctx *ctx, int32_t part, int32_t nparts);
  *   the process, e.g. torch's) for multi-GPU lns_tabu_run; sets the partition to (rank, world).
  *   The communicator is not freed by the library. comm = NULL detaches. Errors: ENCCL. */
 lns_status lns_attach_comm(lns_ctx *ctx, void *nccl_comm, int32_t rank, int32_t world);
+
+/* Device-initiated multi-GPU exchange (the partition of P:448-454 with
+ * the per-iteration argmin moved inside the persistent kernel, no host collective):
+ *   Every partition's kernel owns a 512-byte exchange buffer in its device memory. At iteration t
+ *   every CTA of every partition MINs its best key into slot t mod 3 of EVERY partition's buffer
+ *   (red.min.sys over NVLink peer memory) and then bumps every partition's arrival counter
+ *   (red.release.sys); it proceeds once its own counter shows all CTAs of all partitions
+ *   (ld.acquire.sys), reads its own slot (the global minimum) and applies the move. A partition
+ *   that does not arrive within timeout_ms ends the run with LNS_EPEER (no hang).
+ *   lns_exchange_buffer      -- this context's exchange buffer (device pointer; allocated here).
+ *   lns_exchange_ipc_handle  -- its cudaIpcMemHandle_t (LNS_IPC_HANDLE_BYTES, host) for other
+ *                               processes (one process per GPU).
+ *   lns_attach_peers         -- set the partition (part of nparts) and the exchange buffers of all
+ *                               partitions, bufs[q] a device pointer usable from this context's
+ *                               device (bufs[part] = this context's own buffer; peers on other
+ *                               GPUs need peer access enabled). nparts = 1 or bufs = NULL detaches.
+ *   lns_attach_peers_ipc     -- the same from nparts handles (host, nparts x LNS_IPC_HANDLE_BYTES,
+ *                               gathered from every partition); opens the other partitions'
+ *                               buffers with cudaIpcOpenMemHandle (closed by lns_destroy).
+ *   lns_exchange_reset       -- clear this context's own buffer and wait for it. Before EVERY
+ *                               lns_tabu_run with peers attached, every partition must reset its
+ *                               buffer and pass a host barrier, then all call lns_tabu_run with
+ *                               identical arguments (each evaluates its slice; the trajectory is
+ *                               the single-GPU one). Only lns_tabu_run uses the peers.
+ *   Errors: EINVAL (bad partition / pointers), ENOMEM, ECUDA (IPC); lns_tabu_run: EPEER. */
+lns_status lns_exchange_buffer(lns_ctx *ctx, void **buf_dev);
+lns_status lns_exchange_ipc_handle(lns_ctx *ctx, void *handle_out);
+lns_status lns_attach_peers(lns_ctx *ctx, int32_t part, int32_t nparts, void *const *bufs,
+                            int64_t timeout_ms);
+lns_status lns_attach_peers_ipc(lns_ctx *ctx, int32_t part, int32_t nparts, const void *handles,
+                                int64_t timeout_ms);
+lns_status lns_exchange_reset(lns_ctx *ctx, void *stream);
 
 /* Stepped interface (one iteration at a time; used by multi-process drivers that own the
  * collective, e.g. torch.distributed):

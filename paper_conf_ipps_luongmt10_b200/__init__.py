@@ -26,10 +26,13 @@ LNS_ENOMEM = -3
 LNS_ECUDA = -4
 LNS_ENCCL = -5
 LNS_ENOADMISSIBLE = -6
+LNS_EPEER = -7
 LNS_STOP_ON_ZERO = 1
 LNS_FORCE_STEPPED = 2
 LNS_ASPIRATION = 4
+LNS_PLAIN_LAUNCH = 8
 KEY_NONE = (1 << 63) - 1
+LNS_IPC_HANDLE_BYTES = 64
 
 RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_iter", "solved")
 
@@ -61,6 +64,11 @@ _SIGS = {
     "lns_unrank": (_i32, [_i32, _i32, _vp, _i64, _vp, _vp]),
     "lns_set_partition": (_i32, [_vp, _i32, _i32]),
     "lns_attach_comm": (_i32, [_vp, _vp, _i32, _i32]),
+    "lns_exchange_buffer": (_i32, [_vp, ctypes.POINTER(_vp)]),
+    "lns_exchange_ipc_handle": (_i32, [_vp, _vp]),
+    "lns_attach_peers": (_i32, [_vp, _i32, _i32, ctypes.POINTER(_vp), _i64]),
+    "lns_attach_peers_ipc": (_i32, [_vp, _i32, _i32, _vp, _i64]),
+    "lns_exchange_reset": (_i32, [_vp, _vp]),
     "lns_step_begin": (_i32, [_vp, _i32, _i64, _i64, _u64, _vp, _i32, _vp]),
     "lns_step_eval": (_i32, [_vp, _vp, _vp]),
     "lns_step_apply": (_i32, [_vp, _vp, _vp]),
@@ -190,6 +198,42 @@ def lns_set_partition(ctx: int, part: int, nparts: int) -> None:
 
 def lns_attach_comm(ctx: int, comm_ptr: Optional[int], rank: int, world: int) -> None:
     _check(load().lns_attach_comm(ctx, comm_ptr, rank, world), "lns_attach_comm")
+
+
+def lns_exchange_buffer(ctx: int) -> int:
+    """Device pointer of this context's 512-byte exchange buffer (device-initiated exchange)."""
+    p = _vp()
+    _check(load().lns_exchange_buffer(ctx, ctypes.byref(p)), "lns_exchange_buffer")
+    return int(p.value)
+
+
+def lns_exchange_ipc_handle(ctx: int) -> bytes:
+    """cudaIpcMemHandle_t (LNS_IPC_HANDLE_BYTES) of the exchange buffer, for other processes."""
+    buf = ctypes.create_string_buffer(LNS_IPC_HANDLE_BYTES)
+    _check(load().lns_exchange_ipc_handle(ctx, buf), "lns_exchange_ipc_handle")
+    return buf.raw
+
+
+def lns_attach_peers(ctx: int, part: int, nparts: int, bufs, timeout_ms: int = 10000) -> None:
+    """Partition `part` of `nparts` with the partitions' exchange buffers (device pointers usable
+    from this context's device); nparts = 1 / bufs = None detaches."""
+    arr = None
+    if bufs is not None:
+        arr = (_vp * len(bufs))(*[int(b) for b in bufs])
+    _check(load().lns_attach_peers(ctx, part, nparts, arr, timeout_ms), "lns_attach_peers")
+
+
+def lns_attach_peers_ipc(ctx: int, part: int, nparts: int, handles: bytes, timeout_ms: int = 10000) -> None:
+    """As lns_attach_peers from the concatenated IPC handles of all partitions (one process per GPU)."""
+    if len(handles) != nparts * LNS_IPC_HANDLE_BYTES:
+        raise ValueError("handles must hold nparts x LNS_IPC_HANDLE_BYTES bytes")
+    buf = ctypes.create_string_buffer(handles, len(handles))
+    _check(load().lns_attach_peers_ipc(ctx, part, nparts, buf, timeout_ms), "lns_attach_peers_ipc")
+
+
+def lns_exchange_reset(ctx: int, stream=None) -> None:
+    """Clear this context's exchange buffer (before every peer run, then a host barrier)."""
+    _check(load().lns_exchange_reset(ctx, _stream(stream)), "lns_exchange_reset")
 
 
 def lns_eval_neighborhood(ctx: int, k: int, V, Y, tabu_bits=None, stream=None) -> tuple[int, int]:

@@ -32,7 +32,10 @@
 #include <cmath>
 #include <cstdio>
 #include <cstring>
+#include <ctime>
 #include <string>
+#include <map>
+#include <mutex>
 #include <vector>
 
 #define LNS_VERSION_NUM 200
@@ -82,6 +85,8 @@ struct DevInst {
 
 // fstate layout (int64): current f, iterations done, best f, best iter, first zero iter, done, error
 enum { FS_F = 0, FS_T, FS_BEST, FS_BESTIT, FS_ZERO, FS_DONE, FS_ERR, FS_N };
+// FS_ERR: 1 = bad V0, 2 = no admissible move, 3 = peer exchange timed out
+#define MAX_PEERS 16
 
 struct SearchArgs {
     DevInst I;
@@ -110,6 +115,13 @@ struct SearchArgs {
     int64_t *slots;         // 3 x MAX_SLOTS parity-tagged keys (persistent) / accumulator (stepped)
     unsigned *counter;      // stepped: last-CTA counter
     int64_t *trace_r, *trace_f;
+    // device-initiated multi-GPU exchange (lns_attach_peers): npeers > 0 = every CTA of
+    // every partition meets in the exchange buffers peers[0..npeers), own buffer peers[part]
+    unsigned long long *const *peers;
+    int32_t npeers, part;
+    int64_t nb_total;       // CTAs over all partitions (the arrival count per exchange)
+    int64_t timeout_ns;     // a partition missing for this long ends the run (FS_ERR = 3)
+    int32_t plain_launch;   // LNS_PLAIN_LAUNCH: cudaLaunchKernel instead of the cooperative launch
 };
 
 // The CTA's X (sorted sign bits): shared memory, or its own slot of the global fallback buffer.
@@ -1095,6 +1107,10 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         ubase = blo;
     }
     const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
+    __shared__ unsigned long long *s_peers[MAX_PEERS];
+    __shared__ int s_xto;
+    if (threadIdx.x < A.npeers) s_peers[threadIdx.x] = A.peers[threadIdx.x];
+    if (threadIdx.x == 0) s_xto = 0;
     __syncthreads();
     const uint2 *tri = nullptr;
     if (A.tri_smem) {
@@ -1142,7 +1158,49 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             PH(4);
             unsigned long long key = ps.key;
             tg++;
-            if (nb > 1) {
+            if (A.npeers > 0) {
+                // cross-GPU exchange (lns_attach_peers): this CTA's MIN into slot tg%3 of every
+                // partition's buffer, then one arrival on every partition's counter (the release
+                // orders all the MINs before it); wait until the own counter shows every CTA of
+                // every partition, then the own slot holds the global minimum. CTA 0 resets its
+                // own slot (tg+2)%3: it was last read at exchange tg-1 by this partition's CTAs,
+                // all of which have arrived at tg, and is next written at tg+2 by CTAs that have
+                // seen this CTA's (later, releasing) arrival at tg+1.
+                if (threadIdx.x == 0) {
+                    const int s3 = (int)(tg % 3);
+                    if (key != (unsigned long long)KEY_NONE)
+                        for (int q = 0; q < A.npeers; q++)
+                            asm volatile("red.relaxed.sys.global.min.u64 [%0], %1;" ::"l"(s_peers[q] + 16 * s3), "l"(key)
+                                         : "memory");
+                    for (int q = 0; q < A.npeers; q++)
+                        asm volatile("red.release.sys.global.add.u64 [%0], 1;" ::"l"(s_peers[q] + 48) : "memory");
+                    unsigned long long *own = s_peers[A.part];
+                    const unsigned long long target = (unsigned long long)A.nb_total * tg;
+                    unsigned long long seen, t_start, t_now;
+                    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_start));
+                    bool late = false;
+                    for (;;) {
+                        asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(seen) : "l"(own + 48) : "memory");
+                        if (seen >= target) break;
+                        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
+                        if ((long long)(t_now - t_start) > A.timeout_ns) { late = true; break; }
+                    }
+                    if (late) {
+                        s_xto = 1;
+                        ps.gkey = (unsigned long long)KEY_NONE;
+                    } else {
+                        unsigned long long gk;
+                        asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(gk) : "l"(own + 16 * s3) : "memory");
+                        ps.gkey = gk;
+                        if (bid == 0)
+                            asm volatile("st.relaxed.sys.global.u64 [%0], %1;" ::"l"(own + 16 * ((tg + 2) % 3)),
+                                         "l"((unsigned long long)KEY_NONE) : "memory");
+                    }
+                }
+                __syncthreads();
+                key = ps.gkey;
+                if (s_xto) { failed = true; break; }
+            } else if (nb > 1) {
                 // exchange: u64 MIN of this CTA's key into slot tg%3 (each slot on its own 128-B
                 // line), then one arrival on the group's monotonic 64-bit counter; when it reaches
                 // nb * tg every CTA's MIN has landed and the slot holds the group minimum. Slot
@@ -1207,7 +1265,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                 if (threadIdx.x == 0) {
                     A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
                     A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
-                    if (failed) A.fs[FS_ERR] = 2;
+                    if (failed) A.fs[FS_ERR] = s_xto ? 3 : 2;
                 }
             }
         }
@@ -1380,6 +1438,12 @@ struct lns_ctx {
     nccl_allreduce_fn nccl_allreduce = nullptr;
     int blocks_override = 0;
     int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
+    // device-initiated exchange (lns_attach_peers)
+    unsigned long long *d_xbuf = nullptr;            // own 64-word exchange buffer (its own allocation)
+    unsigned long long **d_peers = nullptr;          // device array of the partitions' buffers
+    int npeers = 0;
+    int64_t peer_timeout_ms = 0;
+    std::vector<void *> ipc_opened;                   // peer buffers opened by lns_attach_peers_ipc
     // run state
     uint32_t *d_vb = nullptr;
     int32_t *d_Y = nullptr;
@@ -1543,6 +1607,8 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
+    A.peers = nullptr; A.npeers = 0; A.part = 0; A.nb_total = 0; A.timeout_ns = 0;
+    A.plain_launch = (flags & LNS_PLAIN_LAUNCH) ? 1 : 0;
     return A;
 }
 
@@ -1579,6 +1645,7 @@ lns_status search_finish(lns_ctx *c, int8_t *V_out, int64_t *trace_rank, int64_t
     CK(cudaStreamSynchronize(st));
     if (fs[FS_ERR] == 1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
     if (fs[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
+    if (fs[FS_ERR] == 3) return fail(LNS_EPEER, "a partition did not reach the exchange in time");
     const int64_t done = fs[FS_T];
     if (trace_rank && done > 0) CK(cudaMemcpyAsync(trace_rank, c->d_tr, done * 8, cudaMemcpyDefault, st));
     if (trace_fit && done > 0) CK(cudaMemcpyAsync(trace_fit, c->d_tf, done * 8, cudaMemcpyDefault, st));
@@ -1615,6 +1682,23 @@ size_t cache_geometry(SearchArgs &A, const Geometry &g, int nb, int budget)
     return smem;
 }
 
+// Raise a kernel's dynamic shared-memory limit once per (kernel, device): cudaFuncSetAttribute on a
+// kernel that is running (another context's search on another stream) waits for it, which would
+// serialise concurrent searches of one process.
+cudaError_t allow_smem(const void *fn, int bytes)
+{
+    static std::mutex mu;
+    static std::map<std::pair<const void *, int>, int> done;
+    int dev = 0;
+    cudaGetDevice(&dev);
+    std::lock_guard<std::mutex> lk(mu);
+    int &have = done[{fn, dev}];
+    if (have >= bytes) return cudaSuccess;
+    const cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes);
+    if (e == cudaSuccess) have = bytes;
+    return e;
+}
+
 // Padded placement pays off when a CTA evaluates many neighbours per plan (it adds a serial warp
 // pass to every plan build): the same slice test as the contiguous-run evaluation path.
 inline int pad_for(const Geometry &g, uint32_t span, int nb)
@@ -1623,23 +1707,25 @@ inline int pad_for(const Geometry &g, uint32_t span, int nb)
 }
 
 template <int K>
-lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st)
+lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st, int nb_force = 0)
 {
     // persistent geometry: first the CTA count at the eval footprint, then cache the until[]
     // slice in shared memory if it fits next to it
     const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
-    CK(cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, budget));
+    CK(allow_smem((const void *)k_search<K>, budget));
     int occ = 0;
     CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
-    const int nb = search_blocks(c, A.hi - A.lo, 1);
+    const int nb = nb_force > 0 ? nb_force : search_blocks(c, A.hi - A.lo, 1);
+    if (A.npeers > 0) A.nb_total = (int64_t)nb * A.npeers;
     A.I.pad = pad_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
     k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
-    CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
+    if (A.plain_launch) CK(cudaLaunchKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
+    else CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     return LNS_OK;
 }
@@ -1649,7 +1735,7 @@ template <int K>
 lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int G, int nb, int64_t *gslots, cudaStream_t st)
 {
     const int budget = c->smemOptin - 1024;
-    CK(cudaFuncSetAttribute(k_search<K>, cudaFuncAttributeMaxDynamicSharedMemorySize, budget));
+    CK(allow_smem((const void *)k_search<K>, budget));
     A.I.pad = pad_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
     if (!A.until_smem) {  // one global until[] per concurrent group
@@ -1671,8 +1757,9 @@ template <int K>
 lns_status launch_step_eval(lns_ctx *c, const SearchArgs &A, const Geometry &g, int64_t *key_out, int32_t *fit_out,
                             bool all, cudaStream_t st)
 {
-    CK(cudaFuncSetAttribute(k_step_eval<K, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)g.smem_eval));
-    CK(cudaFuncSetAttribute(k_step_eval<K, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)g.smem_eval));
+    const int budget = c->smemOptin - 1024;
+    CK(allow_smem((const void *)k_step_eval<K, false>, budget));
+    CK(allow_smem((const void *)k_step_eval<K, true>, budget));
     int occ = 0;
     CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_step_eval<K, false>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "eval kernel does not fit on an SM");
@@ -1700,12 +1787,12 @@ lns_status launch_step_apply(const SearchArgs &A, const int64_t *key, cudaStream
     return LNS_OK;
 }
 
-lns_status dispatch_search(lns_ctx *c, int k, const SearchArgs &A, const Geometry &g, cudaStream_t st)
+lns_status dispatch_search(lns_ctx *c, int k, const SearchArgs &A, const Geometry &g, cudaStream_t st, int nb_force = 0)
 {
     switch (k) {
-    case 1: return launch_search<1>(c, A, g, st);
-    case 2: return launch_search<2>(c, A, g, st);
-    default: return launch_search<3>(c, A, g, st);
+    case 1: return launch_search<1>(c, A, g, st, nb_force);
+    case 2: return launch_search<2>(c, A, g, st, nb_force);
+    default: return launch_search<3>(c, A, g, st, nb_force);
     }
 }
 lns_status dispatch_step_eval(lns_ctx *c, int k, const SearchArgs &A, const Geometry &g, int64_t *key_out,
@@ -1750,6 +1837,7 @@ const char *lns_strerror(lns_status s)
     case LNS_ECUDA: return "CUDA error";
     case LNS_ENCCL: return "NCCL error";
     case LNS_ENOADMISSIBLE: return "no admissible neighbour";
+    case LNS_EPEER: return "peer exchange timed out";
     default: return "unknown status";
     }
 }
@@ -1825,6 +1913,8 @@ void lns_destroy(lns_ctx *c)
     cudaFree(c->d_slots); cudaFree(c->d_counter); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_bits);
     cudaFree(c->d_until); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
     cudaFree(c->d_V0s); cudaFree(c->d_res); cudaFree(c->d_vouts); cudaFree(c->d_gslots); cudaFree(c->d_X);
+    for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
+    cudaFree(c->d_xbuf); cudaFree(c->d_peers);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
     delete c;
@@ -1842,7 +1932,7 @@ double lns_last_kernel_ms(lns_ctx *c) { return c ? c->last_ms : 0.0; }
 lns_status lns_set_partition(lns_ctx *c, int32_t part, int32_t nparts)
 {
     if (!c || nparts < 1 || part < 0 || part >= nparts) return fail(LNS_EINVAL, "bad partition");
-    c->part = part; c->nparts = nparts;
+    c->part = part; c->nparts = nparts; c->npeers = 0;
     return LNS_OK;
 }
 
@@ -1857,8 +1947,94 @@ lns_status lns_attach_comm(lns_ctx *c, void *comm, int32_t rank, int32_t world)
     if (!sym) return fail(LNS_ENCCL, "ncclAllReduce not found (load torch's libnccl first)");
     c->nccl_allreduce = (nccl_allreduce_fn)sym;
     c->comm = comm;
-    c->part = rank; c->nparts = world;
+    c->part = rank; c->nparts = world; c->npeers = 0;
     return LNS_OK;
+}
+
+lns_status lns_exchange_buffer(lns_ctx *c, void **buf_dev)
+{
+    if (!c || !buf_dev) return fail(LNS_EINVAL, "null argument");
+    DeviceGuard dg(c->device);
+    if (!c->d_xbuf) {
+        if (cudaMalloc(&c->d_xbuf, 64 * sizeof(unsigned long long)) != cudaSuccess) {
+            cudaGetLastError();
+            return fail(LNS_ENOMEM, "exchange buffer");
+        }
+        lns_status s = lns_exchange_reset(c, nullptr);
+        if (s != LNS_OK) return s;
+    }
+    *buf_dev = c->d_xbuf;
+    return LNS_OK;
+}
+
+lns_status lns_exchange_ipc_handle(lns_ctx *c, void *handle_out)
+{
+    if (!c || !handle_out) return fail(LNS_EINVAL, "null argument");
+    static_assert(sizeof(cudaIpcMemHandle_t) == LNS_IPC_HANDLE_BYTES, "IPC handle size");
+    void *buf = nullptr;
+    lns_status s = lns_exchange_buffer(c, &buf);
+    if (s != LNS_OK) return s;
+    DeviceGuard dg(c->device);
+    cudaIpcMemHandle_t h;
+    CK(cudaIpcGetMemHandle(&h, buf));
+    memcpy(handle_out, &h, sizeof(h));
+    return LNS_OK;
+}
+
+lns_status lns_exchange_reset(lns_ctx *c, void *stream)
+{
+    if (!c || !c->d_xbuf) return fail(LNS_EINVAL, "no exchange buffer (lns_exchange_buffer first)");
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    k_init_slots<<<1, 64, 0, st>>>((int64_t *)c->d_xbuf, 1);
+    CK(cudaGetLastError());
+    CK(cudaStreamSynchronize(st));
+    return LNS_OK;
+}
+
+lns_status lns_attach_peers(lns_ctx *c, int32_t part, int32_t nparts, void *const *bufs, int64_t timeout_ms)
+{
+    if (!c) return fail(LNS_EINVAL, "null context");
+    DeviceGuard dg(c->device);
+    if (nparts <= 1 || !bufs) { c->npeers = 0; c->part = 0; c->nparts = 1; return LNS_OK; }
+    if (part < 0 || part >= nparts || nparts > MAX_PEERS) return fail(LNS_EINVAL, "bad partition (at most 16)");
+    if (timeout_ms <= 0) return fail(LNS_EINVAL, "timeout_ms must be positive");
+    void *own = nullptr;
+    lns_status s = lns_exchange_buffer(c, &own);
+    if (s != LNS_OK) return s;
+    if (bufs[part] != own) return fail(LNS_EINVAL, "bufs[part] must be this context's exchange buffer");
+    for (int q = 0; q < nparts; q++)
+        if (!bufs[q]) return fail(LNS_EINVAL, "null peer buffer");
+    if (!c->d_peers && cudaMalloc(&c->d_peers, MAX_PEERS * sizeof(void *)) != cudaSuccess) {
+        cudaGetLastError();
+        return fail(LNS_ENOMEM, "peer table");
+    }
+    CK(cudaMemcpy(c->d_peers, bufs, nparts * sizeof(void *), cudaMemcpyHostToDevice));
+    c->npeers = nparts; c->part = part; c->nparts = nparts; c->comm = nullptr;
+    c->peer_timeout_ms = timeout_ms;
+    return LNS_OK;
+}
+
+lns_status lns_attach_peers_ipc(lns_ctx *c, int32_t part, int32_t nparts, const void *handles, int64_t timeout_ms)
+{
+    if (!c || !handles || nparts < 1 || part < 0 || part >= nparts || nparts > MAX_PEERS)
+        return fail(LNS_EINVAL, "bad partition / handles");
+    DeviceGuard dg(c->device);
+    for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
+    c->ipc_opened.clear();
+    std::vector<void *> bufs(nparts, nullptr);
+    lns_status s = lns_exchange_buffer(c, &bufs[part]);
+    if (s != LNS_OK) return s;
+    for (int q = 0; q < nparts; q++) {
+        if (q == part) continue;
+        cudaIpcMemHandle_t h;
+        memcpy(&h, (const char *)handles + (size_t)q * LNS_IPC_HANDLE_BYTES, sizeof(h));
+        void *p = nullptr;
+        CK(cudaIpcOpenMemHandle(&p, h, cudaIpcMemLazyEnablePeerAccess));
+        c->ipc_opened.push_back(p);
+        bufs[q] = p;
+    }
+    return lns_attach_peers(c, part, nparts, bufs.data(), timeout_ms);
 }
 
 lns_status lns_eval_neighborhood(lns_ctx *c, int32_t k, const int8_t *V, const int32_t *Y, const uint32_t *tabu_bits,
@@ -1989,11 +2165,19 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     cudaStream_t st = (cudaStream_t)stream;
     if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
     SearchArgs A = make_args(c, g, iters, L, flags);
-    const bool stepped = c->comm != nullptr || c->nparts > 1 || (flags & LNS_FORCE_STEPPED);
-    if (!stepped) {
+    if (c->npeers > 0) {
+        // device-initiated exchange: one persistent kernel per partition, meeting in the peers'
+        // exchange buffers every iteration; every partition uses the same CTA count
+        A.peers = c->d_peers; A.npeers = c->npeers; A.part = c->part;
+        A.timeout_ns = c->peer_timeout_ms * 1000000LL;
+        const uint32_t span = (uint32_t)((g.M + (uint64_t)c->nparts - 1) / (uint64_t)c->nparts);
+        const int nb = search_blocks(c, span, 1);
+        if (iters > 0 && (s = dispatch_search(c, k, A, g, st, nb)) != LNS_OK) return s;
+    } else if (!(c->comm != nullptr || c->nparts > 1 || (flags & LNS_FORCE_STEPPED))) {
         if (iters > 0 && (s = dispatch_search(c, k, A, g, st)) != LNS_OK) return s;
     } else {
-        if (c->nparts > 1 && !c->comm) return fail(LNS_EINVAL, "partitioned run needs a communicator (or use the stepped API)");
+        if (c->nparts > 1 && !c->comm)
+            return fail(LNS_EINVAL, "partitioned run needs a communicator or attached peers (or use the stepped API)");
         int64_t *kb = c->d_slots + SLOT_OUT;
         CK(cudaEventRecord(c->ev0, st));
         for (int64_t t = 0; t < iters; t++) {

@@ -12,6 +12,11 @@ Two ways to use several GPUs, both from SURVEY.md §8(e) / DESIGN.md §8:
   ``Stepper`` and any torch.distributed backend (it is what the gloo tests exercise).
 * **Independent restarts**: restart r runs on rank r mod world (``restart_shard``); no data-path
   collective, only a final gather of the per-restart results (``sharded_restarts``).
+* **Device-initiated exchange** (``peer_tabu_run``): the partitioned search
+  with the per-iteration MIN done by the persistent kernels themselves -- every CTA MINs its key
+  into every GPU's exchange buffer over NVLink peer memory and waits on its own arrival counter --
+  so there is no host collective and no per-iteration launch. Buffers are shared once per run as
+  CUDA IPC handles (``gather_exchange_handles``).
 
 Nothing here computes on the CPU: the GPU ``LnsStepper`` drives the kernels of liblns.so.
 """
@@ -135,3 +140,40 @@ def sharded_restarts(run_one: Callable[[int], dict], R: int, group=None) -> list
     for p in parts:
         merged.update(p)
     return [merged[r] for r in range(R)]
+
+
+# ------------------------------------------------------------------ device-initiated exchange (f3)
+def gather_exchange_handles(handle: bytes, group=None) -> bytes:
+    """Every rank's exchange-buffer IPC handle, concatenated in rank order (what
+    lns_attach_peers_ipc takes). Pure host logic: works over gloo or NCCL process groups."""
+    world = dist.get_world_size(group) if dist.is_initialized() else 1
+    if world == 1:
+        return bytes(handle)
+    got = [None] * world
+    dist.all_gather_object(got, bytes(handle), group=group)
+    if any(len(h) != len(handle) for h in got):
+        raise ValueError("exchange handles differ in size across ranks")
+    return b"".join(got)
+
+
+def peer_tabu_run(ctx: int, k: int, iters: int, tenure: int = -1, seed: int = 0, V0=None, flags: int = 0,
+                  group=None, timeout_ms: int = 10000, V_out=None, trace_rank=None, trace_fit=None, stream=None):
+    """One search over all ranks of `group`, one process per GPU, with the per-iteration argmin
+    exchanged by the persistent kernels themselves through NVLink peer memory (lns_attach_peers_ipc;
+    SURVEY.md §8(f) f3) instead of a host all-reduce. Rank r evaluates slice r of the rank space;
+    the trajectory equals the single-GPU one. Returns this rank's lns_tabu_run result dict (outputs
+    as in lns_tabu_run)."""
+    from . import (lns_attach_peers, lns_attach_peers_ipc, lns_exchange_ipc_handle, lns_exchange_reset,
+                   lns_tabu_run)
+    rank = dist.get_rank(group) if dist.is_initialized() else 0
+    world = dist.get_world_size(group) if dist.is_initialized() else 1
+    if world > 1:
+        handles = gather_exchange_handles(lns_exchange_ipc_handle(ctx), group)
+        lns_attach_peers_ipc(ctx, rank, world, handles, timeout_ms)
+        lns_exchange_reset(ctx, stream)
+        dist.barrier(group)  # every partition's buffer is clear before any kernel starts
+    try:
+        return lns_tabu_run(ctx, k, iters, tenure, seed, V0, flags, V_out, trace_rank, trace_fit, stream)
+    finally:
+        if world > 1:
+            lns_attach_peers(ctx, 0, 1, None)

@@ -413,3 +413,89 @@ def test_eval_all_large_slices(L, orc, m, n, k):
             assert np.array_equal(got.astype(np.int64), want)
     finally:
         L.lns_destroy(ctx)
+
+
+# ------------------------------------------------------------------ device-initiated exchange (f3)
+def _peer_pair(L, inst, nb):
+    ctxs = [L.lns_create(inst.A, inst.S) for _ in range(2)]
+    for c in ctxs:
+        L.lns_config(c, nb)
+    bufs = [L.lns_exchange_buffer(c) for c in ctxs]
+    return ctxs, bufs
+
+
+@pytest.mark.parametrize("cfg,iters", [("C4", 120), ("C3", 300), ("C2", 400)])
+def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters):
+    """two partitions, each a persistent kernel of 32 CTAs on its own stream,
+    exchange the per-iteration MIN through each other's exchange buffers (red.min.sys /
+    red.release.sys / ld.acquire.sys) with no host step. Both must reproduce the single-context
+    trajectory bit for bit (same device here, so plain launches: the driver serialises cooperative
+    ones; across GPUs the buffers are NVLink peer memory and each GPU runs one cooperative kernel)."""
+    import threading
+
+    import torch
+
+    c = pi.CONFIGS[cfg]
+    inst = pi.config_instance(cfg)
+    k, n = c["k"], inst.n
+    V0 = pi.start_vector(n, pi.config_seed(cfg))
+    ref = L.lns_create(inst.A, inst.S)
+    try:
+        tr0, tf0 = np.zeros(iters, np.int64), np.zeros(iters, np.int64)
+        v0 = np.zeros(n, np.int8)
+        r0 = L.lns_tabu_run(ref, k, iters, -1, 0, V0, 0, v0, tr0, tf0)
+    finally:
+        L.lns_destroy(ref)
+    ctxs, bufs = _peer_pair(L, inst, 32)
+    try:
+        # a plain run first: every buffer the run needs is allocated now (cudaMalloc synchronises
+        # the device, which would serialise the two partitions' kernels in one process)
+        for cx in ctxs:
+            L.lns_tabu_run(cx, k, iters, -1, 0, V0, 0)
+        for p, cx in enumerate(ctxs):
+            L.lns_attach_peers(cx, p, 2, bufs, 20000)
+        for cx in ctxs:
+            L.lns_exchange_reset(cx)
+        outs = [dict(tr=np.zeros(iters, np.int64), tf=np.zeros(iters, np.int64), v=np.zeros(n, np.int8))
+                for _ in ctxs]
+        errs = [None, None]
+        streams = [torch.cuda.Stream() for _ in ctxs]
+
+        def run(p):
+            try:
+                o = outs[p]
+                o["res"] = L.lns_tabu_run(ctxs[p], k, iters, -1, 0, V0, L.LNS_PLAIN_LAUNCH, o["v"], o["tr"], o["tf"],
+                                          streams[p])
+            except Exception as e:  # noqa: BLE001 - reported below
+                errs[p] = e
+
+        th = [threading.Thread(target=run, args=(p,)) for p in range(2)]
+        for t in th:
+            t.start()
+        for t in th:
+            t.join()
+        assert errs == [None, None], errs
+        for o in outs:
+            assert np.array_equal(o["tr"], tr0) and np.array_equal(o["tf"], tf0)
+            assert np.array_equal(o["v"], v0) and o["res"] == r0
+    finally:
+        for cx in ctxs:
+            L.lns_destroy(cx)
+
+
+def test_peer_exchange_missing_partition_times_out(L):
+    """A partition that never arrives ends the run with LNS_EPEER after the timeout (no hang)."""
+    inst = pi.config_instance("C3")
+    ctxs, bufs = _peer_pair(L, inst, 16)
+    try:
+        L.lns_attach_peers(ctxs[0], 0, 2, bufs, 300)
+        L.lns_exchange_reset(ctxs[0])
+        with pytest.raises(L.LnsError) as ei:
+            L.lns_tabu_run(ctxs[0], 3, 50, -1, 0, pi.start_vector(inst.n, 4), 0)
+        assert ei.value.status == L.LNS_EPEER
+        L.lns_attach_peers(ctxs[0], 0, 1, None)  # detached: a plain run works again
+        res = L.lns_tabu_run(ctxs[0], 3, 5, -1, 0, pi.start_vector(inst.n, 4), 0)
+        assert res["iters_done"] == 5
+    finally:
+        for cx in ctxs:
+            L.lns_destroy(cx)

@@ -94,7 +94,7 @@ def _worker(rank, world, port, cfg, out):
                                     cfg["stop"])
             tr, tf, V, f = par.partitioned_tabu_run(st, cfg["iters"], check_every=1)
             out[rank] = (tr.tolist(), tf.tolist(), V.tolist(), f)
-        else:
+        elif cfg["kind"] == "restarts":
             import oracle
 
             inst = pi.planted_instance(cfg["m"], cfg["n"], cfg["seed"])
@@ -107,6 +107,10 @@ def _worker(rank, world, port, cfg, out):
                 return res
 
             out[rank] = par.sharded_restarts(run_one, cfg["R"])
+        if cfg["kind"] == "handles":
+            # each rank's (fake) 64-byte IPC handle; every rank must get all, in rank order
+            mine = bytes([rank + 1]) * 64
+            out[rank] = par.gather_exchange_handles(mine)
     finally:
         dist.destroy_process_group()
 
@@ -168,3 +172,13 @@ def test_sharded_restarts_gloo(orc):
             V0 = pi.start_vector(21, pi.restart_seed(9, r))
             _, _, _, res = orc.tabu_run(inst.A, inst.S, 1, V0, 300, 3)
             assert {key: g[key] for key in res} == res
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_gather_exchange_handles_gloo(world):
+    """Host side of the device-initiated exchange (f3): the partitions' exchange-buffer IPC handles
+    are gathered in rank order, which is what lns_attach_peers_ipc indexes by partition."""
+    out = _spawn(world, dict(kind="handles"))
+    want = b"".join(bytes([r + 1]) * 64 for r in range(world))
+    for rank in range(world):
+        assert out[rank] == want
