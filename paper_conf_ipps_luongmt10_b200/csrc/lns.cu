@@ -1159,43 +1159,79 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             unsigned long long key = ps.key;
             tg++;
             if (A.npeers > 0) {
-                // cross-GPU exchange (lns_attach_peers): this CTA's MIN into slot tg%3 of every
-                // partition's buffer, then one arrival on every partition's counter (the release
-                // orders all the MINs before it); wait until the own counter shows every CTA of
-                // every partition, then the own slot holds the global minimum. CTA 0 resets its
-                // own slot (tg+2)%3: it was last read at exchange tg-1 by this partition's CTAs,
-                // all of which have arrived at tg, and is next written at tg+2 by CTAs that have
-                // seen this CTA's (later, releasing) arrival at tg+1.
+                // cross-GPU exchange (lns_attach_peers), two levels:
+                //  1. inside the partition as below (.gpu scope): MIN into the local slot tg%3, one
+                //     arrival on the local counter;
+                //  2. CTA 0 waits for the local arrivals, MINs the partition's key into slot tg%3 of
+                //     EVERY partition's exchange buffer and arrives on every partition's counter
+                //     (.sys scope, NVLink peer memory), waits until its own counter shows all
+                //     partitions, and reads its own slot: the global minimum;
+                //  3. CTA 0 writes that key into the local slot and releases the local flag = tg;
+                //     the other CTAs wait for the flag and read the slot.
+                // Local slot (tg+2)%3 is reset by CTA 0 after the local arrivals at tg (its readers
+                // read it at tg-1, before arriving at tg); its next writers pass the flag of tg+1,
+                // which CTA 0 releases after the reset. The same holds per exchange buffer.
                 if (threadIdx.x == 0) {
                     const int s3 = (int)(tg % 3);
+                    unsigned long long *slot = gslots + 16 * s3;
+                    unsigned long long *ctr = gslots + 48, *flag = gslots + 56;
                     if (key != (unsigned long long)KEY_NONE)
-                        for (int q = 0; q < A.npeers; q++)
-                            asm volatile("red.relaxed.sys.global.min.u64 [%0], %1;" ::"l"(s_peers[q] + 16 * s3), "l"(key)
-                                         : "memory");
-                    for (int q = 0; q < A.npeers; q++)
-                        asm volatile("red.release.sys.global.add.u64 [%0], 1;" ::"l"(s_peers[q] + 48) : "memory");
-                    unsigned long long *own = s_peers[A.part];
-                    const unsigned long long target = (unsigned long long)A.nb_total * tg;
-                    unsigned long long seen, t_start, t_now;
+                        asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
+                    asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
+                    unsigned long long t_start, t_now, seen;
                     asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_start));
                     bool late = false;
-                    for (;;) {
-                        asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(seen) : "l"(own + 48) : "memory");
-                        if (seen >= target) break;
-                        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
-                        if ((long long)(t_now - t_start) > A.timeout_ns) { late = true; break; }
-                    }
-                    if (late) {
-                        s_xto = 1;
-                        ps.gkey = (unsigned long long)KEY_NONE;
-                    } else {
-                        unsigned long long gk;
-                        asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(gk) : "l"(own + 16 * s3) : "memory");
-                        ps.gkey = gk;
-                        if (bid == 0)
-                            asm volatile("st.relaxed.sys.global.u64 [%0], %1;" ::"l"(own + 16 * ((tg + 2) % 3)),
+                    if (bid == 0) {
+                        const unsigned long long local_target = (unsigned long long)nb * tg;
+                        for (;;) {
+                            asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+                            if (seen >= local_target) break;
+                            asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
+                            if ((long long)(t_now - t_start) > A.timeout_ns) { late = true; break; }
+                        }
+                        if (!late) {
+                            unsigned long long lk;
+                            asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(lk) : "l"(slot) : "memory");
+                            asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(gslots + 16 * ((tg + 2) % 3)),
                                          "l"((unsigned long long)KEY_NONE) : "memory");
+                            if (lk != (unsigned long long)KEY_NONE)
+                                for (int q = 0; q < A.npeers; q++)
+                                    asm volatile("red.relaxed.sys.global.min.u64 [%0], %1;" ::"l"(s_peers[q] + 16 * s3),
+                                                 "l"(lk) : "memory");
+                            for (int q = 0; q < A.npeers; q++)
+                                asm volatile("red.release.sys.global.add.u64 [%0], 1;" ::"l"(s_peers[q] + 48) : "memory");
+                            unsigned long long *own = s_peers[A.part];
+                            const unsigned long long target = (unsigned long long)A.npeers * tg;
+                            for (;;) {
+                                asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(seen) : "l"(own + 48) : "memory");
+                                if (seen >= target) break;
+                                asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
+                                if ((long long)(t_now - t_start) > A.timeout_ns) { late = true; break; }
+                            }
+                            if (!late) {
+                                unsigned long long gk;
+                                asm volatile("ld.relaxed.sys.global.u64 %0, [%1];" : "=l"(gk) : "l"(own + 16 * s3) : "memory");
+                                asm volatile("st.relaxed.sys.global.u64 [%0], %1;" ::"l"(own + 16 * ((tg + 2) % 3)),
+                                             "l"((unsigned long long)KEY_NONE) : "memory");
+                                ps.gkey = gk;
+                                asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(slot), "l"(gk) : "memory");
+                                asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(flag), "l"(tg) : "memory");
+                            }
+                        }
+                    } else {
+                        for (;;) {
+                            asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(flag) : "memory");
+                            if (seen >= tg) break;
+                            asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
+                            if ((long long)(t_now - t_start) > A.timeout_ns) { late = true; break; }
+                        }
+                        if (!late) {
+                            unsigned long long gk;
+                            asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
+                            ps.gkey = gk;
+                        }
                     }
+                    if (late) { s_xto = 1; ps.gkey = (unsigned long long)KEY_NONE; }
                 }
                 __syncthreads();
                 key = ps.gkey;
