@@ -360,16 +360,24 @@ def main():
         except (OSError, ValueError):
             traffic = None
     nbr_per_s_kernel = (my_iters / args.steps) * M / kern_avg_s if kern_avg_s > 0 else 0.0
+    # "the 'fraction of integer-pipe peak' uses achieved issued int instructions /
+    # peak, and the model figure is reported beside it, not instead of it" -- the bit-sliced kernel
+    # issues fewer instructions than the m(k+4) model counts, so the model figure can exceed 1
+    model = {"ops_per_neighbor": ops_per_nbr, "achieved": achieved, "frac": achieved / peak,
+             "note": "SURVEY.md §8(d) model: m(k+4) integer ops per neighbour (k sign reads, Y' add, "
+                     "penalty, 2 histogram moves per row); a bit-sliced kernel needs fewer, so frac > 1 is possible"}
     roofline = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tops/s", "frac": achieved / peak,
                 "traffic": traffic, "kernel": "k_search<3> (persistent, batched searches)",
                 "peak_source": f"{sms} SMs x 128 int lanes/clk x {mhz:.0f} MHz ({src} sm_max_mhz)",
-                "ops_per_neighbor": ops_per_nbr,
-                "ops_model": "SURVEY.md §8(d): m(k+4) integer ops per neighbour; the bit-sliced kernel issues fewer"}
+                "achieved_is": "model ops (no ncu capture found)", "model": model}
     if per_nbr:
         # what the kernel actually issues (ncu source page of the committed capture, same kernel and job)
         ipn, ppn = per_nbr["issued_instructions"], per_nbr["popc"]
-        roofline["issued"] = {"instructions_per_neighbor": ipn, "achieved": nbr_per_s_kernel * ipn / 1e12,
-                              "frac": nbr_per_s_kernel * ipn / 1e12 / peak}
+        issued = nbr_per_s_kernel * ipn / 1e12
+        roofline.update({"achieved": issued, "frac": issued / peak,
+                         "achieved_is": "issued thread-instructions/s = live neighbours/s x issued instructions "
+                                        "per neighbour (ncu source page of the committed capture)",
+                         "instructions_per_neighbor": ipn})
         # the pipe that binds the piece loop: POPC on XU at 1/8 of the issue rate (16 lanes/clk/SM)
         xu_ceiling = sms * 16 * mhz * 1e6 / ppn
         roofline["binding_pipe"] = {"pipe": "xu (POPC, 16 lanes/clk/SM)", "popc_per_neighbor": ppn,

@@ -210,6 +210,19 @@ const char *lns_strerror(lns_status status);
 const char *lns_last_error(void);
 int32_t lns_version(void); /* major*10000 + minor*100 + patch */
 
+/* Device-memory cache of the library (a runtime component, not a passage of the paper).
+ * Context buffers (lns_create, the per-run until[] / trace / restart arrays) come from a per-device
+ * caching allocator: lns_destroy returns them to a cache keyed by (device, power-of-two size
+ * class) instead of cudaFree, so create -> run -> destroy cycles do not pay cudaMalloc / cudaFree
+ * (which synchronises the device). The cache holds at most LNS_POOL_CAP_MB (environment, read once,
+ * default 4096) MiB; beyond that blocks are freed. An allocation that fails retries once after
+ * releasing the cache.
+ * lns_pool_trim -- cudaFree every cached (unused) block on every device. Thread-safe; never fails.
+ * lns_pool_stats -- bytes currently cached (unused) and handed out (in use by live contexts);
+ *                   either pointer may be NULL. */
+void lns_pool_trim(void);
+void lns_pool_stats(int64_t *cached_bytes, int64_t *live_bytes);
+
 #ifdef __cplusplus
 }
 #endif

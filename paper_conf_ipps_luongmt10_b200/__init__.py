@@ -79,6 +79,8 @@ _SIGS = {
     "lns_strerror": (ctypes.c_char_p, [_i32]),
     "lns_last_error": (ctypes.c_char_p, []),
     "lns_version": (_i32, []),
+    "lns_pool_trim": (None, []),
+    "lns_pool_stats": (None, [ctypes.POINTER(_i64), ctypes.POINTER(_i64)]),
 }
 
 
@@ -159,6 +161,18 @@ def _stream(stream) -> Optional[int]:
 # --------------------------------------------------------------------------- C ABI, same names
 def lns_version() -> int:
     return int(load().lns_version())
+
+
+def lns_pool_trim() -> None:
+    """Release the library's cached device blocks (include/lns.h, device-memory cache)."""
+    load().lns_pool_trim()
+
+
+def lns_pool_stats() -> tuple[int, int]:
+    """(cached bytes, live bytes) of the library's device-memory cache."""
+    c, l_ = _i64(0), _i64(0)
+    load().lns_pool_stats(ctypes.byref(c), ctypes.byref(l_))
+    return int(c.value), int(l_.value)
 
 
 def lns_strerror(status: int) -> str:

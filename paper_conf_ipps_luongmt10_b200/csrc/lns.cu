@@ -1534,13 +1534,99 @@ int64_t comb_k(int64_t n, int k)
 
 DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->W, 0, c->d_Arow, c->d_H, c->maxS}; }
 
+// Per-device caching allocator for context buffers (lns_pool_*). cudaMalloc / cudaFree cost tens
+// of microseconds to milliseconds each and cudaFree synchronises the device, so a user who creates a
+// context per instance (the e2e path: lns_create -> run -> lns_destroy) would pay them on every
+// call. Freed blocks are kept per (device, power-of-two size class) and handed to the next request
+// of that class; the cache is bounded (LNS_POOL_CAP_MB, default 4096) and lns_pool_trim() returns
+// it to the driver. Every public call that launches work synchronises its stream before it
+// returns, so a block is never recycled while a kernel still uses it (lns_destroy synchronises the
+// device first when a stepped search is still open).
+struct Pool {
+    std::mutex mu;
+    std::multimap<std::pair<int, size_t>, void *> cache;   // (device, class) -> free block
+    std::map<void *, std::pair<int, size_t>> live;          // block -> (device, class)
+    size_t cached = 0, live_bytes = 0, cap = 0;
+};
+Pool &pool()
+{
+    static Pool *p = [] {
+        Pool *q = new Pool();  // never destroyed: no dependence on static teardown order
+        const char *e = getenv("LNS_POOL_CAP_MB");
+        q->cap = (size_t)(e ? atol(e) : 4096) << 20;
+        return q;
+    }();
+    return *p;
+}
+size_t size_class(size_t b)
+{
+    size_t c = 256;
+    while (c < b) c <<= 1;
+    return c;
+}
+cudaError_t pool_alloc(void **out, size_t bytes)
+{
+    int dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return e;
+    const size_t cls = size_class(bytes);
+    Pool &P = pool();
+    {
+        std::lock_guard<std::mutex> lk(P.mu);
+        auto it = P.cache.find({dev, cls});
+        if (it != P.cache.end()) {
+            *out = it->second;
+            P.cache.erase(it);
+            P.cached -= cls;
+            P.live[*out] = {dev, cls};
+            P.live_bytes += cls;
+            return cudaSuccess;
+        }
+    }
+    e = cudaMalloc(out, cls);
+    if (e != cudaSuccess) {
+        cudaGetLastError();
+        lns_pool_trim();  // retry once with the cache released
+        e = cudaMalloc(out, cls);
+        if (e != cudaSuccess) { cudaGetLastError(); *out = nullptr; return e; }
+    }
+    std::lock_guard<std::mutex> lk(P.mu);
+    P.live[*out] = {dev, cls};
+    P.live_bytes += cls;
+    return cudaSuccess;
+}
+template <typename T>
+cudaError_t pool_alloc(T **out, size_t bytes) { return pool_alloc((void **)out, bytes); }
+void pool_free(void *p)
+{
+    if (!p) return;
+    Pool &P = pool();
+    std::unique_lock<std::mutex> lk(P.mu);
+    auto it = P.live.find(p);
+    if (it == P.live.end()) return;  // not ours (never happens)
+    const auto key = it->second;
+    P.live.erase(it);
+    P.live_bytes -= key.second;
+    if (P.cached + key.second <= P.cap) {
+        P.cache.insert({key, p});
+        P.cached += key.second;
+        return;
+    }
+    lk.unlock();
+    int cur = 0;
+    cudaGetDevice(&cur);
+    if (cur != key.first) cudaSetDevice(key.first);
+    cudaFree(p);
+    if (cur != key.first) cudaSetDevice(cur);
+}
+
 template <typename T>
 lns_status grow(T *&p, size_t &cap, size_t need)
 {
     if (need <= cap && p) return LNS_OK;
-    if (p) cudaFree(p);
+    pool_free(p);
     p = nullptr; cap = 0;
-    if (cudaMalloc(&p, need * sizeof(T) + 16) != cudaSuccess) { cudaGetLastError(); return fail(LNS_ENOMEM, "cudaMalloc failed"); }
+    if (pool_alloc(&p, need * sizeof(T) + 16) != cudaSuccess) return fail(LNS_ENOMEM, "cudaMalloc failed");
     cap = need;
     return LNS_OK;
 }
@@ -1881,6 +1967,32 @@ const char *lns_strerror(lns_status s)
 const char *lns_last_error(void) { return g_err.c_str(); }
 int32_t lns_version(void) { return LNS_VERSION_NUM; }
 
+void lns_pool_trim(void)
+{
+    Pool &P = pool();
+    std::multimap<std::pair<int, size_t>, void *> drop;
+    {
+        std::lock_guard<std::mutex> lk(P.mu);
+        drop.swap(P.cache);
+        P.cached = 0;
+    }
+    int cur = 0;
+    cudaGetDevice(&cur);
+    for (auto &kv : drop) {
+        cudaSetDevice(kv.first.first);
+        cudaFree(kv.second);
+    }
+    cudaSetDevice(cur);
+}
+
+void lns_pool_stats(int64_t *cached_bytes, int64_t *live_bytes)
+{
+    Pool &P = pool();
+    std::lock_guard<std::mutex> lk(P.mu);
+    if (cached_bytes) *cached_bytes = (int64_t)P.cached;
+    if (live_bytes) *live_bytes = (int64_t)P.live_bytes;
+}
+
 int64_t lns_neighborhood_size(int32_t n, int32_t k)
 {
     if (k < 1 || k > 3) return -1;
@@ -1924,12 +2036,11 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     if (cudaDeviceGetAttribute(&c->numSMs, cudaDevAttrMultiProcessorCount, device) != cudaSuccess ||
         cudaDeviceGetAttribute(&c->smemOptin, cudaDevAttrMaxSharedMemoryPerBlockOptin, device) != cudaSuccess)
         return cleanup(fail(LNS_ECUDA, "device attributes"));
-    if (cudaMalloc(&c->d_Arow, arow.size() * 4) != cudaSuccess || cudaMalloc(&c->d_H, (n + 1) * 4) != cudaSuccess ||
-        cudaMalloc(&c->d_vb, NWn * 4) != cudaSuccess || cudaMalloc(&c->d_Y, m * 4) != cudaSuccess ||
-        cudaMalloc(&c->d_fs, FS_N * 8) != cudaSuccess || cudaMalloc(&c->d_slots, SLOT_N * 8) != cudaSuccess ||
-        cudaMalloc(&c->d_counter, sizeof(unsigned)) != cudaSuccess || cudaMalloc(&c->d_V, n) != cudaSuccess ||
-        cudaMalloc(&c->d_Yin, m * 4) != cudaSuccess) {
-        cudaGetLastError();
+    if (pool_alloc(&c->d_Arow, arow.size() * 4) != cudaSuccess || pool_alloc(&c->d_H, (n + 1) * 4) != cudaSuccess ||
+        pool_alloc(&c->d_vb, NWn * 4) != cudaSuccess || pool_alloc(&c->d_Y, m * 4) != cudaSuccess ||
+        pool_alloc(&c->d_fs, FS_N * 8) != cudaSuccess || pool_alloc(&c->d_slots, SLOT_N * 8) != cudaSuccess ||
+        pool_alloc(&c->d_counter, sizeof(unsigned)) != cudaSuccess || pool_alloc(&c->d_V, n) != cudaSuccess ||
+        pool_alloc(&c->d_Yin, m * 4) != cudaSuccess) {
         return cleanup(fail(LNS_ENOMEM, "cudaMalloc failed"));
     }
     if (cudaMemcpy(c->d_Arow, arow.data(), arow.size() * 4, cudaMemcpyHostToDevice) != cudaSuccess ||
@@ -1945,10 +2056,12 @@ void lns_destroy(lns_ctx *c)
 {
     if (!c) return;
     DeviceGuard g(c->device);
-    cudaFree(c->d_Arow); cudaFree(c->d_H); cudaFree(c->d_vb); cudaFree(c->d_Y); cudaFree(c->d_fs);
-    cudaFree(c->d_slots); cudaFree(c->d_counter); cudaFree(c->d_V); cudaFree(c->d_Yin); cudaFree(c->d_bits);
-    cudaFree(c->d_until); cudaFree(c->d_tr); cudaFree(c->d_tf); cudaFree(c->d_fit);
-    cudaFree(c->d_V0s); cudaFree(c->d_res); cudaFree(c->d_vouts); cudaFree(c->d_gslots); cudaFree(c->d_X);
+    if (c->step_active) cudaDeviceSynchronize();  // an open stepped search may still run kernels
+    for (void *p : {(void *)c->d_Arow, (void *)c->d_H, (void *)c->d_vb, (void *)c->d_Y, (void *)c->d_fs,
+                    (void *)c->d_slots, (void *)c->d_counter, (void *)c->d_V, (void *)c->d_Yin, (void *)c->d_bits,
+                    (void *)c->d_until, (void *)c->d_tr, (void *)c->d_tf, (void *)c->d_fit, (void *)c->d_V0s,
+                    (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X})
+        pool_free(p);
     for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
     cudaFree(c->d_xbuf); cudaFree(c->d_peers);
     if (c->ev0) cudaEventDestroy(c->ev0);

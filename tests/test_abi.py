@@ -53,6 +53,8 @@ def test_host_only_entry_points():
             assert L.lns_neighborhood_size(n, k) == comb(n, k)
     assert L.lns_neighborhood_size(10, 4) == -1
     assert L.lns_strerror(L.LNS_ENOADMISSIBLE) == "no admissible neighbour"
+    cached, live = L.lns_pool_stats()  # host-only: the device-memory cache's counters
+    assert cached >= 0 and live >= 0
 
 
 def test_no_cpu_fallback_without_gpu():

@@ -499,3 +499,31 @@ def test_peer_exchange_missing_partition_times_out(L):
     finally:
         for cx in ctxs:
             L.lns_destroy(cx)
+
+
+def test_pool_recycles_context_buffers(L, orc):
+    """create -> batch -> destroy cycles reuse the library's cached device blocks (include/lns.h,
+    device-memory cache): the second cycle allocates nothing new, every block is returned at
+    destroy, and recycled (not re-zeroed) buffers give the same oracle-exact results."""
+    inst = pi.config_instance("C3")
+    seed, R, iters = 77, 4, 30
+    ten = pi.default_tenure(inst.n, 3)
+    outs, footprint = [], []
+    for _ in range(3):
+        ctx = L.lns_create(inst.A, inst.S, 0)
+        Vo = np.empty((R, inst.n), np.int8)
+        outs.append((L.lns_tabu_run_batch(ctx, 3, R, iters, -1, seed, None, 0, Vo), Vo.copy()))
+        cached, live = L.lns_pool_stats()
+        assert live > 0
+        L.lns_destroy(ctx)
+        cached2, live2 = L.lns_pool_stats()
+        assert cached2 == cached + live and live2 == 0
+        footprint.append(cached2)
+    assert footprint[1] == footprint[0] == footprint[2]
+    for res, Vo in outs[1:]:
+        assert res == outs[0][0] and np.array_equal(Vo, outs[0][1])
+    V0 = pi.start_vector(inst.n, pi.restart_seed(seed, 1))
+    _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0, iters, ten, stop_on_zero=False)
+    assert outs[2][0][1] == ores and np.array_equal(outs[2][1][1], oVo)
+    L.lns_pool_trim()
+    assert L.lns_pool_stats() == (0, 0)
