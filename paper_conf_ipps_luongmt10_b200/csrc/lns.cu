@@ -183,13 +183,16 @@ struct PlanScalars {
     // destinations negative: cost linear, aggregated as cneg - 240 sum t over the first rneg sorted
     // rows); points u >= utop land only above max(S) (zero cost) and are skipped
     int uneg, utop, rneg, cneg;
-    // packed path (abs form): sum of H_b over the walked bins [uneg, utop + 2K),
-    // H of the 2K trailing bins as bytes, and whether any trailing bin is negative (w != 0)
-    int hwalk, trlin;
+    // packed path (abs form): sum of H_b over the walked bins
+    int hwalk;
     int Wp;    // row words X holds this plan (ceil(row slots / 32); padded slots are holes)
     int rtop;  // rows below the top cut (points < utop), unpadded
-    uint32_t htr_lo, htr_hi;
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
+    // packed path, parity walks (build_plan_pk): records of walk 0 are [0, pkb1),
+    // of walk 1 [pkb1, P); first row word, initial byte window, last point, trailing H bytes and
+    // "a trailing bin is negative" of each walk
+    int pkb1, pkw0[2], pkz[2], pktrl[2];
+    uint32_t pkwin[2], pkhtr[2];
     unsigned long long key, gkey;
     int red[2 * NWARP + 2];
 };
@@ -315,6 +318,196 @@ __device__ __forceinline__ void range_publish(int mn, int mx, PlanScalars &ps)
     }
 }
 
+// Plan step D: X[w][c], per (row word, column word) pair, lane l loads sorted row 32w+l's sign
+// bits of columns 32cw..32cw+31 (rowAt[p] = -1 marks a hole) and a 5-round shuffle transpose turns
+// rows into columns; zero cnt[] for the next plan.
+__device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L,
+                                               const PlanScalars &ps, uint32_t *X, int Uc)
+{
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int m = I.m, n = I.n, NWn = I.NWn;
+    const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
+    const int *rowAt = (const int *)(sm + L.rowAt);
+    int *cnt = (int *)(sm + L.cnt);
+    for (int u = tid; u < Uc; u += NT) cnt[u] = 0;
+    const int Wp = ps.Wp;
+    for (int pr = warp; pr < Wp * NWn; pr += NWARP) {
+        const int w = pr / NWn, cw = pr - w * NWn;
+        const int p = 32 * w + lane;
+        const int j = I.pad ? rowAt[p] : (p < m ? rowAt[p] : -1);
+        uint32_t x = j >= 0 ? (Ar[(size_t)j * NWn + cw] ^ vbs[cw]) : 0u;
+#pragma unroll
+        for (int j = 16; j >= 1; j >>= 1) {
+            const uint32_t mk = j == 16 ? 0x0000FFFFu : j == 8 ? 0x00FF00FFu : j == 4 ? 0x0F0F0F0Fu
+                              : j == 2 ? 0x33333333u : 0x55555555u;
+            const uint32_t y = __shfl_xor_sync(FULL, x, j);
+            x = (lane & j) ? ((x & ~mk) | ((y & ~mk) >> j)) : ((x & mk) | ((y & mk) << j));
+        }
+        const int c = 32 * cw + lane;
+        if (c < n) X[w * n + c] = x;
+    }
+    __syncthreads();
+    PH(3);
+}
+
+// ------------------------------------------------------------------------------------------
+// Plan of the packed path (m <= 255, every bin count fits a byte), DESIGN.md §5.9. A row at lattice
+// point u moves to bin u + 2t (t = #{i in F : x_ji = 1}), so bins of one parity of u only receive
+// rows of that parity: the walked points [uneg, utop) split into two independent WALKS, walk p =
+// points uneg + p, uneg + p + 2, ... In half-lattice units a point's rows land in its own bin and
+// the next K bins of its walk, so a walk's open bins fit the four bytes of ONE 32-bit window.
+// Row order: deep points (u < uneg, all destinations negative: linear cost, no records), walk 0,
+// walk 1 (segments padded so that one of <= 32 rows never straddles a row word when I.pad), then
+// the points above the top cut (no records; every such row costs 1). Records (uint4), one per
+// (point, row word) piece, in walk order:
+//   final piece of point u: (mask, L(u + 8), H_b << 8 | 8, 0x4404 | w_b << 16), b = vmin + 2(u - K)
+//   earlier pieces:         (mask, 0,        0,            0x4444)
+// L(u + 8) = rows of the point four steps ahead in the same walk (0 past utop): the funnel shift that
+// completes bin u inserts it as the window's new top byte. w_b = 60|b| - 1 for b < 0, else 0.
+// pstart[w] = first record in row word w (INT_MAX if none).
+// ------------------------------------------------------------------------------------------
+template <int K, bool XG = false>
+__device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                              uint32_t *Xarg)
+{
+    uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int m = I.m, n = I.n;
+    const int *Ys = (const int *)(sm + L.Y);
+    const int *Hs = (const int *)(sm + L.H);
+    int *cnt = (int *)(sm + L.cnt);
+    int *seg = (int *)(sm + L.seg);
+    int *cur = (int *)(sm + L.cur);
+    int *pofs = (int *)(sm + L.pofs);
+    int *rowAt = (int *)(sm + L.rowAt);
+    int2 *bins = (int2 *)(sm + L.bins);
+    uint4 *pk = (uint4 *)(sm + L.pk);
+    int *pstart = (int *)(sm + L.pstart);
+    const int vlo = ps.vlo, Uc = ps.Uc;
+
+    // A. counting sort over the conservative lattice; holes; no record starts anywhere yet
+    for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
+    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
+    for (int w = tid; w <= I.XW; w += NT) pstart[w] = INT_MAX;
+    __syncthreads();
+    PH(0);
+    // B. warp 0: exact range, cuts, and the placement in the order deep | walk 0 | walk 1 | top
+    if (warp == 0) {
+        int uf = -1, ul = -1;
+        for (int b0 = 0; b0 < Uc; b0 += 32) {
+            const unsigned bal = __ballot_sync(FULL, b0 + lane < Uc && cnt[b0 + lane] > 0);
+            if (bal) {
+                if (uf < 0) uf = b0 + __ffs(bal) - 1;
+                ul = b0 + 31 - __clz(bal);
+            }
+        }
+        const int U = ul - uf + 1;
+        const int vmin = vlo + 2 * uf;
+        int uneg = (-2 * K - vmin + 1) >> 1;  // least u with vmin + 2u >= -2K
+        uneg = min(max(uneg, 0), U);
+        int utop = ((I.maxS + 2 * K - vmin) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
+        utop = min(max(utop, uneg), U);
+        const int n0 = (utop - uneg + 1) >> 1, n1 = (utop - uneg) >> 1;  // points of walk 0 / 1
+        int pos = 0, rows = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0;
+        for (int q0 = 0; q0 < U; q0 += 32) {
+            const int q = q0 + lane;
+            const int v = q < uneg ? q : q < uneg + n0 ? uneg + 2 * (q - uneg)
+                        : q < utop ? uneg + 1 + 2 * (q - uneg - n0) : q;
+            const int Lq = q < U ? cnt[uf + v] : 0;
+            int myP = 0, myO = 0;
+            const int nv = min(32, U - q0);
+            for (int i = 0; i < nv; i++) {
+                const int Li = __shfl_sync(FULL, Lq, i);
+                const int qi = q0 + i;
+                const bool walk = qi >= uneg && qi < utop;
+                if (qi == uneg) rneg = rows;
+                if (qi == uneg + n0) pkb1 = runp;
+                if (qi == utop) rtop = rows;
+                if (walk && I.pad && Li > 0 && (pos & 31) != 0 && (pos & 31) + Li > 32) pos = (pos + 31) & ~31;
+                if (lane == i) { myP = pos; myO = runp; }
+                if (walk) runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : 1;
+                pos += Li;
+                rows += Li;
+            }
+            if (q < U) { seg[v] = myP; cur[uf + v] = myP; pofs[v] = myO; }
+        }
+        if (uneg >= U) rneg = rows;
+        if (uneg + n0 >= U) pkb1 = runp;
+        if (utop >= U) rtop = rows;
+        if (lane < 2) {  // walk p = lane: first / last point, initial window, trailing bins
+            const int np = lane ? n1 : n0, a = uneg + lane, z = a + 2 * (np - 1);
+            uint32_t win = 0, htr = 0;
+            int trl = 0;
+            if (np > 0) {
+                for (int i = 0; i < 4; i++)
+                    if (a + 2 * i <= z) win |= (uint32_t)cnt[uf + a + 2 * i] << (8 * i);
+                for (int i = 1; i <= K; i++) {
+                    const int b = vmin + 2 * (z + 2 * i - K);
+                    if (b >= 0 && b <= n) htr |= (uint32_t)Hs[b] << (8 * (i - 1));
+                    if (b < 0) trl = 1;
+                }
+            }
+            ps.pkwin[lane] = win; ps.pkhtr[lane] = htr; ps.pktrl[lane] = trl; ps.pkz[lane] = np > 0 ? z : -1;
+            ps.pkw0[lane] = 0;
+        }
+        if (lane == 0) {
+            ps.P = runp; ps.pkb1 = pkb1; ps.Wp = (pos + 31) >> 5;
+            ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
+            ps.uneg = uneg; ps.utop = utop; ps.rneg = rneg; ps.rtop = rtop; ps.cneg = 0; ps.hwalk = 0;
+            ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
+            ps.key = (unsigned long long)KEY_NONE;
+            ps.gkey = (unsigned long long)KEY_NONE;
+        }
+    }
+    __syncthreads();
+    PH(1);
+    // C. place rows; emit the records (one thread per walked point); bin constants; deep constant
+    const int vmin = ps.vmin, U = ps.U, NB = ps.NB, uf = ps.ufirst, uneg = ps.uneg, utop = ps.utop;
+    for (int j = tid; j < m; j += NT) {
+        const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
+        rowAt[p] = j;
+    }
+    for (int v = uneg + tid; v < utop; v += NT) {
+        const int st = seg[v], Lv = cnt[uf + v], en = st + Lv;
+        int p = pofs[v];
+        const int b = vmin + 2 * (v - K);
+        const uint32_t Hfin = ((b >= 0 && b <= n) ? (uint32_t)Hs[b] << 8 : 0u) | 8u;
+        const uint32_t wfin = 0x4404u | ((b < 0 ? (uint32_t)(60 * (-b) - 1) : 0u) << 16);
+        const uint32_t src = v + 8 < utop ? (uint32_t)cnt[uf + v + 8] : 0u;
+        if (Lv == 0) {  // empty point: one zero record (in the previous row word) that completes its bin
+            const int w = max(0, (st - 1) >> 5);
+            pk[p] = make_uint4(0u, src, Hfin, wfin);
+            atomicMin(&pstart[w], p);
+            if (v - uneg < 2) ps.pkw0[v - uneg] = w;
+            continue;
+        }
+        const int w0 = st >> 5, w1 = (en - 1) >> 5;
+        if (v - uneg < 2) ps.pkw0[v - uneg] = w0;
+        for (int w = w0; w <= w1; w++, p++) {
+            const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
+            const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
+            pk[p] = w == w1 ? make_uint4(mask, src, Hfin, wfin) : make_uint4(mask, 0u, 0u, 0x4444u);
+            atomicMin(&pstart[w], p);
+        }
+    }
+    for (int v = tid; v < uneg; v += NT)  // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form)
+        if (cnt[uf + v] > 0)
+            atomicAdd((unsigned *)&ps.cneg, (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v))));
+    const int z0 = ps.pkz[0], z1 = ps.pkz[1];
+    for (int beta = tid; beta < NB; beta += NT) {
+        const int b = vmin + 2 * (beta - K);
+        const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
+        bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
+        // walked bins: [first point, last point + 2K] of the walk of beta's parity
+        const int zp = ((beta - uneg) & 1) ? z1 : z0;
+        if (Hb && beta >= uneg && zp >= 0 && beta <= zp + 2 * K) atomicAdd(&ps.hwalk, Hb);
+    }
+    __syncthreads();
+    PH(2);
+    // D. X
+    plan_transpose(I, Ar, sm, L, ps, X, Uc);
+}
+
 // ------------------------------------------------------------------------------------------
 // Plan: per-iteration shared-memory structures of the current state (Y, V). Requires cnt[] = 0
 // and a lattice ps.vlo / Uc covering every Y (the exact range after load_state, or the previous
@@ -333,11 +526,11 @@ template <int K, bool XG = false>
 __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
                            uint32_t *Xarg)
 {
+    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg); return; }
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
-    const int m = I.m, n = I.n, NWn = I.NWn;
+    const int m = I.m, n = I.n;
     const int *Ys = (const int *)(sm + L.Y);
-    const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
     const int *Hs = (const int *)(sm + L.H);
     int *cnt = (int *)(sm + L.cnt);
     int *seg = (int *)(sm + L.seg);
@@ -349,9 +542,8 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     int *pstart = (int *)(sm + L.pstart);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
-    // A. counting sort over the conservative lattice (and mark every row slot a hole)
+    // A. counting sort over the conservative lattice
     for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
-    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
     __syncthreads();
     PH(0);
     // B. warp 0: exact range (first / last non-empty point), exclusive scans of the row and piece
@@ -387,39 +579,13 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         uneg = min(max(uneg, 0), U);
         int utop = ((I.maxS + 2 * K - vmin_) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
-        int Wp = (m + 31) >> 5;
+        const int Wp = (m + 31) >> 5;
         __syncwarp();
-        if (lane == 0) ps.rtop = utop < U ? seg[utop] : runr;  // unpadded rows below the top cut
-        if (I.pad) {
-            // padded placement: segments go in order; one that would straddle a row
-            // word while starting mid-word starts at the next word instead, so it stays one piece.
-            // At most 2W + 1 words (a word is left short only when the next segment does not fit).
-            __syncwarp();
-            int pos = 0;
-            runp = 0;
-            for (int b0 = 0; b0 < U; b0 += 32) {
-                const int v_ = b0 + lane;
-                const int L = v_ < U ? cnt[uf + v_] : 0;
-                int myP = 0, myO = 0;
-                const int nv = min(32, U - b0);
-                for (int i = 0; i < nv; i++) {
-                    const int Li = __shfl_sync(FULL, L, i);
-                    if (Li > 0 && (pos & 31) != 0 && (pos & 31) + Li > 32) pos = (pos + 31) & ~31;
-                    if (lane == i) { myP = pos; myO = runp; }
-                    runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : 1;
-                    pos += Li;
-                }
-                if (v_ < U) { seg[v_] = myP; cur[uf + v_] = myP; pofs[v_] = myO; }
-            }
-            runr = pos;
-            Wp = (pos + 31) >> 5;
-        }
         if (lane == 0) {
             const int vmin = vmin_;
             seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[Wp] = runp; ps.Wp = Wp;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
             ps.uneg = uneg; ps.utop = utop; ps.cneg = 0;
-            ps.hwalk = 0; ps.trlin = 0; ps.htr_lo = 0; ps.htr_hi = 0;
             ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
             ps.key = (unsigned long long)KEY_NONE;
             ps.gkey = (unsigned long long)KEY_NONE;
@@ -435,27 +601,15 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         rowAt[p] = j;
     }
     const int uneg = ps.uneg;
-    uint4 *pk = (uint4 *)(sm + L.pk);
-    const bool packed = m <= PACKED_MAX_M;
     for (int v = tid; v < U; v += NT) {
-        const int st = seg[v], en = st + cnt[uf + v];  // padded start, real length
+        const int st = seg[v], en = st + cnt[uf + v];
         int p = pofs[v];
-        // packed-path record of this point's last piece (it completes bin beta = v, b = vmin + 2(v - K)):
-        //   (mask, len, H_b << 8 | 8, PK_SEL_FIN | w_b << 16)
-        // earlier pieces: (mask, 0, 0, PK_SEL_NONE) -- no shift, and h reads an always-zero byte.
-        // The low byte of z is the window shift; the SAD of hb (byte 0 = 0) against z adds it to f,
-        // 8 per final piece, which the constant C takes back
-        const int bfin = vmin + 2 * (v - K);
-        const uint32_t Hfin = ((bfin >= 0 && bfin <= n) ? (uint32_t)Hs[bfin] << 8 : 0u) | 8u;
-        const uint32_t wfin = PK_SEL_FIN | ((bfin < 0 ? (uint32_t)(60 * (-bfin) - 1) : 0u) << 16);
         // deep-negative constant sum_rows 60(2K - Y_j) - 1 (unsigned: the constant may exceed
         // 2^31 on its own; the fitness it enters does not)
-        // (the packed path's abs form counts 60 |b| per deep row, without the -1: DESIGN.md §5.9)
         if (v < uneg && en > st)
-            atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - (packed ? 0 : 1)));
+            atomicAdd((unsigned *)&ps.cneg, (unsigned)(en - st) * (unsigned)(60 * (2 * K - (vmin + 2 * v)) - 1));
         if (st == en) {  // empty lattice point: a zero piece (in the previous row word) that finalises its bin
             pieces[p] = make_uint2(0u, 1u | ((uint32_t)((st - 1) >> 5) << 1));
-            if (packed) pk[p] = make_uint4(0u, 0u, Hfin, wfin);
             continue;
         }
         const int w0 = st >> 5, w1 = (en - 1) >> 5;
@@ -463,49 +617,17 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
             const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
             pieces[p] = make_uint2(mask, (uint32_t)(w == w1 ? 1 : 0) | ((uint32_t)w << 1) | ((uint32_t)(en - st) << 16));
-            if (packed)
-                pk[p] = w == w1 ? make_uint4(mask, (uint32_t)(en - st), Hfin, wfin)
-                                : make_uint4(mask, 0u, 0u, PK_SEL_NONE);
             if (w > w0 || (st & 31) == 0) pstart[w] = p;
         }
     }
-    const int utop = ps.utop;
     for (int beta = tid; beta < NB; beta += NT) {
         const int b = vmin + 2 * (beta - K);
         const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
         bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
-        if (packed && beta >= uneg && beta < utop + 2 * K) {
-            if (Hb) atomicAdd(&ps.hwalk, Hb);
-            if (beta >= utop) {
-                const int i = beta - utop;
-                if (Hb) atomicOr(i < 4 ? &ps.htr_lo : &ps.htr_hi, (uint32_t)Hb << (8 * (i & 3)));
-                if (b < 0) atomicOr(&ps.trlin, 1);
-            }
-        }
     }
     __syncthreads();
     PH(2);
-    // D. X[w][c]: per (row word, column word) pair, lane l loads sorted row 32w+l's sign bits of
-    //    columns 32cw..32cw+31 and a 5-round shuffle transpose turns rows into columns; zero cnt[]
-    for (int u = tid; u < Uc; u += NT) cnt[u] = 0;
-    const int Wp = ps.Wp;
-    for (int pr = warp; pr < Wp * NWn; pr += NWARP) {
-        const int w = pr / NWn, cw = pr - w * NWn;
-        const int p = 32 * w + lane;
-        const int j = I.pad ? rowAt[p] : (p < m ? rowAt[p] : -1);
-        uint32_t x = j >= 0 ? (Ar[(size_t)j * NWn + cw] ^ vbs[cw]) : 0u;
-#pragma unroll
-        for (int j = 16; j >= 1; j >>= 1) {
-            const uint32_t mk = j == 16 ? 0x0000FFFFu : j == 8 ? 0x00FF00FFu : j == 4 ? 0x0F0F0F0Fu
-                              : j == 2 ? 0x33333333u : 0x55555555u;
-            const uint32_t y = __shfl_xor_sync(FULL, x, j);
-            x = (lane & j) ? ((x & ~mk) | ((y & ~mk) >> j)) : ((x & mk) | ((y & mk) << j));
-        }
-        const int c = 32 * cw + lane;
-        if (c < n) X[w * n + c] = x;
-    }
-    __syncthreads();
-    PH(3);
+    plan_transpose(I, Ar, sm, L, ps, X, Uc);
 }
 
 // One lattice point (segment) of eval_fit: its pieces add POPC counts of the bit-sliced planes
@@ -575,11 +697,6 @@ struct EvalRange {
     int u0, u1;       // lattice points [u0, u1) go through the segment loop (u0 = uneg, u1 = utop)
     int rneg, cneg;   // deep-negative rows [0, rneg) and their constant part
     int p0;           // first piece of point u0
-    int p1;           // first piece of point u1 (packed path)
-    int w0;           // row word of piece p0 (packed path)
-    int cabs;         // packed path: the fitness constant C
-    int trlin;        // packed path: some trailing bin is negative (scalar trailing)
-    uint32_t htr_lo, htr_hi;
 };
 
 // Deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
@@ -655,50 +772,17 @@ __device__ __forceinline__ int eval_fit(const uint32_t *__restrict__ X, const ui
     return f - 2 * smin;
 }
 
-// eval_fit for m <= 255 (every bin count fits a byte): the 2K+1 open bins beta .. beta+2K live as
-// bytes of the 64-bit window (whi:wlo), byte i = bin beta+i. A piece adds its row counts straight
-// into the window (N0 -> byte 0, N1 -> byte 2, N2 -> byte 4, N3 -> byte 6, with N0 = len - sum_t N_t
-// added as -sum_t N_t now and len at the segment's end); byte 0 may go transiently negative, which
-// is harmless because each half is exact modulo 2^32 and its final bytes all lie in [0, 255].
-// Completing bin beta = adding len, reading byte 0, shifting the window down 8 bits. The walk is
-// word-major (the lane's three column words are loaded once per row word) and inside a word every
-// piece but the last finalises its bin, so the inner loop has no branch.
-template <int K>
-__device__ __forceinline__ void packed_add(uint32_t m, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &wlo, uint32_t &whi)
-{
-    const int p1 = __popc(lo & m);
-    if (K == 1) {               // N1 = p1 -> byte 2; -p1 -> byte 0
-        wlo += (uint32_t)p1 * 65535u;
-    } else if (K == 2) {        // N1 = p1 -> byte 2, N2 = p2 -> byte 4
-        const int p2 = __popc(hi & m);
-        wlo += ((uint32_t)p1 << 16) - (uint32_t)p1 - (uint32_t)p2;
-        whi += (uint32_t)p2;
-    } else {                    // N1 = p1 - p3 -> byte 2, N2 = p2 - p3 -> byte 4, N3 = p3 -> byte 6
-        const int p2 = __popc(hi & m), p3 = __popc(lh & m);
-        const uint32_t d1 = (uint32_t)(p1 - p3);
-        wlo += (d1 << 16) - d1 - (uint32_t)p2;
-        whi += (uint32_t)p2 + (uint32_t)p3 * 65535u;
-    }
-}
-
-// One packed record applied to one neighbour's window (see eval_fit_packed).
-template <int K>
-__device__ __forceinline__ void packed_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &wlo,
-                                            uint32_t &whi, int &f)
-{
-    packed_add<K>(r.x, lo, hi, lh, wlo, whi);
-    wlo += r.y;  // len
-    // hb = h << 8 (h = byte 0 of the window, or 0 for a piece that completes no bin); prmt reads
-    // only the low 16 bits of its selector
-    uint32_t hb, fu = (uint32_t)f;
-    asm("prmt.b32 %0, %1, %2, %3;" : "=r"(hb) : "r"(wlo), "r"(whi), "r"(r.w));
-    fu = __dp2a_lo(r.w, hb, fu);  // + w_b h (w_b in the high half of r.w)
-    asm("vabsdiff4.u32.u32.u32.add %0, %1, %2, %3;" : "=r"(fu) : "r"(hb), "r"(r.z), "r"(fu));  // + |h - H_b| (+ shift)
-    f = (int)fu;
-    wlo = __funnelshift_r(wlo, whi, r.z);  // shift = r.z & 31 (8 or 0)
-    whi = __funnelshift_r(whi, 0u, r.z);
-}
-
+// ---- packed path (m <= 255), parity walks (build_plan_pk) ------------------
+// A walk's open bins live in the four bytes of one 32-bit window w: byte i = bin u + 2i of the
+// walk (u = the point being processed), initialised with the rows of those points ("len") and
+// receiving each point's rows as they move: a piece with row counts c1 = |lo & mask|,
+// c2 = |hi & mask|, c3 = |lh & mask| moves N1 = c1 - c3 rows to byte 1, N2 = c2 - c3 to byte 2 and
+// N3 = c3 to byte 3, all out of byte 0:
+//   w += 255 N1 + 65535 N2 + 16777215 N3 = 255 c1 + 65535 c2 + 16711425 c3      (K = 3)
+// Bytes may go transiently negative inside the register; it is exact modulo 2^32 and every byte
+// is a count in [0, 255] whenever it is read or shifted. The final piece of a point completes
+// bin u (byte 0): f += w_b h + |h - H_b| (+ 8, taken out of the constant C), and the funnel shift
+// by 8 drops it and inserts the rows of the point four steps ahead as the new top byte.
 template <int K>
 __device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int a, int b, int c, uint32_t &lo,
                                             uint32_t &hi, uint32_t &lh)
@@ -716,90 +800,126 @@ __device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int
     }
 }
 
-// The 2K bins past the last walked point hold only carried counts (bytes 0 .. 2K-1 of the window;
-// the higher bytes are zero). When none of them is negative their cost is sum |h - H| over the
-// bytes, two SAD instructions against the plan's packed H; otherwise per bin.
 template <int K>
-__device__ __forceinline__ void packed_trail(const EvalRange &er, const int2 *__restrict__ bins, uint32_t wlo,
-                                             uint32_t whi, int &f)
+__device__ __forceinline__ void pk_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &w, int &f)
 {
-    if (!er.trlin) {
-        f += (int)__vsadu4(wlo, er.htr_lo);
-        if (K >= 2) f += (int)__vsadu4(whi, er.htr_hi);
+    w += 255u * (uint32_t)__popc(lo & r.x);
+    if (K >= 2) w += 65535u * (uint32_t)__popc(hi & r.x);
+    if (K == 3) w += 16711425u * (uint32_t)__popc(lh & r.x);
+    // hb: byte 1 = h (byte 0 of w) for a final piece (selector 0x4404), 0 otherwise (0x4444)
+    uint32_t hb, fu = (uint32_t)f;
+    asm("prmt.b32 %0, %1, %2, %3;" : "=r"(hb) : "r"(w), "r"(0u), "r"(r.w));
+    fu = __dp2a_lo(r.w, hb, fu);  // + w_b h (w_b in the high half of r.w; the selector meets byte 0 = 0)
+    asm("vabsdiff4.u32.u32.u32.add %0, %1, %2, %3;" : "=r"(fu) : "r"(hb), "r"(r.z), "r"(fu));  // + |h - H_b| + shift
+    f = (int)fu;
+    w = __funnelshift_r(w, r.y, r.z);  // shift r.z & 31 (8 or 0); r.y byte 0 enters as byte 3
+}
+
+// The packed plan's scalars are read from shared memory (PlanScalars) where they are used, which
+// keeps them out of the registers of the record loop.
+// The K bins past a walk's last point hold only carried rows (bytes 0 .. K-1 of w; the rest are
+// 0): sum |h - H| is one SAD against the packed H, unless one of them is negative (w_b != 0).
+template <int K>
+__device__ __forceinline__ void pk_trail(const PlanScalars &ps, int q, const int2 *__restrict__ bins, uint32_t w, int &f)
+{
+    if (!ps.pktrl[q]) {
+        f += (int)__vsadu4(w, ps.pkhtr[q]);
         return;
     }
-    const int2 *bp = bins + er.u1;
 #pragma unroll
-    for (int i = 0; i < 2 * K; i++) {
-        const int h = (int)(((i < 4 ? wlo >> (8 * i) : whi >> (8 * (i - 4)))) & 0xffu);
-        const int2 bn = bp[i];
+    for (int i = 0; i < K; i++) {
+        const int h = (int)((w >> (8 * i)) & 0xffu);
+        const int2 bn = bins[ps.pkz[q] + 2 * (i + 1)];
         f += bn.y * h + abs(h - bn.x);
     }
 }
 
-// eval_fit for m <= 255, abs form:
-//   f = C + [deep rows] + sum over walked bins beta of ( w_beta h_beta + |h_beta - H_beta| )
-// with C = m - sum_{walked b in [0,n]} H_b + (rows above the top cut). Two neighbours per thread:
-// the record stream, loop control and word bookkeeping are shared.
-template <int K, bool DEEP>
-__device__ __forceinline__ void eval_fit_packed2(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
-                                                 const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
-                                                 const EvalRange &er, int a0, int b0, int c0, int a1, int b1,
-                                                 int c1, int &f0, int &f1)
+// Column words of row word xr: LDS when X is in shared memory (XG = false; a 32-bit shared
+// address), plain loads for the global-memory X of very large instances.
+template <int K, bool XG>
+__device__ __forceinline__ void pk_planes(const uint32_t *__restrict__ Xg, uint32_t xs, int a, int b, int c,
+                                          uint32_t &lo, uint32_t &hi, uint32_t &lh)
 {
-    f0 = er.cabs; f1 = er.cabs;
-    if (DEEP) { f0 = deep_negative<K>(X, n, er, f0, a0, b0, c0); f1 = deep_negative<K>(X, n, er, f1, a1, b1, c1); }
-    uint32_t wl0 = 0, wh0 = 0, wl1 = 0, wh1 = 0;
-    if (er.u1 > er.u0) {
-        const uint4 *pp = pk + er.p0;
-        const uint32_t *xr = X + er.w0 * n;
-        const int *pw = pstart + er.w0 + 1;
-        for (;;) {
-            uint32_t lo0, hi0, lh0, lo1, hi1, lh1;
-            load_planes<K>(xr, a0, b0, c0, lo0, hi0, lh0);
-            load_planes<K>(xr, a1, b1, c1, lo1, hi1, lh1);
-            xr += n;
-            const int pend = min(*pw++, er.p1);
-            const uint4 *pe = pk + pend;
-#pragma unroll kPkUnroll
-            for (; pp < pe; ++pp) {
-                const uint4 r = *pp;
-                packed_step<K>(r, lo0, hi0, lh0, wl0, wh0, f0);
-                packed_step<K>(r, lo1, hi1, lh1, wl1, wh1, f1);
-            }
-            if (pend == er.p1) break;
-        }
+    uint32_t xa, xb = 0, xc = 0;
+    if (XG) {
+        xa = Xg[a];
+        if (K >= 2) xb = Xg[b];
+        if (K == 3) xc = Xg[c];
+    } else {
+        asm("ld.shared.u32 %0, [%1];" : "=r"(xa) : "r"(xs + 4u * a));
+        if (K >= 2) asm("ld.shared.u32 %0, [%1];" : "=r"(xb) : "r"(xs + 4u * b));
+        if (K == 3) asm("ld.shared.u32 %0, [%1];" : "=r"(xc) : "r"(xs + 4u * c));
     }
-    packed_trail<K>(er, bins, wl0, wh0, f0);
-    packed_trail<K>(er, bins, wl1, wh1, f1);
+    if (K == 1) {
+        lo = xa; hi = 0; lh = 0;
+    } else if (K == 2) {
+        lo = xa ^ xb; hi = xa & xb; lh = 0;
+    } else {
+        lo = xa ^ xb ^ xc;
+        hi = (xa & xb) | (xc & (xa ^ xb));
+        lh = lo & hi;
+    }
 }
 
-// One neighbour per thread (slices of at most one block pass).
-template <int K, bool DEEP>
-__device__ __forceinline__ int eval_fit_packed(const uint32_t *__restrict__ X, const uint4 *__restrict__ pk,
-                                               const int *__restrict__ pstart, const int2 *__restrict__ bins, int n,
-                                               const EvalRange &er, int a, int b, int c)
+// One walk q of NB neighbours (NB = 1 or 2, the second in a1, b1, c1): word-major (the lane's
+// column words are loaded once per row word), the record stream shared by the neighbours.
+template <int K, int NB, bool XG>
+__device__ __forceinline__ void pk_walk(const PlanScalars &ps, int q, const uint32_t *__restrict__ X,
+                                        const uint4 *__restrict__ pk, const int *__restrict__ pstart,
+                                        const int2 *__restrict__ bins, int n, int a0, int b0, int c0, int a1, int b1,
+                                        int c1, int &f0, int &f1)
 {
-    int f = er.cabs;
-    if (DEEP) f = deep_negative<K>(X, n, er, f, a, b, c);
-    uint32_t wlo = 0, whi = 0;
-    if (er.u1 > er.u0) {
-        const uint4 *pp = pk + er.p0;
-        const uint32_t *xr = X + er.w0 * n;
-        const int *pw = pstart + er.w0 + 1;
-        for (;;) {
-            uint32_t lo, hi, lh;
-            load_planes<K>(xr, a, b, c, lo, hi, lh);
-            xr += n;
-            const int pend = min(*pw++, er.p1);
-            const uint4 *pe = pk + pend;
+    const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
+    if (pb == pe) return;
+    uint32_t w0 = ps.pkwin[q], w1 = w0;
+    const uint4 *pp = pk + pb;
+    const int wd = ps.pkw0[q];
+    const uint32_t *xg = XG ? X + wd * n : nullptr;
+    uint32_t xs = XG ? 0u : (uint32_t)__cvta_generic_to_shared(X + wd * n);
+    const int *pw = pstart + wd + 1;
+    for (;;) {
+        uint32_t lo0, hi0, lh0, lo1 = 0, hi1 = 0, lh1 = 0;
+        pk_planes<K, XG>(xg, xs, a0, b0, c0, lo0, hi0, lh0);
+        if (NB == 2) pk_planes<K, XG>(xg, xs, a1, b1, c1, lo1, hi1, lh1);
+        if (XG) xg += n; else xs += 4u * n;
+        const int pend = min(*pw++, pe);
+        const uint4 *pz = pk + pend;
 #pragma unroll kPkUnroll
-            for (; pp < pe; ++pp) packed_step<K>(*pp, lo, hi, lh, wlo, whi, f);
-            if (pend == er.p1) break;
+        for (; pp < pz; ++pp) {
+            const uint4 r = *pp;
+            pk_step<K>(r, lo0, hi0, lh0, w0, f0);
+            if (NB == 2) pk_step<K>(r, lo1, hi1, lh1, w1, f1);
         }
+        if (pend == pe) break;
     }
-    packed_trail<K>(er, bins, wlo, whi, f);
-    return f;
+    pk_trail<K>(ps, q, bins, w0, f0);
+    if (NB == 2) pk_trail<K>(ps, q, bins, w1, f1);
+}
+
+// Deep rows (DEEP): every destination negative, cost cneg - 240 sum t (abs form).
+template <int K>
+__device__ __forceinline__ int pk_deep(const uint32_t *__restrict__ X, int n, const PlanScalars &ps, int f, int a,
+                                       int b, int c)
+{
+    EvalRange er;
+    er.rneg = ps.rneg; er.cneg = ps.cneg;
+    return deep_negative<K>(X, n, er, f, a, b, c);
+}
+
+template <int K, int NB, bool DEEP, bool XG>
+__device__ __forceinline__ void eval_pk(const PlanScalars &ps, int cabs, const uint32_t *__restrict__ X,
+                                        const uint4 *__restrict__ pk, const int *__restrict__ pstart,
+                                        const int2 *__restrict__ bins, int n, int a0, int b0, int c0, int a1, int b1,
+                                        int c1, int &f0, int &f1)
+{
+    f0 = cabs;
+    if (NB == 2) f1 = cabs;
+    if (DEEP) {
+        f0 = pk_deep<K>(X, n, ps, f0, a0, b0, c0);
+        if (NB == 2) f1 = pk_deep<K>(X, n, ps, f1, a1, b1, c1);
+    }
+    pk_walk<K, NB, XG>(ps, 0, X, pk, pstart, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
+    pk_walk<K, NB, XG>(ps, 1, X, pk, pstart, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
 }
 
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
@@ -821,12 +941,9 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     EvalRange er;
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
-    er.p1 = ((const int *)(sm + L.pofs))[er.u1];
-    if (packed) {  // abs form (deep rows: 60 |b| each, accumulated so by build_plan); C as in eval_fit_packed2
-        er.cabs = 2 * I.m - ps.hwalk - ps.rtop - 8 * (er.u1 - er.u0);
-        er.trlin = ps.trlin; er.htr_lo = ps.htr_lo; er.htr_hi = ps.htr_hi;
-    }
-    er.w0 = (int)((pieces[er.p0].y >> 1) & 0x7fffu);
+    // packed path, abs form: C = m - (H of the walked bins) + (rows above the top cut) - 8 (completed
+    // bins); deep rows cost 60 |b| each (cneg, accumulated so by build_plan_pk)
+    const int cabs = packed ? 2 * I.m - ps.hwalk - ps.rtop - 8 * (ps.utop - ps.uneg) : 0;
     const int *pstart = (const int *)(sm + L.pstart);
     const uint4 *pk = (const uint4 *)(sm + L.pk);
     unsigned long long best = (unsigned long long)KEY_NONE;
@@ -847,8 +964,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const uint32_t rb = vB ? rB : rA;
             if (!vB) { a1 = a0; b1 = b0; c1 = c0; }
             int fA, fB;
-            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
-            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
+            if (ps.rneg > 0) eval_pk<K, 2, true, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_pk<K, 2, false, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
             const bool tA = until && until[rA - ubase] >= t;
             const bool tB = until && until[rb - ubase] >= t;
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
@@ -879,8 +996,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 unrank_tab<K>(rb, I.n, M, T2, T3, a1, b1, c1);
             }
             int fA, fB;
-            if (er.rneg > 0) eval_fit_packed2<K, true>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
-            else eval_fit_packed2<K, false>(X, pk, pstart, bins, I.n, er, a0, b0, c0, a1, b1, c1, fA, fB);
+            if (ps.rneg > 0) eval_pk<K, 2, true, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
+            else eval_pk<K, 2, false, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
             const bool tA = until && until[rA - ubase] >= t;
             const bool tB = until && until[rb - ubase] >= t;
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
@@ -903,10 +1020,14 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 } else {
                     unrank_tab<K>(r, I.n, M, T2, T3, a, b, c);
                 }
-                const int f = packed ? (er.rneg > 0 ? eval_fit_packed<K, true>(X, pk, pstart, bins, I.n, er, a, b, c)
-                                                    : eval_fit_packed<K, false>(X, pk, pstart, bins, I.n, er, a, b, c))
-                                     : (er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
-                                                    : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c));
+                int f, g_;
+                if (packed) {
+                    if (ps.rneg > 0) eval_pk<K, 1, true, XG>(ps, cabs, X, pk, pstart, bins, I.n, a, b, c, a, b, c, f, g_);
+                    else eval_pk<K, 1, false, XG>(ps, cabs, X, pk, pstart, bins, I.n, a, b, c, a, b, c, f, g_);
+                } else {
+                    f = er.rneg > 0 ? eval_fit<K, true>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c)
+                                    : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c);
+                }
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 // admissible: not tabu, or (aspiration) better than the best fitness so far
