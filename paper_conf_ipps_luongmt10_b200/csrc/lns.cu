@@ -408,7 +408,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         int utop = ((I.maxS + 2 * K - vmin) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
         const int n0 = (utop - uneg + 1) >> 1, n1 = (utop - uneg) >> 1;  // points of walk 0 / 1
-        int pos = 0, rows = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0;
+        int pos = 0, rows = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0, prev = 0;
         for (int q0 = 0; q0 < U; q0 += 32) {
             const int q = q0 + lane;
             const int v = q < uneg ? q : q < uneg + n0 ? uneg + 2 * (q - uneg)
@@ -421,11 +421,18 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
                 const int qi = q0 + i;
                 const bool walk = qi >= uneg && qi < utop;
                 if (qi == uneg) rneg = rows;
-                if (qi == uneg + n0) pkb1 = runp;
+                if (qi == uneg + n0) { pkb1 = runp; prev = 0; }
                 if (qi == utop) rtop = rows;
                 if (walk && I.pad && Li > 0 && (pos & 31) != 0 && (pos & 31) + Li > 32) pos = (pos + 31) & ~31;
-                if (lane == i) { myP = pos; myO = runp; }
-                if (walk) runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : 1;
+                // an empty point whose bin and its predecessor's are non-negative is absorbed: the
+                // predecessor's final record completes both bins (no record of its own)
+                const bool nonneg = vmin + 2 * (__shfl_sync(FULL, v, i) - K) >= 0;
+                const bool absorbed = walk && Li == 0 && nonneg && prev == 2;
+                if (lane == i) { myP = pos; myO = absorbed ? -1 : runp; }
+                if (walk) {
+                    runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : (absorbed ? 0 : 1);
+                    prev = absorbed ? 1 : (nonneg ? 2 : 1);  // 2: a record that may absorb the next point
+                }
                 pos += Li;
                 rows += Li;
             }
@@ -470,10 +477,20 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     for (int v = uneg + tid; v < utop; v += NT) {
         const int st = seg[v], Lv = cnt[uf + v], en = st + Lv;
         int p = pofs[v];
+        if (p < 0) continue;  // absorbed by its predecessor
         const int b = vmin + 2 * (v - K);
-        const uint32_t Hfin = ((b >= 0 && b <= n) ? (uint32_t)Hs[b] << 8 : 0u) | 8u;
-        const uint32_t wfin = 0x4404u | ((b < 0 ? (uint32_t)(60 * (-b) - 1) : 0u) << 16);
-        const uint32_t src = v + 8 < utop ? (uint32_t)cnt[uf + v + 8] : 0u;
+        uint32_t Hfin = ((b >= 0 && b <= n) ? (uint32_t)Hs[b] << 8 : 0u) | 8u;
+        uint32_t wfin = 0x4404u | ((b < 0 ? (uint32_t)(60 * (-b) - 1) : 0u) << 16);
+        uint32_t src = v + 8 < utop ? (uint32_t)cnt[uf + v + 8] : 0u;
+        if (v + 2 < utop && pofs[v + 2] < 0) {
+            // two bins: v and the absorbed v + 2 (both weights 0): h_v -> byte 1, h_v+2 -> byte 2 of
+            // hb, H in bytes 1, 2 of z, shift 16 (the SAD adds 16 = 8 per bin), and the rows of the
+            // points v + 8, v + 10 enter as the new bytes 2, 3
+            const int b2 = b + 4;
+            Hfin = (b2 <= n ? (uint32_t)Hs[b2] << 16 : 0u) | (b <= n ? (uint32_t)Hs[b] << 8 : 0u) | 16u;
+            wfin = 0x4104u;
+            src |= (v + 10 < utop ? (uint32_t)cnt[uf + v + 10] : 0u) << 8;
+        }
         if (Lv == 0) {  // empty point: one zero record (in the previous row word) that completes its bin
             const int w = max(0, (st - 1) >> 5);
             pk[p] = make_uint4(0u, src, Hfin, wfin);
