@@ -87,6 +87,7 @@ struct DevInst {
 enum { FS_F = 0, FS_T, FS_BEST, FS_BESTIT, FS_ZERO, FS_DONE, FS_ERR, FS_N };
 // FS_ERR: 1 = bad V0, 2 = no admissible move, 3 = peer exchange timed out
 #define MAX_PEERS 16
+#define LNS_MAXPH 4
 
 struct SearchArgs {
     DevInst I;
@@ -105,6 +106,11 @@ struct SearchArgs {
     // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
     // search from the state in (vb, Y, fs).
     int32_t groups, R;
+    // batched schedule: phase q runs runs [phr0[q], phr0[q] + phR[q]) on phG[q] groups of phnb[q]
+    // CTAs (group g takes runs phr0 + g, phr0 + g + phG, ...); phase groups have their own exchange
+    // slots and until[] arrays (global group index phgb[q] + g), so no grid barrier separates phases
+    int32_t nph;
+    int32_t phG[LNS_MAXPH], phnb[LNS_MAXPH], phgb[LNS_MAXPH], phr0[LNS_MAXPH], phR[LNS_MAXPH];
     const int8_t *V0s;      // R x n
     int64_t *res;           // R x FS_N
     uint32_t *vouts;        // R x NWn
@@ -1224,18 +1230,29 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
-    const int G = A.groups > 0 ? A.groups : 1;
-    const int nb = (int)gridDim.x / G;
-    const int g = (int)blockIdx.x / nb, bid = (int)blockIdx.x - g * nb;
-    if (g >= G) return;
     const bool batch = A.R > 0;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
+    __shared__ unsigned long long *s_peers[MAX_PEERS];
+    __shared__ int s_xto;
+    if (threadIdx.x < A.npeers) s_peers[threadIdx.x] = A.peers[threadIdx.x];
+    if (threadIdx.x == 0) s_xto = 0;
+    __syncthreads();
+#ifdef LNS_PHASE_TIMING
+    if (threadIdx.x == 0) { for (int i = 0; i < NPH; i++) s_ph[i] = 0; s_last = clock64(); }
+#endif
+    for (int phq = 0; phq < (batch ? A.nph : 1); phq++) {
+    const int G = batch ? A.phG[phq] : 1;
+    const int nb = batch ? A.phnb[phq] : (int)gridDim.x;
+    const int g = (int)blockIdx.x / nb, bid = (int)blockIdx.x - g * nb;
+    if (g >= G) continue;  // idle in this phase
+    const int gg = batch ? A.phgb[phq] + g : 0;  // global group index: exchange slots, until[]
     const bool leader = (bid == 0 && threadIdx.x == 0);
-    unsigned long long *gslots = (unsigned long long *)A.slots + 64 * (size_t)g;
+    unsigned long long *gslots = (unsigned long long *)A.slots + 64 * (size_t)gg;
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, bid, nb, blo, bhi);
     // the CTA's until[] slice: shared-memory copy when it fits, else the group's global array
-    uint32_t *until = A.until + (batch ? (size_t)g * A.M : 0);
+    uint32_t *until = A.until + (batch ? (size_t)gg * A.M : 0);
     uint32_t ubase = 0;
     if (A.until_smem) {
         uint32_t *us = (uint32_t *)(sm + L.a_end);
@@ -1244,16 +1261,11 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         until = us;
         ubase = blo;
     }
-    const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
-    __shared__ unsigned long long *s_peers[MAX_PEERS];
-    __shared__ int s_xto;
-    if (threadIdx.x < A.npeers) s_peers[threadIdx.x] = A.peers[threadIdx.x];
-    if (threadIdx.x == 0) s_xto = 0;
-    __syncthreads();
     const uint2 *tri = nullptr;
     if (A.tri_smem) {
         uint2 *ts = (uint2 *)(sm + L.a_end + 4 * A.slice_cap);
         const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
+        __syncthreads();  // the previous phase's readers of the table are done
         for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) {
             int a, b, c;
             unrank_tab<K>(r, A.I.n, A.M, T2, T3, a, b, c);
@@ -1262,11 +1274,9 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         __syncthreads();
         tri = ts;
     }
-#ifdef LNS_PHASE_TIMING
-    if (threadIdx.x == 0) { for (int i = 0; i < NPH; i++) s_ph[i] = 0; s_last = clock64(); }
-#endif
-    unsigned long long tg = 0;  // iterations run by this group in this launch (exchange clock)
-    for (int rs = batch ? g : 0; rs < (batch ? A.R : 1); rs += G) {
+    unsigned long long tg = 0;  // iterations run by this group in this phase (exchange clock)
+    const int rbeg = batch ? A.phr0[phq] : 0, rend = batch ? A.phr0[phq] + A.phR[phq] : 1;
+    for (int rs = rbeg + (batch ? g : 0); rs < rend; rs += G) {
         int64_t f, best_f, best_it, zero_it, t0;
         if (batch) {
             init_restart<K>(A, Ar, A.V0s + (size_t)rs * A.I.n, sm, L, ps);
@@ -1444,6 +1454,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             }
         }
     }
+    }  // phases
 #ifdef LNS_PHASE_TIMING
     if (threadIdx.x == 0)
         for (int i = 0; i < NPH; i++) atomicAdd(&g_ph[i], (unsigned long long)s_ph[i]);
@@ -1865,6 +1876,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
     A.groups = 1; A.R = 0; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
+    A.nph = 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     A.peers = nullptr; A.npeers = 0; A.part = 0; A.nb_total = 0; A.timeout_ns = 0;
@@ -1990,25 +2002,26 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     return LNS_OK;
 }
 
-// Batched restarts: G groups of nb CTAs (cooperative grid G * nb); A carries V0s / res / vouts.
+// Batched restarts: the phases of A (cooperative grid = the SMs); A carries V0s / res / vouts.
 template <int K>
-lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int G, int nb, int64_t *gslots, cudaStream_t st)
+lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int grid, int ngroups, int nb_min,
+                        int64_t *gslots, cudaStream_t st)
 {
     const int budget = c->smemOptin - 1024;
     CK(allow_smem((const void *)k_search<K>, budget));
-    A.I.pad = pad_for(g, A.hi - A.lo, nb);
-    const size_t smem = cache_geometry(A, g, nb, budget);
-    if (!A.until_smem) {  // one global until[] per concurrent group
-        lns_status s = grow(c->d_until, c->until_cap, (size_t)G * g.M);
+    A.I.pad = pad_for(g, A.hi - A.lo, nb_min);
+    const size_t smem = cache_geometry(A, g, nb_min, budget);
+    if (!A.until_smem) {  // one global until[] per group of every phase
+        lns_status s = grow(c->d_until, c->until_cap, (size_t)ngroups * g.M);
         if (s != LNS_OK) return s;
         A.until = c->d_until;
     }
-    k_init_slots<<<(64 * G + 255) / 256, 256, 0, st>>>(gslots, G);
+    k_init_slots<<<(64 * ngroups + 255) / 256, 256, 0, st>>>(gslots, ngroups);
     A.slots = gslots;
-    A.groups = G;
+    A.groups = 0;
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
-    CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(G * nb), dim3(NT), args, smem, st));
+    CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(grid), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     return LNS_OK;
 }
@@ -2517,38 +2530,59 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
             vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
         }
     }
-    // groups: as many concurrent searches as SMs allow; CTAs per group = SMs / groups; a global
-    // until[] per group (when it is not cached in shared memory) is capped at 8 GiB
-    // choose G to minimise the makespan ceil(R/G) * T(SMs/G) with the iteration-time model
-    // T(nb) = (2 + 7.5e-4 m n) us + 1.63e-5 us * M (m + 32) / nb: a per-iteration cost of every
-    // CTA (plan build, exchange, move, per-thread run start-up; grows with m n) plus evaluation
-    // spread over nb SMs. Fitted on C2-C4 batches of 50 (nb = 2..14).
-    int G = 1;
-    {
-        double best = 1e300;
-        const double work = 1.63e-5 * (double)g.M * (double)(c->m + 32);
-        const double fixed = 2.0 + 7.5e-4 * (double)c->m * (double)c->n;
-        for (int q = 1; q <= std::min<int>(R, c->numSMs); q++) {
-            const int nbq = c->numSMs / q;
-            const double mk = (double)((R + q - 1) / q) * (fixed + work / nbq);
-            if (mk < best * 0.999) { best = mk; G = q; }
-        }
-    }
-    if (c->blocks_override > 0) G = std::min(R, std::max(1, c->numSMs / c->blocks_override));
+    // Schedule: up to two phases, k1 rounds of G1 concurrent searches on
+    // SMs / G1 CTAs each, then the R2 = R - k1 G1 remaining searches at once on SMs / R2 CTAs each,
+    // minimising the makespan under the iteration-time model
+    //   T(nb) = (2 + 7.5e-4 m n) us + 1.45e-5 us * M (m + 32) / nb
+    // (a per-iteration cost of every CTA: plan build, exchange, move; plus the evaluation spread
+    // over nb SMs; fitted on C2-C4 batches of 50, nb = 2..14). The second phase fills the SMs the
+    // rounds of the first would leave idle (50 searches on 148 SMs: 37 x 4 CTAs, then 13 x 11).
+    const int SMs = c->numSMs;
+    const double work = 1.45e-5 * (double)g.M * (double)(c->m + 32);
+    const double fixed = 2.0 + 7.5e-4 * (double)c->m * (double)c->n;
+    auto T = [&](int nbq) { return fixed + work / nbq; };
     const int budget = c->smemOptin - 1024;
+    // a global until[] per group (unless the slice fits in shared memory), capped at 8 GiB in total
     const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / (4LL * g.M));
-    for (;;) {
-        const int nb = c->numSMs / G;
-        const uint64_t slice = ((uint64_t)g.M + nb - 1) / nb + 64;
-        const bool cached = g.smem_eval + 4 * slice <= (size_t)budget;
-        if (cached || G <= cap_groups) break;
-        G = (int)cap_groups;
+    auto fits = [&](int groups, int nb_min) {
+        const uint64_t slice = ((uint64_t)g.M + nb_min - 1) / nb_min + 64;
+        return g.smem_eval + 4 * slice <= (size_t)budget || groups <= cap_groups;
+    };
+    int G1 = 1, k1 = R, R2 = 0;
+    if (c->blocks_override > 0) {
+        G1 = std::min(R, std::max(1, SMs / c->blocks_override));
+        k1 = (R + G1 - 1) / G1;
+    } else {
+        double best = 1e300;
+        for (int q = 1; q <= std::min<int>(R, SMs); q++) {
+            const int nbq = SMs / q;
+            for (int kq = R / q; kq >= 0; kq--) {
+                const int rem = R - kq * q;
+                if (rem > SMs) break;
+                const int nbr = rem > 0 ? SMs / rem : nbq;
+                if (!fits((kq > 0 ? q : 0) + rem, std::min(kq > 0 ? nbq : nbr, nbr))) continue;
+                const double mk = kq * T(nbq) + (rem > 0 ? T(nbr) : 0.0);
+                if (mk < best * 0.999) { best = mk; G1 = q; k1 = kq; R2 = rem; }
+            }
+        }
+        if (best >= 1e300) { G1 = 1; k1 = R; R2 = 0; }  // (only the 8 GiB cap can force this)
     }
-    const int nb = c->numSMs / G;
+    SearchArgs phases;
+    int nph = 0, ngroups = 0, grid = 0, nb_min = SMs, r0 = 0;
+    auto add_phase = [&](int Gq, int nbq, int Rq) {
+        phases.phG[nph] = Gq; phases.phnb[nph] = nbq; phases.phgb[nph] = ngroups;
+        phases.phr0[nph] = r0; phases.phR[nph] = Rq;
+        ngroups += Gq; grid = std::max(grid, Gq * nbq); nb_min = std::min(nb_min, nbq); r0 += Rq; nph++;
+    };
+    if (c->blocks_override > 0) add_phase(G1, std::min(c->blocks_override, SMs), R);
+    else {
+        if (k1 > 0) add_phase(G1, SMs / G1, k1 * G1);
+        if (R2 > 0) add_phase(R2, SMs / R2, R2);
+    }
     if ((s = grow(c->d_V0s, c->v0s_cap, hv.size())) != LNS_OK) return s;
     if ((s = grow(c->d_res, c->res_cap, (size_t)R * FS_N)) != LNS_OK) return s;
     if ((s = grow(c->d_vouts, c->vouts_cap, (size_t)R * c->NWn)) != LNS_OK) return s;
-    if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)G * 64)) != LNS_OK) return s;
+    if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)ngroups * 64)) != LNS_OK) return s;
     if ((s = grow(c->d_until, c->until_cap, std::max<size_t>(g.M, 1))) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
     const int savep = c->part, saven = c->nparts;
@@ -2557,10 +2591,15 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     c->part = savep; c->nparts = saven;
     A.R = R; A.V0s = c->d_V0s; A.res = c->d_res; A.vouts = c->d_vouts;
     A.trace_r = nullptr; A.trace_f = nullptr;
+    A.nph = nph;
+    for (int q = 0; q < nph; q++) {
+        A.phG[q] = phases.phG[q]; A.phnb[q] = phases.phnb[q]; A.phgb[q] = phases.phgb[q];
+        A.phr0[q] = phases.phr0[q]; A.phR[q] = phases.phR[q];
+    }
     switch (k) {
-    case 1: s = launch_batch<1>(c, A, g, G, nb, c->d_gslots, st); break;
-    case 2: s = launch_batch<2>(c, A, g, G, nb, c->d_gslots, st); break;
-    default: s = launch_batch<3>(c, A, g, G, nb, c->d_gslots, st); break;
+    case 1: s = launch_batch<1>(c, A, g, grid, ngroups, nb_min, c->d_gslots, st); break;
+    case 2: s = launch_batch<2>(c, A, g, grid, ngroups, nb_min, c->d_gslots, st); break;
+    default: s = launch_batch<3>(c, A, g, grid, ngroups, nb_min, c->d_gslots, st); break;
     }
     if (s != LNS_OK) return s;
     std::vector<int64_t> hres((size_t)R * FS_N);
