@@ -183,6 +183,11 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
 }
 
 struct PlanScalars {
+    // packed path, per walk q (set at the end of build_plan_pk): pkwk[q] = (X row-word base: shared
+    // byte address, or the word offset of the global X; first record address; end record address;
+    // address of pstart[first word + 1]); pkwt[q] = (initial window, trailing H bytes, trailing
+    // bin negative, last point)
+    uint4 pkwk[2], pkwt[2];
     int vmin, U, NB, P, ufirst;
     int fpen, fhd;  // block_fitness accumulators
     // linear regions: lattice points u < uneg are "deep negative" (all k+1
@@ -394,7 +399,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     // A. counting sort over the conservative lattice; holes; no record starts anywhere yet
     for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
     if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
-    for (int w = tid; w <= I.XW; w += NT) pstart[w] = INT_MAX;
+    for (int w = tid; w <= I.XW; w += NT) pstart[w] = -1;  // = 0xffffffff: no record (addresses, unsigned)
     __syncthreads();
     PH(0);
     // B. warp 0: exact range, cuts, and the placement in the order deep | walk 0 | walk 1 | top
@@ -474,8 +479,10 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     }
     __syncthreads();
     PH(1);
-    // C. place rows; emit the records (one thread per walked point); bin constants; deep constant
+    // C. place rows; emit the records (one thread per walked point); bin constants; deep constant.
+    //    pstart[w] = shared address of the first record in row word w
     const int vmin = ps.vmin, U = ps.U, NB = ps.NB, uf = ps.ufirst, uneg = ps.uneg, utop = ps.utop;
+    const uint32_t pk0 = (uint32_t)__cvta_generic_to_shared(pk);
     for (int j = tid; j < m; j += NT) {
         const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
         rowAt[p] = j;
@@ -500,7 +507,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         if (Lv == 0) {  // empty point: one zero record (in the previous row word) that completes its bin
             const int w = max(0, (st - 1) >> 5);
             pk[p] = make_uint4(0u, src, Hfin, wfin);
-            atomicMin(&pstart[w], p);
+            atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
             if (v - uneg < 2) ps.pkw0[v - uneg] = w;
             continue;
         }
@@ -510,7 +517,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
             const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
             const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
             pk[p] = w == w1 ? make_uint4(mask, src, Hfin, wfin) : make_uint4(mask, 0u, 0u, 0x4444u);
-            atomicMin(&pstart[w], p);
+            atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
         }
     }
     for (int v = tid; v < uneg; v += NT)  // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form)
@@ -527,7 +534,15 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     }
     __syncthreads();
     PH(2);
-    // D. X
+    if (tid < 2) {  // the walks' ready-to-use addresses and constants (read by pk_walk)
+        const int q = tid, wd = ps.pkw0[q];
+        const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
+        const uint32_t xb = XG ? (uint32_t)(wd * n) : (uint32_t)__cvta_generic_to_shared(X + wd * n);
+        ps.pkwk[q] = make_uint4(xb, pk0 + 16u * pb, pk0 + 16u * pe,
+                                (uint32_t)__cvta_generic_to_shared(pstart + wd + 1));
+        ps.pkwt[q] = make_uint4(ps.pkwin[q], ps.pkhtr[q], (uint32_t)ps.pktrl[q], (uint32_t)ps.pkz[q]);
+    }
+    // D. X (its closing barrier also publishes pkwk / pkwt)
     plan_transpose(I, Ar, sm, L, ps, X, Uc);
 }
 
@@ -843,31 +858,31 @@ __device__ __forceinline__ void pk_step(const uint4 &r, uint32_t lo, uint32_t hi
 // The K bins past a walk's last point hold only carried rows (bytes 0 .. K-1 of w; the rest are
 // 0): sum |h - H| is one SAD against the packed H, unless one of them is negative (w_b != 0).
 template <int K>
-__device__ __forceinline__ void pk_trail(const PlanScalars &ps, int q, const int2 *__restrict__ bins, uint32_t w, int &f)
+__device__ __forceinline__ void pk_trail(const uint4 &wt, const int2 *__restrict__ bins, uint32_t w, int &f)
 {
-    if (!ps.pktrl[q]) {
-        f += (int)__vsadu4(w, ps.pkhtr[q]);
+    if (!wt.z) {
+        f += (int)__vsadu4(w, wt.y);
         return;
     }
 #pragma unroll
     for (int i = 0; i < K; i++) {
         const int h = (int)((w >> (8 * i)) & 0xffu);
-        const int2 bn = bins[ps.pkz[q] + 2 * (i + 1)];
+        const int2 bn = bins[(int)wt.w + 2 * (i + 1)];
         f += bn.y * h + abs(h - bn.x);
     }
 }
 
-// Column words of row word xr: LDS when X is in shared memory (XG = false; a 32-bit shared
-// address), plain loads for the global-memory X of very large instances.
+// Column words of one row word: LDS from the 32-bit shared address xs (XG = false), or plain loads
+// from the global-memory X of very large instances (XG = true, xg).
 template <int K, bool XG>
-__device__ __forceinline__ void pk_planes(const uint32_t *__restrict__ Xg, uint32_t xs, int a, int b, int c,
+__device__ __forceinline__ void pk_planes(const uint32_t *__restrict__ xg, uint32_t xs, int a, int b, int c,
                                           uint32_t &lo, uint32_t &hi, uint32_t &lh)
 {
     uint32_t xa, xb = 0, xc = 0;
     if (XG) {
-        xa = Xg[a];
-        if (K >= 2) xb = Xg[b];
-        if (K == 3) xc = Xg[c];
+        xa = xg[a];
+        if (K >= 2) xb = xg[b];
+        if (K == 3) xc = xg[c];
     } else {
         asm("ld.shared.u32 %0, [%1];" : "=r"(xa) : "r"(xs + 4u * a));
         if (K >= 2) asm("ld.shared.u32 %0, [%1];" : "=r"(xb) : "r"(xs + 4u * b));
@@ -885,38 +900,42 @@ __device__ __forceinline__ void pk_planes(const uint32_t *__restrict__ Xg, uint3
 }
 
 // One walk q of NB neighbours (NB = 1 or 2, the second in a1, b1, c1): word-major (the lane's
-// column words are loaded once per row word), the record stream shared by the neighbours.
+// column words are loaded once per row word), the record stream shared by the neighbours. All
+// addresses are 32-bit shared-window addresses prepared by build_plan_pk (the asm loads read plan
+// memory that only changes across the plan's barriers, and every address derives from a fresh
+// load of pkwk, so no load can be reused across plans).
 template <int K, int NB, bool XG>
 __device__ __forceinline__ void pk_walk(const PlanScalars &ps, int q, const uint32_t *__restrict__ X,
-                                        const uint4 *__restrict__ pk, const int *__restrict__ pstart,
                                         const int2 *__restrict__ bins, int n, int a0, int b0, int c0, int a1, int b1,
                                         int c1, int &f0, int &f1)
 {
-    const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
-    if (pb == pe) return;
-    uint32_t w0 = ps.pkwin[q], w1 = w0;
-    const uint4 *pp = pk + pb;
-    const int wd = ps.pkw0[q];
-    const uint32_t *xg = XG ? X + wd * n : nullptr;
-    uint32_t xs = XG ? 0u : (uint32_t)__cvta_generic_to_shared(X + wd * n);
-    const int *pw = pstart + wd + 1;
+    const uint4 wk = ps.pkwk[q];
+    if (wk.y == wk.z) return;
+    const uint4 wt = ps.pkwt[q];
+    uint32_t w0 = wt.x, w1 = wt.x;
+    uint32_t pp = wk.y, pw = wk.w, xs = wk.x;
+    const uint32_t pe = wk.z;
+    const uint32_t *xg = XG ? X + wk.x : nullptr;
     for (;;) {
         uint32_t lo0, hi0, lh0, lo1 = 0, hi1 = 0, lh1 = 0;
         pk_planes<K, XG>(xg, xs, a0, b0, c0, lo0, hi0, lh0);
         if (NB == 2) pk_planes<K, XG>(xg, xs, a1, b1, c1, lo1, hi1, lh1);
         if (XG) xg += n; else xs += 4u * n;
-        const int pend = min(*pw++, pe);
-        const uint4 *pz = pk + pend;
+        uint32_t pend;
+        asm("ld.shared.u32 %0, [%1];" : "=r"(pend) : "r"(pw));
+        pw += 4u;
+        pend = min(pend, pe);
 #pragma unroll kPkUnroll
-        for (; pp < pz; ++pp) {
-            const uint4 r = *pp;
+        for (; pp < pend; pp += 16u) {
+            uint4 r;
+            asm("ld.shared.v4.u32 {%0, %1, %2, %3}, [%4];" : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "r"(pp));
             pk_step<K>(r, lo0, hi0, lh0, w0, f0);
             if (NB == 2) pk_step<K>(r, lo1, hi1, lh1, w1, f1);
         }
         if (pend == pe) break;
     }
-    pk_trail<K>(ps, q, bins, w0, f0);
-    if (NB == 2) pk_trail<K>(ps, q, bins, w1, f1);
+    pk_trail<K>(wt, bins, w0, f0);
+    if (NB == 2) pk_trail<K>(wt, bins, w1, f1);
 }
 
 // Deep rows (DEEP): every destination negative, cost cneg - 240 sum t (abs form).
@@ -941,8 +960,8 @@ __device__ __forceinline__ void eval_pk(const PlanScalars &ps, int cabs, const u
         f0 = pk_deep<K>(X, n, ps, f0, a0, b0, c0);
         if (NB == 2) f1 = pk_deep<K>(X, n, ps, f1, a1, b1, c1);
     }
-    pk_walk<K, NB, XG>(ps, 0, X, pk, pstart, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
-    pk_walk<K, NB, XG>(ps, 1, X, pk, pstart, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
+    pk_walk<K, NB, XG>(ps, 0, X, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
+    pk_walk<K, NB, XG>(ps, 1, X, bins, n, a0, b0, c0, a1, b1, c1, f0, f1);
 }
 
 // Evaluate ranks [blo, bhi) (blo 32-aligned) of this CTA at iteration t; returns this thread's best
