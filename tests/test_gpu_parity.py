@@ -350,6 +350,25 @@ def test_batched_restarts_grouped_kernel(L, orc, cfg, R, iters, stop):
         assert np.array_equal(Vo[r], oVo), r
 
 
+@pytest.mark.parametrize("cfg,R,iters", [("C4", 50, 12), ("C3", 50, 30), ("C2", 149, 40)])
+def test_batched_two_phase_schedule(L, orc, cfg, R, iters):
+    """The bench's job shape: the makespan model splits R searches into two phases with different
+    CTAs per search (C4/C3, 50 runs: one search on every SM, then 49 searches on 3 CTAs each;
+    C2, 149 runs: more searches than SMs). Sampled runs of both phases must equal the oracle."""
+    c = pi.CONFIGS[cfg]
+    inst = pi.config_instance(cfg)
+    seed = 99
+    ten = pi.default_tenure(inst.n, c["k"])
+    with L.Instance(inst.A, inst.S) as I:
+        Vo = np.empty((R, inst.n), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, c["k"], R, iters, -1, seed, None, 0, Vo)
+    for r in (0, 1, R // 2, R - 2, R - 1):
+        V0 = pi.start_vector(inst.n, pi.restart_seed(seed, r))
+        _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, c["k"], V0, iters, ten, stop_on_zero=False)
+        assert batch[r] == ores, r
+        assert np.array_equal(Vo[r], oVo), r
+
+
 def test_batched_restarts_given_start_vectors(L, orc):
     inst = pi.planted_instance(45, 37, 31)
     rng = np.random.default_rng(3)
