@@ -361,6 +361,44 @@ __device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t 
     PH(3);
 }
 
+// A pending move (the previous iteration's accepted flip set), applied by the next plan's step A
+// while it counts the rows: Y'_j = Y_j - 2 sum_{i in F} B_ji, B_ji = V_i A_ji;
+// thread 0 flips V's bits after step A's barrier (step D is the next reader of V).
+struct Move {
+    int on, a, b, c;
+};
+
+template <int K>
+__device__ __forceinline__ int move_delta(const uint32_t *__restrict__ ar, const uint32_t *__restrict__ vbs, const Move &mv)
+{
+    int d = (((ar[mv.a >> 5] ^ vbs[mv.a >> 5]) >> (mv.a & 31)) & 1u) ? -1 : 1;
+    if (K >= 2) d += (((ar[mv.b >> 5] ^ vbs[mv.b >> 5]) >> (mv.b & 31)) & 1u) ? -1 : 1;
+    if (K == 3) d += (((ar[mv.c >> 5] ^ vbs[mv.c >> 5]) >> (mv.c & 31)) & 1u) ? -1 : 1;
+    return d;
+}
+
+// Step A of both plan builders: apply the pending move to Y and count the rows per lattice point.
+template <int K>
+__device__ __forceinline__ void plan_count(const DevInst &I, const uint32_t *Ar, int *Ys, const uint32_t *vbs,
+                                           int *cnt, int vlo, const Move &mv)
+{
+    for (int j = threadIdx.x; j < I.m; j += NT) {
+        int y = Ys[j];
+        if (mv.on) {
+            y -= 2 * move_delta<K>(Ar + (size_t)j * I.NWn, vbs, mv);
+            Ys[j] = y;
+        }
+        atomicAdd(&cnt[(y - vlo) >> 1], 1);
+    }
+}
+
+__device__ __forceinline__ void flip_bits(uint32_t *vbs, int K, const Move &mv)
+{
+    vbs[mv.a >> 5] ^= 1u << (mv.a & 31);
+    if (K >= 2) vbs[mv.b >> 5] ^= 1u << (mv.b & 31);
+    if (K == 3) vbs[mv.c >> 5] ^= 1u << (mv.c & 31);
+}
+
 // ------------------------------------------------------------------------------------------
 // Plan of the packed path (m <= 255, every bin count fits a byte), DESIGN.md §5.9. A row at lattice
 // point u moves to bin u + 2t (t = #{i in F : x_ji = 1}), so bins of one parity of u only receive
@@ -379,7 +417,7 @@ __device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t 
 // ------------------------------------------------------------------------------------------
 template <int K, bool XG = false>
 __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
-                              uint32_t *Xarg)
+                              uint32_t *Xarg, const Move &mv)
 {
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
@@ -396,13 +434,14 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     int *pstart = (int *)(sm + L.pstart);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
-    // A. counting sort over the conservative lattice; holes; no record starts anywhere yet
-    for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
+    // A. pending move; counting sort over the conservative lattice; holes; no record starts yet
+    plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
     if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
     for (int w = tid; w <= I.XW; w += NT) pstart[w] = -1;  // = 0xffffffff: no record (addresses, unsigned)
     __syncthreads();
     PH(0);
     // B. warp 0: exact range, cuts, and the placement in the order deep | walk 0 | walk 1 | top
+    if (tid == 0 && mv.on) flip_bits((uint32_t *)(sm + L.vb), K, mv);
     if (warp == 0) {
         int uf = -1, ul = -1;
         for (int b0 = 0; b0 < Uc; b0 += 32) {
@@ -419,39 +458,74 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         int utop = ((I.maxS + 2 * K - vmin) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
         const int n0 = (utop - uneg + 1) >> 1, n1 = (utop - uneg) >> 1;  // points of walk 0 / 1
-        int pos = 0, rows = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0, prev = 0;
-        for (int q0 = 0; q0 < U; q0 += 32) {
-            const int q = q0 + lane;
-            const int v = q < uneg ? q : q < uneg + n0 ? uneg + 2 * (q - uneg)
-                        : q < utop ? uneg + 1 + 2 * (q - uneg - n0) : q;
-            const int Lq = q < U ? cnt[uf + v] : 0;
-            int myP = 0, myO = 0;
-            const int nv = min(32, U - q0);
-            for (int i = 0; i < nv; i++) {
-                const int Li = __shfl_sync(FULL, Lq, i);
-                const int qi = q0 + i;
-                const bool walk = qi >= uneg && qi < utop;
-                if (qi == uneg) rneg = rows;
-                if (qi == uneg + n0) { pkb1 = runp; prev = 0; }
-                if (qi == utop) rtop = rows;
-                if (walk && I.pad && Li > 0 && (pos & 31) != 0 && (pos & 31) + Li > 32) pos = (pos + 31) & ~31;
-                // an empty point whose bin and its predecessor's are non-negative is absorbed: the
-                // predecessor's final record completes both bins (no record of its own)
-                const bool nonneg = vmin + 2 * (__shfl_sync(FULL, v, i) - K) >= 0;
-                const bool absorbed = walk && Li == 0 && nonneg && prev == 2;
-                if (lane == i) { myP = pos; myO = absorbed ? -1 : runp; }
-                if (walk) {
-                    runp += Li > 0 ? ((pos + Li - 1) >> 5) - (pos >> 5) + 1 : (absorbed ? 0 : 1);
-                    prev = absorbed ? 1 : (nonneg ? 2 : 1);  // 2: a record that may absorb the next point
-                }
-                pos += Li;
-                rows += Li;
+        // the placement is sequential (padding depends on the position within the row word), so
+        // one thread walks the points: deep (contiguous), walk 0, walk 1 (padded), top (contiguous)
+        int pos = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0;
+        if (!I.pad) {
+            // unpadded: positions and record offsets are prefix sums (warp scans over the points in
+            // placement order); an empty point is absorbed only by a non-empty predecessor here
+            int sel = 0;  // lane holding q == uneg / uneg + n0 / utop: bits 0 / 1 / 2
+            for (int q0 = 0; q0 < U; q0 += 32) {
+                const int q = q0 + lane;
+                const bool valid = q < U;
+                const int v = q < uneg ? q : q < uneg + n0 ? uneg + 2 * (q - uneg)
+                            : q < utop ? uneg + 1 + 2 * (q - uneg - n0) : q;
+                const int Lq = valid ? cnt[uf + v] : 0;
+                const bool walk = valid && q >= uneg && q < utop;
+                const bool absorbed = walk && Lq == 0 && v - 2 >= uneg && vmin + 2 * (v - 2 - K) >= 0 &&
+                                      cnt[uf + v - 2] > 0;
+                int inc = Lq;
+                for (int o = 1; o < 32; o <<= 1) { const int t_ = __shfl_up_sync(FULL, inc, o); if (lane >= o) inc += t_; }
+                const int st = pos + inc - Lq, en = st + Lq;
+                const int np = walk ? (Lq > 0 ? ((en - 1) >> 5) - (st >> 5) + 1 : (absorbed ? 0 : 1)) : 0;
+                int incp = np;
+                for (int o = 1; o < 32; o <<= 1) { const int t_ = __shfl_up_sync(FULL, incp, o); if (lane >= o) incp += t_; }
+                const int p0 = runp + incp - np;
+                if (valid) { seg[v] = st; cur[uf + v] = st; pofs[v] = absorbed ? -1 : p0; }
+                if (q == uneg) { rneg = st; sel |= 1; }
+                if (q == uneg + n0) { pkb1 = p0; sel |= 2; }
+                if (q == utop) { rtop = st; sel |= 4; }
+                pos += __shfl_sync(FULL, inc, 31);
+                runp += __shfl_sync(FULL, incp, 31);
             }
-            if (q < U) { seg[v] = myP; cur[uf + v] = myP; pofs[v] = myO; }
+            // broadcast to lane 0 (the cuts at q = U take the totals)
+            const unsigned b1 = __ballot_sync(FULL, sel & 1), b2 = __ballot_sync(FULL, sel & 2), b4 = __ballot_sync(FULL, sel & 4);
+            rneg = b1 ? __shfl_sync(FULL, rneg, __ffs(b1) - 1) : pos;
+            pkb1 = b2 ? __shfl_sync(FULL, pkb1, __ffs(b2) - 1) : runp;
+            rtop = b4 ? __shfl_sync(FULL, rtop, __ffs(b4) - 1) : pos;
+        } else if (lane == 0) {
+            for (int v = 0; v < uneg; v++) {
+                const int Lv = cnt[uf + v];
+                seg[v] = pos; cur[uf + v] = pos; pofs[v] = 0;
+                pos += Lv;
+            }
+            rneg = pos;
+            int rows = pos;
+            for (int q = 0; q < 2; q++) {
+                if (q == 1) pkb1 = runp;
+                int prev = 0;  // 2: the previous point's record may absorb this one
+#pragma unroll 4
+                for (int v = uneg + q; v < utop; v += 2) {
+                    const int Lv = cnt[uf + v];
+                    if (I.pad && Lv > 0 && (pos & 31) != 0 && (pos & 31) + Lv > 32) pos = (pos + 31) & ~31;
+                    // an empty point whose bin and its predecessor's are non-negative is absorbed:
+                    // the predecessor's final record completes both bins (no record of its own)
+                    const bool nonneg = vmin + 2 * (v - K) >= 0;
+                    const bool absorbed = Lv == 0 && nonneg && prev == 2;
+                    seg[v] = pos; cur[uf + v] = pos; pofs[v] = absorbed ? -1 : runp;
+                    runp += Lv > 0 ? ((pos + Lv - 1) >> 5) - (pos >> 5) + 1 : (absorbed ? 0 : 1);
+                    prev = absorbed ? 1 : (nonneg ? 2 : 1);
+                    pos += Lv;
+                    rows += Lv;
+                }
+            }
+            rtop = rows;
+            for (int v = utop; v < U; v++) {
+                const int Lv = cnt[uf + v];
+                seg[v] = pos; cur[uf + v] = pos; pofs[v] = 0;
+                pos += Lv;
+            }
         }
-        if (uneg >= U) rneg = rows;
-        if (uneg + n0 >= U) pkb1 = runp;
-        if (utop >= U) rtop = rows;
         if (lane < 2) {  // walk p = lane: first / last point, initial window, trailing bins
             const int np = lane ? n1 : n0, a = uneg + lane, z = a + 2 * (np - 1);
             uint32_t win = 0, htr = 0;
@@ -562,9 +636,9 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
 // ------------------------------------------------------------------------------------------
 template <int K, bool XG = false>
 __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
-                           uint32_t *Xarg)
+                           uint32_t *Xarg, const Move &mv = Move{0, 0, 0, 0})
 {
-    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg); return; }
+    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv); return; }
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int m = I.m, n = I.n;
@@ -580,10 +654,11 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     int *pstart = (int *)(sm + L.pstart);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
-    // A. counting sort over the conservative lattice
-    for (int j = tid; j < m; j += NT) atomicAdd(&cnt[(Ys[j] - vlo) >> 1], 1);
+    // A. pending move; counting sort over the conservative lattice
+    plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
     __syncthreads();
     PH(0);
+    if (tid == 0 && mv.on) flip_bits((uint32_t *)(sm + L.vb), K, mv);
     // B. warp 0: exact range (first / last non-empty point), exclusive scans of the row and piece
     //    offsets over it, and the lattice of the next plan
     if (warp == 0) {
@@ -1310,10 +1385,11 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         }
         int64_t t = t0 + 1;
         bool failed = false;
+        Move mv{0, 0, 0, 0};  // accepted, not yet applied
         for (; t <= t0 + A.iters; t++) {
             if (A.stop_on_zero && f == 0) break;
-            if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
-            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr);
+            if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
+            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr, mv);
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
                                                   nullptr, tri, A.aspiration, (int)best_f)
@@ -1443,11 +1519,12 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             }
             if (f < best_f) { best_f = f; best_it = t; }  // every thread (aspiration needs it)
             if (f == 0 && zero_it < 0) zero_it = t;
-            int a, b, c;
-            unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), a, b, c);
-            apply_move<K>(A.I, Ar, Ys, vbs, a, b, c);
+            // the move is applied by the next plan's step A (or below, after the last iteration)
+            mv.on = 1;
+            unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), mv.a, mv.b, mv.c);
             PH(6);
         }
+        if (mv.on) apply_move<K>(A.I, Ar, Ys, vbs, mv.a, mv.b, mv.c);
         __syncthreads();  // the last move's V flip (thread 0) before V is written out / reused
         if (batch) {
             if (bid == 0) {
