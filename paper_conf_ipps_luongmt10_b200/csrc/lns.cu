@@ -654,8 +654,9 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     int *pstart = (int *)(sm + L.pstart);
     const int vlo = ps.vlo, Uc = ps.Uc;
 
-    // A. pending move; counting sort over the conservative lattice
+    // A. pending move; counting sort over the conservative lattice; holes of a padded placement
     plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
+    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
     __syncthreads();
     PH(0);
     if (tid == 0 && mv.on) flip_bits((uint32_t *)(sm + L.vb), K, mv);
@@ -692,8 +693,29 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         uneg = min(max(uneg, 0), U);
         int utop = ((I.maxS + 2 * K - vmin_) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
-        const int Wp = (m + 31) >> 5;
+        int Wp = (m + 31) >> 5;
         __syncwarp();
+        if (I.pad && lane == 0) {
+            // budgeted padded placement: a walked segment that would straddle a
+            // row word while starting mid-word starts at the next word, when the rows still to
+            // place fit in the XW words X has even if nothing else is padded (fewer pieces, so
+            // fewer POPCs per neighbour); deep rows stay contiguous at the front
+            int pos = 0, left = m;
+            runp = 0;
+            for (int v = 0; v < U; v++) {
+                const int Lv = cnt[uf + v];
+                if (v >= uneg && v < utop && Lv > 0 && (pos & 31) != 0 && (pos & 31) + Lv > 32) {
+                    const int np_ = (pos + 31) & ~31;
+                    if (((np_ + left + 31) >> 5) <= I.XW) pos = np_;
+                }
+                seg[v] = pos; cur[uf + v] = pos; pofs[v] = runp;
+                runp += Lv > 0 ? ((pos + Lv - 1) >> 5) - (pos >> 5) + 1 : 1;
+                pos += Lv;
+                left -= Lv;
+            }
+            runr = pos;
+            Wp = (pos + 31) >> 5;
+        }
         if (lane == 0) {
             const int vmin = vmin_;
             seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[Wp] = runp; ps.Wp = Wp;
@@ -1931,6 +1953,15 @@ lns_status check_k(lns_ctx *c, int k, Geometry &g)
         const Smem pwo = smem_layout(c->m, c->n, XWp, c->NWn, k, 0);
         if (pw.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 1; g.smem_eval = (size_t)pw.a_end; }
         else if (pwo.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 0; g.smem_eval = (size_t)pwo.a_end; }
+        if (g.pad) return LNS_OK;
+    }
+    if (c->m > PACKED_MAX_M && !c->no_pad) {
+        // segment-loop path: padded placement within the largest X (XW words, W < XW <= 2W + 1)
+        // that fits next to the plan (A from global memory)
+        for (int XWp = 2 * c->W + 1; XWp > c->W; XWp--) {
+            const Smem pwo = smem_layout(c->m, c->n, XWp, c->NWn, k, 0);
+            if (pwo.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 0; g.smem_eval = (size_t)pwo.a_end; break; }
+        }
         if (g.pad) return LNS_OK;
     }
     const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1);

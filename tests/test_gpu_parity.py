@@ -227,6 +227,22 @@ def test_trajectory_independent_of_grid_size(L, orc, blocks):
     assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
 
 
+@pytest.mark.parametrize("m,n,k,blocks,iters", [(300, 50, 3, 1, 25), (300, 50, 3, 3, 25), (400, 120, 2, 1, 30),
+                                                 (257, 64, 1, 1, 200)])
+def test_large_m_padded_placement_trajectory(L, orc, m, n, k, blocks, iters):
+    """m > 255 (segment-loop path) with large CTA slices: budgeted padded placement (DESIGN.md
+    §5.4). Random starts give deep-negative rows, empty lattice points and segments of every
+    size; the whole trajectory must equal the oracle's."""
+    inst = pi.planted_instance(m, n, 7000 + m + n + k)
+    V0 = pi.start_vector(n, 11 + k)
+    ten = pi.default_tenure(n, k)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0, iters, ten, stop_on_zero=False)
+    with L.Instance(inst.A, inst.S) as I:
+        L.lns_config(I.ctx, blocks)
+        tr, tf, Vo, res = I.tabu_run(k, iters, -1, V0=V0, stop_on_zero=False)
+    assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+
+
 @pytest.mark.parametrize("G", [2, 3, 8])
 def test_partitioned_search_emulated_on_one_gpu(L, orc, G):
     """The multi-GPU protocol (PAPER.md:448-454 partitioning): G contexts each own a slice of the
