@@ -562,3 +562,26 @@ def test_pool_recycles_context_buffers(L, orc):
     assert outs[2][0][1] == ores and np.array_equal(outs[2][1][1], oVo)
     L.lns_pool_trim()
     assert L.lns_pool_stats() == (0, 0)
+
+
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck"])
+def test_compute_sanitizer_clean(L, tool):
+    """every kernel family (persistent search with one and several CTAs,
+    batched restarts, stepped search, eval_all, the m > 255 path) runs clean under
+    compute-sanitizer on small instances."""
+    import os
+    import shutil
+    import subprocess
+    import sys
+
+    exe = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
+    if not os.path.exists(exe):
+        pytest.skip("compute-sanitizer not found")
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    cmd = [exe, "--tool", tool, "--error-exitcode", "9", sys.executable, os.path.join(root, "scripts", "sanitize_probe.py")]
+    out = subprocess.run(cmd, capture_output=True, text=True, timeout=900, cwd=root)
+    tail = (out.stdout + out.stderr)[-3000:]
+    assert out.returncode == 0, tail
+    assert "sanitize probe done" in out.stdout, tail
+    log = out.stdout + out.stderr
+    assert "ERROR SUMMARY: 0 errors" in log or "SUMMARY: 0 hazards displayed (0 errors" in log, tail
