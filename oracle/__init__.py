@@ -171,9 +171,11 @@ RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_ite
 
 
 def tabu_run(A, S, k: int, V0, iters: int, tenure: int, stop_on_zero: bool = True, nthreads: int = 0,
-             aspiration: bool = False):
+             aspiration: bool = False, tabu_solutions: bool = False):
     """Tabu search of PAPER.md:241-258. Returns (trace_rank, trace_fit, V_out, result dict).
-    aspiration: a tabu move is admissible when it beats the best fitness so far (variant R4')."""
+    aspiration: a tabu move is admissible when it beats the best fitness so far (variant R4').
+    tabu_solutions: the tabu list holds the `tenure` most recently visited solutions instead of
+    move ranks (variant R3', PAPER.md:243-244 read literally)."""
     A, S, m, n = _prep(A, S)
     V0 = np.ascontiguousarray(V0, dtype=np.int8)
     tr = np.full(max(iters, 1), -1, dtype=np.int64)
@@ -182,7 +184,8 @@ def tabu_run(A, S, k: int, V0, iters: int, tenure: int, stop_on_zero: bool = Tru
     res = np.zeros(6, dtype=np.int64)
     rc = _load().oracle_tabu_run(_p(A, _i8p), m, n, _p(S, _i32p), k, _p(V0, _i8p), iters,
                                  tenure, int(bool(stop_on_zero)), _p(tr, _i64p),
-                                 _p(tf, _i64p), _p(Vo, _i8p), _p(res, _i64p), nthreads, int(bool(aspiration)))
+                                 _p(tf, _i64p), _p(Vo, _i8p), _p(res, _i64p), nthreads,
+                                 int(bool(aspiration)) | (2 if tabu_solutions else 0))
     if rc == -2:
         raise ValueError("tenure >= C(n,k): no admissible move would remain")
     if rc != 0:

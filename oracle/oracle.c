@@ -225,9 +225,51 @@ typedef struct { int64_t f, r; } fr_t;
 
 static void flip(uint64_t *vb, int32_t i) { vb[i / 64] ^= 1ULL << (i % 64); }
 
+/* ---------------------------------------------------------------------------------------
+ * Solution list (variant R3', flag 2 of oracle_tabu_run): the tabu list of PAPER.md:243-244
+ * read literally -- "the solutions visited in the recent past". A plain open-addressing hash set
+ * of the listed solutions (bit vectors, compared word for word), rebuilt from the list every
+ * iteration.
+ * ------------------------------------------------------------------------------------- */
+typedef struct {
+    int32_t nw;              /* words per solution */
+    int64_t cap;             /* table slots (power of two) */
+    const uint64_t **slot;   /* pointer to a listed solution, or NULL */
+} solset_t;
+
+static uint64_t hash_words(const uint64_t *v, int32_t nw)
+{
+    uint64_t h = 0x9E3779B97F4A7C15ULL;
+    for (int32_t i = 0; i < nw; i++) {
+        h ^= v[i];
+        h *= 0xBF58476D1CE4E5B9ULL;
+        h ^= h >> 31;
+    }
+    return h;
+}
+
+static int solset_contains(const solset_t *S, const uint64_t *v)
+{
+    for (int64_t i = (int64_t)(hash_words(v, S->nw) & (uint64_t)(S->cap - 1));; i = (i + 1) & (S->cap - 1)) {
+        if (!S->slot[i]) return 0;
+        if (memcmp(S->slot[i], v, sizeof(uint64_t) * (size_t)S->nw) == 0) return 1;
+    }
+}
+
+static void solset_insert(solset_t *S, const uint64_t *v)
+{
+    int64_t i = (int64_t)(hash_words(v, S->nw) & (uint64_t)(S->cap - 1));
+    while (S->slot[i]) {
+        if (memcmp(S->slot[i], v, sizeof(uint64_t) * (size_t)S->nw) == 0) return; /* already listed */
+        i = (i + 1) & (S->cap - 1);
+    }
+    S->slot[i] = v;
+}
+
 static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k, int mode,
                                int64_t *f_all, const int32_t *until, int64_t t,
-                               const int64_t *sample, int64_t nsample, int nthreads, int64_t aspire_below)
+                               const int64_t *sample, int64_t nsample, int nthreads, int64_t aspire_below,
+                               const solset_t *sols)
 {
     int32_t n = P->n;
     int64_t *base = malloc(sizeof(int64_t) * (size_t)(n + 1));
@@ -260,12 +302,16 @@ static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k
                     if (mode == 2) {
                         if (q >= nsample || sample[q] != r) continue;
                     }
-                    const int tabu = (mode == 1 && until && !(until[r] < t));
+                    int tabu = (mode == 1 && until && !(until[r] < t));
                     if (tabu && aspire_below < 0) continue; /* tabu, no aspiration */
                     memcpy(vb, vb0, sizeof(uint64_t) * (size_t)P->nw);
                     flip(vb, i1);
                     if (k >= 2) flip(vb, i2);
                     if (k == 3) flip(vb, i3);
+                    if (mode == 1 && sols && solset_contains(sols, vb)) { /* V' is a listed solution */
+                        tabu = 1;
+                        if (aspire_below < 0) continue;
+                    }
                     int64_t f = fitness_packed(P, vb, Y, Hp);
                     /* aspiration (reading R4'): a tabu move is admissible if it beats the best
                      * fitness found so far */
@@ -294,7 +340,7 @@ int32_t oracle_eval_all(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    scan_neighbourhood(&P, vb, k, 0, f_all, NULL, 0, NULL, 0, nthreads, -1);
+    scan_neighbourhood(&P, vb, k, 0, f_all, NULL, 0, NULL, 0, nthreads, -1, NULL);
     free(vb); free_packed(&P);
     return 0;
 }
@@ -308,7 +354,7 @@ int32_t oracle_eval_ranks(const int8_t *A, int32_t m, int32_t n, const int32_t *
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    scan_neighbourhood(&P, vb, k, 2, f_out, NULL, 0, ranks, cnt, nthreads, -1);
+    scan_neighbourhood(&P, vb, k, 2, f_out, NULL, 0, ranks, cnt, nthreads, -1, NULL);
     free(vb); free_packed(&P);
     return 0;
 }
@@ -328,7 +374,7 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     pack_vector(V, n, vb);
-    fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, 1, NULL, 0, nthreads, -1);
+    fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, 1, NULL, 0, nthreads, -1, NULL);
     *best_f = b.f == INT64_MAX ? -1 : b.f;
     *best_r = b.r;
     free(vb); free_packed(&P); free(until);
@@ -341,8 +387,10 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
  * replaces the current solution.
  *   - tabu list: FIFO of the last L accepted move ranks (reading R3), implemented literally as
  *     until[r]: a rank accepted at iteration t is tabu for t+1 .. t+L;
- *   - no aspiration by default (reading R4); with aspiration != 0 a tabu move is admissible when
- *     it is better than the best fitness seen so far (Taillard's criterion, variant R4');
+ *   - no aspiration by default (reading R4); with flags & 1 a tabu move is admissible when it is
+ *     better than the best fitness seen so far (Taillard's criterion, variant R4');
+ *   - with flags & 2 the tabu list holds visited SOLUTIONS instead of move ranks (variant R3',
+ *     PAPER.md:243-244 read literally), see the solution set above;
  *     lowest rank wins ties (reading R5);
  *   - stop when f = 0 if stop_on_zero (checked before every iteration, also before t = 1),
  *     otherwise after `iters` iterations (reading R11).
@@ -351,23 +399,43 @@ int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S
 int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S, int32_t k,
                         const int8_t *V0, int64_t iters, int64_t L, int32_t stop_on_zero,
                         int64_t *trace_r, int64_t *trace_f, int8_t *V_out, int64_t *res,
-                        int32_t nthreads, int32_t aspiration)
+                        int32_t nthreads, int32_t flags)
 {
+    /* flags: 1 = aspiration (R4'), 2 = solution list (R3'): at iteration t the tabu list holds the
+     * L most recently visited solutions V_{t-L} .. V_{t-1} (V_0 = the start, V_{t-1} = the current
+     * solution, which is never a neighbour); a neighbour is tabu iff it equals one of them. */
+    const int aspiration = flags & 1, solutions = (flags & 2) != 0;
     if (k < 1 || k > 3 || n < k || m < 1 || iters < 0 || L < 0) return -1;
     int64_t M = oracle_neighborhood_size(n, k);
     if (L >= M) return -2;
+    if (solutions && L < 1) return -1;
     packed_t P;
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
     int32_t *Y = malloc(sizeof(int32_t) * (size_t)m);
     int32_t *Hp = malloc(sizeof(int32_t) * (size_t)(n + 1));
     int32_t *until = calloc((size_t)M, sizeof(int32_t)); /* until[r] = 0: admissible from t = 1 */
+    uint64_t *visited = NULL; /* V_s in slot s mod L */
+    solset_t sols = { P.nw, 0, NULL };
+    if (solutions) {
+        visited = malloc(sizeof(uint64_t) * (size_t)P.nw * (size_t)L);
+        sols.cap = 1;
+        while (sols.cap < 2 * L) sols.cap <<= 1;
+        sols.slot = malloc(sizeof(uint64_t *) * (size_t)sols.cap);
+    }
     pack_vector(V0, n, vb);
+    if (solutions) memcpy(visited, vb, sizeof(uint64_t) * (size_t)P.nw); /* V_0 */
     int64_t f = fitness_packed(&P, vb, Y, Hp);
     int64_t best_f = f, best_iter = 0, first_zero = (f == 0) ? 0 : -1, t;
     for (t = 1; t <= iters; t++) {
         if (stop_on_zero && f == 0) break;
-        fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, until, t, NULL, 0, nthreads, aspiration ? best_f : -1);
+        if (solutions) { /* the list of iteration t: V_s for max(0, t - L) <= s <= t - 1 */
+            memset(sols.slot, 0, sizeof(uint64_t *) * (size_t)sols.cap);
+            for (int64_t q = (t - L > 0 ? t - L : 0); q <= t - 1; q++)
+                solset_insert(&sols, visited + (size_t)(q % L) * (size_t)P.nw);
+        }
+        fr_t b = scan_neighbourhood(&P, vb, k, 1, NULL, solutions ? NULL : until, t, NULL, 0, nthreads,
+                                    aspiration ? best_f : -1, solutions ? &sols : NULL);
         if (b.r < 0) break; /* unreachable for L < M */
         /* apply: V <- V xor F_{r*}; flip set of r* found by walking the same nested loops */
         int32_t F[3];
@@ -375,6 +443,7 @@ int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
         for (int32_t q = 0; q < k; q++) flip(vb, F[q]);
         f = b.f;
         until[b.r] = (int32_t)(t + L);
+        if (solutions) memcpy(visited + (size_t)(t % L) * (size_t)P.nw, vb, sizeof(uint64_t) * (size_t)P.nw); /* V_t */
         if (trace_r) trace_r[t - 1] = b.r;
         if (trace_f) trace_f[t - 1] = b.f;
         if (f < best_f) { best_f = f; best_iter = t; }
@@ -385,7 +454,7 @@ int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
         for (int32_t i = 0; i < n; i++) V_out[i] = ((vb[i / 64] >> (i % 64)) & 1) ? -1 : 1;
     res[0] = done; res[1] = f; res[2] = best_f; res[3] = best_iter; res[4] = first_zero;
     res[5] = best_f == 0;
-    free(vb); free(Y); free(Hp); free(until); free_packed(&P);
+    free(vb); free(Y); free(Hp); free(until); free_packed(&P); free(visited); free(sols.slot);
     return 0;
 }
 

@@ -340,3 +340,48 @@ def test_tabu_aspiration_variant(orc, k, L):
     tr, tf, Vo, res = orc.tabu_run(I.A, I.S, k, V0, 50, L, stop_on_zero=False, aspiration=True)
     V = _check_tabu_trace(orc, I.A, I.S, k, V0, L, tr, tf, res, False, aspiration=True)
     assert np.array_equal(V, Vo)
+
+
+def _check_solution_tabu_trace(orc, A, S, k, V0, L, tr, tf, res, aspiration=False):
+    """Variant R3' (PAPER.md:243-244 read literally: "the tabu list contains the solutions ...
+    visited in the recent past"): at iteration t a neighbour is tabu iff its vector equals one of
+    the L most recently visited solutions V_{t-L} .. V_{t-1} (V_0 = the start). Re-derived here by
+    brute force on explicit +-1 vectors, not through the oracle's hash set."""
+    n = A.shape[1]
+    visited = [tuple(int(x) for x in V0)]
+    V = V0.copy()
+    best = orc.fitness(A, S, V)
+    flips = list(itertools.combinations(range(n), k))
+    for t in range(len(tr)):
+        recent = set(visited[max(0, len(visited) - L):])
+        fa = orc.eval_all(A, S, V, k)
+        tabu = np.array([tuple(int(x) for x in _flip(V, fs)) in recent for fs in flips])
+        if aspiration:
+            tabu &= ~(fa < best)
+        masked = np.where(tabu, np.iinfo(np.int64).max, fa)
+        assert tr[t] == int(np.argmin(masked)), t
+        assert tf[t] == fa[tr[t]]
+        V = _flip(V, flips[tr[t]])
+        visited.append(tuple(int(x) for x in V))
+        best = min(best, int(tf[t]))
+    assert res["iters_done"] == len(tr) and res["best_f"] == best
+    return V
+
+
+@pytest.mark.parametrize("k,L,aspiration", [(1, 3, False), (1, 8, False), (2, 25, False), (3, 40, False),
+                                            (2, 25, True), (1, 1, False)])
+def test_tabu_solution_list_variant(orc, k, L, aspiration):
+    I = pi.planted_instance(15, 16, 1200 + k + L)
+    V0 = pi.start_vector(16, 70 + k)
+    tr, tf, Vo, res = orc.tabu_run(I.A, I.S, k, V0, 45, L, stop_on_zero=False, aspiration=aspiration,
+                                   tabu_solutions=True)
+    V = _check_solution_tabu_trace(orc, I.A, I.S, k, V0, L, tr, tf, res, aspiration)
+    assert np.array_equal(V, Vo)
+    if not aspiration and L > 1:  # no solution revisited while listed
+        seen = [tuple(V0)]
+        Vc = V0.copy()
+        for t in range(len(tr)):
+            (fs,) = orc.flipsets(16, k, [tr[t]])
+            Vc = _flip(Vc, fs)
+            assert tuple(Vc) not in set(seen[max(0, len(seen) - L):])
+            seen.append(tuple(Vc))
