@@ -56,6 +56,12 @@ typedef int32_t lns_status;
 #define LNS_FORCE_STEPPED 2     /* run one launch sequence per iteration instead of the persistent kernel */
 #define LNS_ASPIRATION 4        /* variant (not the default, reading R4'): a tabu move is admissible when its
                                    fitness is below the best fitness found so far (Taillard [11]) */
+#define LNS_TABU_SOLUTIONS 16   /* variant (not the default, reading R3'): the tabu list holds the `tenure`
+                                   most recently visited SOLUTIONS V_{t-L} .. V_{t-1} (PAPER.md:243-244 read
+                                   literally), not move ranks; a neighbour is tabu iff it equals one of
+                                   them. lns_tabu_run (persistent kernel, also with peers) and
+                                   lns_tabu_run_batch only; tenure >= 1. The visited ring costs tenure x
+                                   ceil(n/32) x 4 bytes of device memory per concurrent search. */
 #define LNS_PLAIN_LAUNCH 8      /* lns_tabu_run: launch the persistent kernel with a plain launch instead of
                                    a cooperative one. The driver serialises cooperative launches, so several
                                    peer partitions on ONE device (tests, emulation) need this; co-residency

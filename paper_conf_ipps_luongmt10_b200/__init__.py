@@ -30,6 +30,7 @@ LNS_EPEER = -7
 LNS_STOP_ON_ZERO = 1
 LNS_FORCE_STEPPED = 2
 LNS_ASPIRATION = 4
+LNS_TABU_SOLUTIONS = 16
 LNS_PLAIN_LAUNCH = 8
 KEY_NONE = (1 << 63) - 1
 LNS_IPC_HANDLE_BYTES = 64

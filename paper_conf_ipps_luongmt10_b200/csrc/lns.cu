@@ -101,7 +101,9 @@ struct SearchArgs {
     int32_t tri_smem;       // cache the flip sets of the CTA's slice in shared memory (1 = yes)
     int32_t slice_cap;      // capacity (ranks) of the per-CTA shared caches
     int32_t aspiration;     // a tabu move is admissible when it beats the best fitness so far
-    uint32_t *Xg;           // non-null: X lives in global memory, XW * n words per CTA (large m x n)
+    int32_t sol_list;       // LNS_TABU_SOLUTIONS (reading R3'): the tabu list holds visited solutions
+    uint32_t *ring;         // sol_list: V_s in slot s mod L, L x NWn words per group (group gg at gg L NWn)
+    uint32_t *Xg;          // non-null: X lives in global memory, XW * n words per CTA (large m x n)
     // batched restarts (lns_tabu_run_batch): the grid is split into `groups` groups of CTAs; group g
     // runs restarts g, g + groups, ... each from V0s[r] and writes res[r] / vouts[r]. R = 0: one
     // search from the state in (vb, Y, fs).
@@ -1283,6 +1285,61 @@ __device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, co
     return Ar;
 }
 
+// Variant R3' (LNS_TABU_SOLUTIONS; PAPER.md:243-244 read literally, "the tabu list contains the
+// solutions that have been visited in the recent past"): at iteration t the list holds
+// V_{t-L} .. V_{t-1}. A neighbour V xor F equals a listed W iff F = V xor W, i.e. iff W differs
+// from V in exactly k positions, and then F is those positions: each listed W marks at most one
+// rank. The group's CTAs share the list (ring slot s mod L holds V_s); every CTA scans a strided
+// share of it against vbs = V_{t-1} and writes until[rank] = t for the ranks of this device's
+// slice (tabu at t, admissible again at t + 1: nothing to clear). CTA 0 stores V_{t-1} into its
+// slot first (it is not among the listed entries scanned at t). A group barrier (arrival counter
+// bar, monotonic, nb arrivals per pass) then publishes until[] before the evaluation reads it.
+template <int K>
+__device__ void sol_tabu(const SearchArgs &A, const unsigned char *sm, const Smem &L, const uint32_t *vbs,
+                         uint32_t *ring, uint32_t *until, int64_t t, int bid, int nb, unsigned long long *bar,
+                         unsigned long long &tb)
+{
+    const int NW = A.I.NWn, n = A.I.n;
+    const int64_t Lt = A.L;
+    const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
+    __syncthreads();  // vbs = V_{t-1}: the previous move was applied by the plan
+    const int64_t skip = (t - 1) % Lt;  // slot of V_{t-1} (held V_{t-1-L}, no longer listed)
+    if (bid == 0)
+        for (int w = threadIdx.x; w < NW; w += NT) ring[(size_t)skip * NW + w] = vbs[w];
+    // listed besides V_{t-1}: V_s, max(0, t-L) <= s <= t-2, i.e. every slot but `skip` once the
+    // ring has wrapped, else slots 0 .. t-2
+    const int64_t nlisted = min(t - 1, Lt - 1);
+    for (int64_t j = (int64_t)bid * NT + threadIdx.x; j < nlisted; j += (int64_t)nb * NT) {
+        const uint32_t *w = ring + (size_t)(j < skip ? j : j + 1) * NW;
+        int d = 0;
+        for (int q = 0; q < NW; q++) d += __popc(__ldcg(w + q) ^ vbs[q]);
+        if (d != K) continue;
+        int f[3] = {0, 0, 0}, cnt = 0;
+        for (int q = 0; q < NW && cnt < K; q++)
+            for (uint32_t x = __ldcg(w + q) ^ vbs[q]; x && cnt < K; x &= x - 1) f[cnt++] = 32 * q + __ffs(x) - 1;
+        uint32_t r;
+        if (K == 1) r = (uint32_t)f[0];
+        else if (K == 2) r = A.M - 1u - (T2[n - 1 - f[0]] + (uint32_t)(n - 1 - f[1]));
+        else r = A.M - 1u - (T3[n - 1 - f[0]] + T2[n - 1 - f[1]] + (uint32_t)(n - 1 - f[2]));
+        if (r >= A.lo && r < A.hi) until[r] = (uint32_t)t;
+    }
+    if (nb > 1) {
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            tb++;
+            __threadfence();
+            asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(bar) : "memory");
+            const unsigned long long target = (unsigned long long)nb * tb;
+            unsigned long long seen;
+            do {
+                asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(bar) : "memory");
+            } while (seen < target);
+            __threadfence();
+        }
+    }
+    __syncthreads();
+}
+
 // ------------------------------------------------------------------------------------------
 // Kernels
 // ------------------------------------------------------------------------------------------
@@ -1391,6 +1448,8 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         tri = ts;
     }
     unsigned long long tg = 0;  // iterations run by this group in this phase (exchange clock)
+    unsigned long long tb = 0;  // solution-list barrier passes (LNS_TABU_SOLUTIONS)
+    uint32_t *ring = A.sol_list ? A.ring + (size_t)gg * (size_t)A.L * A.I.NWn : nullptr;
     const int rbeg = batch ? A.phr0[phq] : 0, rend = batch ? A.phr0[phq] + A.phR[phq] : 1;
     for (int rs = rbeg + (batch ? g : 0); rs < rend; rs += G) {
         int64_t f, best_f, best_it, zero_it, t0;
@@ -1412,6 +1471,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (A.stop_on_zero && f == 0) break;
             if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
             else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr, mv);
+            if (A.sol_list) sol_tabu<K>(A, sm, L, vbs, ring, until, t, bid, nb, gslots + 24, tb);
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
                                                   nullptr, tri, A.aspiration, (int)best_f)
@@ -1534,7 +1594,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
             const uint32_t r = (uint32_t)(key & 0xffffffffu);
             f = (int64_t)(key >> 32);
-            if (threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
+            if (!A.sol_list && threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
             if (leader) {
                 if (A.trace_r) A.trace_r[t - 1] = r;
                 if (A.trace_f) A.trace_f[t - 1] = f;
@@ -1712,7 +1772,7 @@ __global__ void k_init_slots(int64_t *slots, int G)
 {
     for (int i = blockIdx.x * blockDim.x + threadIdx.x; i < 64 * G; i += gridDim.x * blockDim.x) {
         const int q = i & 63;
-        slots[i] = q < 48 ? KEY_NONE : 0;
+        slots[i] = (q < 48 && q != 24) ? KEY_NONE : 0;  // q = 24: solution-list barrier counter
     }
 }
 
@@ -1764,6 +1824,7 @@ struct lns_ctx {
     uint32_t *d_vouts = nullptr; size_t vouts_cap = 0;
     int64_t *d_gslots = nullptr; size_t gslots_cap = 0;
     uint32_t *d_X = nullptr; size_t X_cap = 0;                // global X fallback (per CTA)
+    uint32_t *d_ring = nullptr; size_t ring_cap = 0;          // LNS_TABU_SOLUTIONS: visited solutions
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
     double last_ms = 0.0;
     // stepped search
@@ -1999,6 +2060,8 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
     A.iters = iters; A.L = L; A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
+    A.sol_list = (flags & LNS_TABU_SOLUTIONS) ? 1 : 0;
+    A.ring = c->d_ring;
     A.Xg = g.x_global ? c->d_X : nullptr;
     A.a_in_smem = g.a_in_smem;
     A.until_smem = 0; A.tri_smem = 0; A.slice_cap = 0;
@@ -2071,6 +2134,10 @@ size_t cache_geometry(SearchArgs &A, const Geometry &g, int nb, int budget)
     size_t smem = g.smem_eval;
     A.slice_cap = (int32_t)std::min<uint64_t>(slice, 1u << 30);
     A.until_smem = 0; A.tri_smem = 0;
+    if (A.sol_list) {  // until[] stays in global memory: every CTA of the group writes into it
+        if (g.smem_eval + 12 * slice <= (size_t)budget) { A.tri_smem = 1; smem = g.smem_eval + 12 * slice; }
+        return smem;
+    }
     if (g.smem_eval + 12 * slice <= (size_t)budget) {  // until[] slice + flip-set table
         A.until_smem = 1; A.tri_smem = 1;
         smem = g.smem_eval + 12 * slice;
@@ -2338,7 +2405,7 @@ void lns_destroy(lns_ctx *c)
     for (void *p : {(void *)c->d_Arow, (void *)c->d_H, (void *)c->d_vb, (void *)c->d_Y, (void *)c->d_fs,
                     (void *)c->d_slots, (void *)c->d_counter, (void *)c->d_V, (void *)c->d_Yin, (void *)c->d_bits,
                     (void *)c->d_until, (void *)c->d_tr, (void *)c->d_tf, (void *)c->d_fit, (void *)c->d_V0s,
-                    (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X})
+                    (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X, (void *)c->d_ring})
         pool_free(p);
     for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
     cudaFree(c->d_xbuf); cudaFree(c->d_peers);
@@ -2540,6 +2607,7 @@ lns_status lns_step_begin(lns_ctx *c, int32_t k, int64_t max_iters, int64_t tenu
     if (max_iters < 0) return fail(LNS_EINVAL, "iters < 0");
     int64_t L;
     if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
+    if (flags & LNS_TABU_SOLUTIONS) return fail(LNS_EINVAL, "LNS_TABU_SOLUTIONS needs the persistent kernel (lns_tabu_run)");
     DeviceGuard dg(c->device);
     if ((s = search_setup(c, g, max_iters, seed, V0, (cudaStream_t)stream)) != LNS_OK) return s;
     c->step_active = true; c->step_K = k; c->step_iters = max_iters; c->step_L = L; c->step_flags = flags;
@@ -2588,8 +2656,13 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     int64_t L;
     if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
     if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    const bool sols = (flags & LNS_TABU_SOLUTIONS) != 0;
+    if (sols && L < 1) return fail(LNS_EINVAL, "LNS_TABU_SOLUTIONS needs tenure >= 1");
+    if (sols && c->npeers == 0 && (c->comm != nullptr || c->nparts > 1 || (flags & LNS_FORCE_STEPPED)))
+        return fail(LNS_EINVAL, "LNS_TABU_SOLUTIONS needs the persistent kernel (no stepped / NCCL path)");
     DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
+    if (sols && (s = grow(c->d_ring, c->ring_cap, (size_t)L * c->NWn)) != LNS_OK) return s;
     if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
     SearchArgs A = make_args(c, g, iters, L, flags);
     if (c->npeers > 0) {
@@ -2641,6 +2714,8 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     int64_t L;
     if ((s = resolve_tenure(g.M, tenure, L)) != LNS_OK) return s;
     if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    const bool sols = (flags & LNS_TABU_SOLUTIONS) != 0;
+    if (sols && L < 1) return fail(LNS_EINVAL, "LNS_TABU_SOLUTIONS needs tenure >= 1");
     if (R == 0) return LNS_OK;
     DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
@@ -2671,7 +2746,10 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     const int budget = c->smemOptin - 1024;
     // a global until[] per group (unless the slice fits in shared memory), capped at 8 GiB in total
     const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / (4LL * g.M));
+    // LNS_TABU_SOLUTIONS: a global until[] and a visited ring per group, 8 GiB in total at most
+    const int64_t cap_sol = std::max<int64_t>(1, (8LL << 30) / (4LL * ((int64_t)g.M + L * c->NWn)));
     auto fits = [&](int groups, int nb_min) {
+        if (sols) return groups <= cap_sol;
         const uint64_t slice = ((uint64_t)g.M + nb_min - 1) / nb_min + 64;
         return g.smem_eval + 4 * slice <= (size_t)budget || groups <= cap_groups;
     };
@@ -2710,6 +2788,7 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     if ((s = grow(c->d_res, c->res_cap, (size_t)R * FS_N)) != LNS_OK) return s;
     if ((s = grow(c->d_vouts, c->vouts_cap, (size_t)R * c->NWn)) != LNS_OK) return s;
     if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)ngroups * 64)) != LNS_OK) return s;
+    if (sols && (s = grow(c->d_ring, c->ring_cap, (size_t)ngroups * L * c->NWn)) != LNS_OK) return s;
     if ((s = grow(c->d_until, c->until_cap, std::max<size_t>(g.M, 1))) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
     const int savep = c->part, saven = c->nparts;
@@ -2717,6 +2796,7 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     SearchArgs A = make_args(c, g, iters, L, flags);
     c->part = savep; c->nparts = saven;
     A.R = R; A.V0s = c->d_V0s; A.res = c->d_res; A.vouts = c->d_vouts;
+    A.ring = c->d_ring;
     A.trace_r = nullptr; A.trace_f = nullptr;
     A.nph = nph;
     for (int q = 0; q < nph; q++) {

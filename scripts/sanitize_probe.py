@@ -23,6 +23,8 @@ try:
     L.lns_tabu_run(ctx, 3, 6, -1, 1, None, 0)
     L.lns_tabu_run(ctx, 2, 6, -1, 1, None, L.LNS_FORCE_STEPPED)
     L.lns_tabu_run_batch(ctx, 3, 3, 4, -1, 7, None, 0)
+    L.lns_tabu_run(ctx, 2, 8, 3, 1, None, L.LNS_TABU_SOLUTIONS)  # solution list: scan + group barrier
+    L.lns_tabu_run_batch(ctx, 1, 2, 8, 2, 7, None, L.LNS_TABU_SOLUTIONS)
 finally:
     L.lns_destroy(ctx)
 big = pi.planted_instance(260, 40, 5)  # m > 255: segment-loop path, padded placement

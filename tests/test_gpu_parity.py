@@ -412,6 +412,54 @@ def test_aspiration_variant_bit_exact(L, orc, k, L_ten, iters):
         assert batch[0] == ores and np.array_equal(Vb[0], oVo)
 
 
+@pytest.mark.parametrize("k,L_ten,iters,blocks", [(1, 4, 200, 1), (1, 30, 200, 3), (2, 1, 120, 2), (2, 50, 150, 5),
+                                                  (3, 7, 80, 4), (3, -1, 60, 148)])
+@pytest.mark.parametrize("aspiration", [False, True])
+def test_solution_list_variant_bit_exact(L, orc, k, L_ten, iters, blocks, aspiration):
+    """LNS_TABU_SOLUTIONS (variant R3', PAPER.md:243-244 read literally): the tabu list holds the
+    L most recently visited solutions. Persistent kernel on 1..148 CTAs (the group barrier that
+    publishes the scanned ranks) and batched restarts, against the oracle's hash-set variant.
+    Short tenures wrap the visited ring many times."""
+    inst = pi.planted_instance(41, 35, 900 + k)
+    V0 = pi.start_vector(35, 80 + k)
+    ten = pi.default_tenure(35, k) if L_ten < 0 else L_ten
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0, iters, ten, stop_on_zero=False,
+                                       aspiration=aspiration, tabu_solutions=True)
+    flags = L.LNS_TABU_SOLUTIONS | (L.LNS_ASPIRATION if aspiration else 0)
+    with L.Instance(inst.A, inst.S) as I:
+        L.lns_config(I.ctx, blocks)
+        tr, tf, Vo, res = I.tabu_run(k, iters, L_ten, V0=V0, stop_on_zero=False, flags=flags)
+        assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+        L.lns_config(I.ctx, 0)
+        Vb = np.empty((3, 35), np.int8)
+        V0s = np.stack([V0, pi.start_vector(35, 1), pi.start_vector(35, 2)])
+        batch = L.lns_tabu_run_batch(I.ctx, k, 3, iters, L_ten, 0, V0s, flags, Vb)
+    assert batch[0] == ores and np.array_equal(Vb[0], oVo)
+    for r in (1, 2):
+        _, _, oV, orr = orc.tabu_run(inst.A, inst.S, k, V0s[r], iters, ten, stop_on_zero=False,
+                                     aspiration=aspiration, tabu_solutions=True)
+        assert batch[r] == orr and np.array_equal(Vb[r], oV)
+
+
+def test_solution_list_variant_C3_and_errors(L, orc):
+    """C3 shape (85,320 neighbours, 148 CTAs, the flip-set cache) with the solution list of the
+    paper's size L = C(n,3)/6, and the argument errors: tenure 0, the stepped path."""
+    inst = pi.config_instance("C3")
+    V0 = pi.start_vector(81, 3)
+    ten = pi.default_tenure(81, 3)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0, 40, ten, stop_on_zero=False, tabu_solutions=True)
+    with L.Instance(inst.A, inst.S) as I:
+        tr, tf, Vo, res = I.tabu_run(3, 40, -1, V0=V0, stop_on_zero=False, flags=L.LNS_TABU_SOLUTIONS)
+        assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+        for ten_bad, fl in ((0, L.LNS_TABU_SOLUTIONS), (5, L.LNS_TABU_SOLUTIONS | L.LNS_FORCE_STEPPED)):
+            with pytest.raises(L.LnsError) as ei:
+                I.tabu_run(3, 5, ten_bad, V0=V0, stop_on_zero=False, flags=fl)
+            assert ei.value.status == L.LNS_EINVAL
+        with pytest.raises(L.LnsError) as ei:
+            L.lns_step_begin(I.ctx, 3, 5, 5, 0, V0, L.LNS_TABU_SOLUTIONS)
+        assert ei.value.status == L.LNS_EINVAL
+
+
 @pytest.mark.parametrize("k", [1, 2])
 def test_large_instance_global_X_fallback(L, orc, k):
     """1201 x 1217 (the Fig. 8 ladder): the sorted sign bits X no longer fit in
@@ -459,8 +507,9 @@ def _peer_pair(L, inst, nb):
     return ctxs, bufs
 
 
-@pytest.mark.parametrize("cfg,iters", [("C4", 120), ("C3", 300), ("C2", 400)])
-def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters):
+@pytest.mark.parametrize("cfg,iters,sols", [("C4", 120, False), ("C3", 300, False), ("C2", 400, False),
+                                           ("C3", 150, True)])
+def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters, sols):
     """two partitions, each a persistent kernel of 32 CTAs on its own stream,
     exchange the per-iteration MIN through each other's exchange buffers (red.min.sys /
     red.release.sys / ld.acquire.sys) with no host step. Both must reproduce the single-context
@@ -474,11 +523,12 @@ def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters):
     inst = pi.config_instance(cfg)
     k, n = c["k"], inst.n
     V0 = pi.start_vector(n, pi.config_seed(cfg))
+    fl = L.LNS_TABU_SOLUTIONS if sols else 0  # the solution list (R3') is scanned per partition
     ref = L.lns_create(inst.A, inst.S)
     try:
         tr0, tf0 = np.zeros(iters, np.int64), np.zeros(iters, np.int64)
         v0 = np.zeros(n, np.int8)
-        r0 = L.lns_tabu_run(ref, k, iters, -1, 0, V0, 0, v0, tr0, tf0)
+        r0 = L.lns_tabu_run(ref, k, iters, -1, 0, V0, fl, v0, tr0, tf0)
     finally:
         L.lns_destroy(ref)
     ctxs, bufs = _peer_pair(L, inst, 32)
@@ -486,7 +536,7 @@ def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters):
         # a plain run first: every buffer the run needs is allocated now (cudaMalloc synchronises
         # the device, which would serialise the two partitions' kernels in one process)
         for cx in ctxs:
-            L.lns_tabu_run(cx, k, iters, -1, 0, V0, 0)
+            L.lns_tabu_run(cx, k, iters, -1, 0, V0, fl)
         for p, cx in enumerate(ctxs):
             L.lns_attach_peers(cx, p, 2, bufs, 20000)
         for cx in ctxs:
@@ -499,7 +549,7 @@ def test_peer_exchange_two_partitions_one_gpu(L, cfg, iters):
         def run(p):
             try:
                 o = outs[p]
-                o["res"] = L.lns_tabu_run(ctxs[p], k, iters, -1, 0, V0, L.LNS_PLAIN_LAUNCH, o["v"], o["tr"], o["tf"],
+                o["res"] = L.lns_tabu_run(ctxs[p], k, iters, -1, 0, V0, L.LNS_PLAIN_LAUNCH | fl, o["v"], o["tr"], o["tf"],
                                           streams[p])
             except Exception as e:  # noqa: BLE001 - reported below
                 errs[p] = e
