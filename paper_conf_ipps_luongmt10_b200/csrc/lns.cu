@@ -81,6 +81,7 @@ struct DevInst {
     const uint32_t *Arow;  // m x NWn, bit (i%32) of word i/32 = 1 <=> A[j][i] = -1
     const int32_t *H;      // n+1 bins of S
     int32_t maxS;          // largest b with H_b > 0
+    int32_t pkw;           // m > 255: the packed (byte-window) plan is tried per iteration
 };
 
 // fstate layout (int64): current f, iterations done, best f, best iter, first zero iter, done, error
@@ -158,7 +159,8 @@ constexpr int kPkUnroll = PK_UNROLL;  // unroll of the packed piece loop
 #endif
 
 // XW = row words of X (I.XW: W, or 2W + 1 with padded placement)
-__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0)
+__host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K, int a_in_smem, int x_global = 0,
+                                            int pkw = 0)
 {
     Smem s;
     int o = 0;
@@ -173,7 +175,7 @@ __host__ __device__ inline Smem smem_layout(int m, int n, int W, int NWn, int K,
     s.rowAt = o;  o = align16(o + 4 * (m > 32 * W ? m : 32 * W));  // row slots (holes = -1 when padded)
     s.bins = o;   o = align16(o + 8 * (n + 1 + 2 * K));  // NB = U + 2K bins
     s.pieces = o; o = align16(o + 8 * (n + 2 + W));      // P <= U + W - 1 pieces (+1 prefetch pad)
-    s.pk = o;     o = align16(o + (m <= PACKED_MAX_M ? 16 * (n + 2 + W) : 0));  // packed-path pieces
+    s.pk = o;     o = align16(o + ((m <= PACKED_MAX_M || pkw) ? 16 * (n + 2 + W) : 0));  // packed-path records
     s.pstart = o; o = align16(o + 4 * (W + 1));
     s.T2 = o;     o = align16(o + 4 * n);                // C(y,2), y < n (u32)
     s.T3 = o;     o = align16(o + 4 * n);                // C(z,3), z < n (u32: C(n,3) < 2^32)
@@ -198,6 +200,7 @@ struct PlanScalars {
     int uneg, utop, rneg, cneg;
     // packed path (abs form): sum of H_b over the walked bins
     int hwalk;
+    int pkok;  // this plan is the packed one (always for m <= 255; per iteration for m > 255, §5.11)
     int Wp;    // row words X holds this plan (ceil(row slots / 32); padded slots are holes)
     int rtop;  // rows below the top cut (points < utop), unpadded
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
@@ -419,7 +422,7 @@ __device__ __forceinline__ void flip_bits(uint32_t *vbs, int K, const Move &mv)
 // ------------------------------------------------------------------------------------------
 template <int K, bool XG = false>
 __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
-                              uint32_t *Xarg, const Move &mv)
+                              uint32_t *Xarg, const Move &mv, bool a_done = false)
 {
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
@@ -437,10 +440,13 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     const int vlo = ps.vlo, Uc = ps.Uc;
 
     // A. pending move; counting sort over the conservative lattice; holes; no record starts yet
-    plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
-    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
+    //    (a_done: the caller ran the counting sort and its barrier, build_plan for m > 255)
+    if (!a_done) {
+        plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
+        if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
+    }
     for (int w = tid; w <= I.XW; w += NT) pstart[w] = -1;  // = 0xffffffff: no record (addresses, unsigned)
-    __syncthreads();
+    __syncthreads();  // also: every thread has read ps.vlo / Uc before step B rewrites them
     PH(0);
     // B. warp 0: exact range, cuts, and the placement in the order deep | walk 0 | walk 1 | top
     if (tid == 0 && mv.on) flip_bits((uint32_t *)(sm + L.vb), K, mv);
@@ -509,7 +515,11 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
 #pragma unroll 4
                 for (int v = uneg + q; v < utop; v += 2) {
                     const int Lv = cnt[uf + v];
-                    if (I.pad && Lv > 0 && (pos & 31) != 0 && (pos & 31) + Lv > 32) pos = (pos + 31) & ~31;
+                    // m > 255: X may have fewer than 2W + 1 words, so a pad is taken only while the
+                    // rows still to place fit (m <= 255: X has 2W + 1 words, every pad fits)
+                    if (I.pad && Lv > 0 && (pos & 31) != 0 && (pos & 31) + Lv > 32 &&
+                        (m <= PACKED_MAX_M || ((((pos + 31) & ~31) + (m - rows) + 31) >> 5) <= I.XW))
+                        pos = (pos + 31) & ~31;
                     // an empty point whose bin and its predecessor's are non-negative is absorbed:
                     // the predecessor's final record completes both bins (no record of its own)
                     const bool nonneg = vmin + 2 * (v - K) >= 0;
@@ -548,6 +558,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
             ps.P = runp; ps.pkb1 = pkb1; ps.Wp = (pos + 31) >> 5;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
             ps.uneg = uneg; ps.utop = utop; ps.rneg = rneg; ps.rtop = rtop; ps.cneg = 0; ps.hwalk = 0;
+            if (!a_done) ps.pkok = 1;
             ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
             ps.key = (unsigned long long)KEY_NONE;
             ps.gkey = (unsigned long long)KEY_NONE;
@@ -637,10 +648,9 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
 // Leaves cnt[] zeroed, ps.key / gkey = KEY_NONE and ps.vlo / Uc set for the next plan.
 // ------------------------------------------------------------------------------------------
 template <int K, bool XG = false>
-__device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
-                           uint32_t *Xarg, const Move &mv = Move{0, 0, 0, 0})
+__device__ void build_plan_seg(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                               uint32_t *Xarg, const Move &mv, bool a_done)
 {
-    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv); return; }
     uint32_t *X = XG ? Xarg : (uint32_t *)(sm + L.X);
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int m = I.m, n = I.n;
@@ -657,9 +667,11 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     const int vlo = ps.vlo, Uc = ps.Uc;
 
     // A. pending move; counting sort over the conservative lattice; holes of a padded placement
-    plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
-    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
-    __syncthreads();
+    if (!a_done) {
+        plan_count<K>(I, Ar, (int *)Ys, (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
+        if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) rowAt[p] = -1;
+    }
+    __syncthreads();  // also: every thread has read ps.vlo / Uc before step B rewrites them
     PH(0);
     if (tid == 0 && mv.on) flip_bits((uint32_t *)(sm + L.vb), K, mv);
     // B. warp 0: exact range (first / last non-empty point), exclusive scans of the row and piece
@@ -723,6 +735,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
             seg[U] = runr; pofs[U] = runp; ps.P = runp; pstart[Wp] = runp; ps.Wp = Wp;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
             ps.uneg = uneg; ps.utop = utop; ps.cneg = 0;
+            if (!a_done) ps.pkok = 0;  // (a_done: set by build_plan, read by every thread)
             ps.vlo = vmin - 2 * K; ps.Uc = U + 2 * K;
             ps.key = (unsigned long long)KEY_NONE;
             ps.gkey = (unsigned long long)KEY_NONE;
@@ -765,6 +778,56 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
     __syncthreads();
     PH(2);
     plan_transpose(I, Ar, sm, L, ps, X, Uc);
+}
+
+// The plan of the current state. m <= 255: the packed plan (every bin count fits a byte). m > 255
+// with I.pkw: the packed plan whenever this state's counts still fit bytes, i.e.
+// every byte the walk window can hold -- a walked bin's own rows plus the rows K points below it in
+// its walk -- is <= 255, and so is H_b of every walked bin; else the segment plan. Decided per
+// iteration by warp 0 after the shared counting sort.
+template <int K, bool XG = false>
+__device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                           uint32_t *Xarg, const Move &mv = Move{0, 0, 0, 0})
+{
+    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv); return; }
+    if (!I.pkw) { build_plan_seg<K, XG>(I, Ar, sm, L, ps, Xarg, mv, false); return; }
+    const int tid = threadIdx.x, lane = tid & 31;
+    int *cnt = (int *)(sm + L.cnt);
+    const int *Hs = (const int *)(sm + L.H);
+    const int vlo = ps.vlo, Uc = ps.Uc;
+    plan_count<K>(I, Ar, (int *)(sm + L.Y), (const uint32_t *)(sm + L.vb), cnt, vlo, mv);
+    if (I.pad) for (int p = tid; p < 32 * I.XW; p += NT) ((int *)(sm + L.rowAt))[p] = -1;
+    __syncthreads();
+    if (tid < 32) {
+        int uf = -1, ul = -1;
+        for (int b0 = 0; b0 < Uc; b0 += 32) {
+            const unsigned bal = __ballot_sync(FULL, b0 + lane < Uc && cnt[b0 + lane] > 0);
+            if (bal) {
+                if (uf < 0) uf = b0 + __ffs(bal) - 1;
+                ul = b0 + 31 - __clz(bal);
+            }
+        }
+        const int U = ul - uf + 1, vmin = vlo + 2 * uf;
+        int uneg = (-2 * K - vmin + 1) >> 1;
+        uneg = min(max(uneg, 0), U);
+        int utop = ((I.maxS + 2 * K - vmin) >> 1) + 1;
+        utop = min(max(utop, uneg), U);
+        bool bad = false;
+        for (int v = uneg + lane; v < utop + 2 * K; v += 32) {  // bins of both walks
+            int s4 = 0;
+            for (int t = 0; t <= K; t++) {
+                const int p = v - 2 * t;
+                if (p >= uneg && p < utop) s4 += cnt[uf + p];
+            }
+            const int b = vmin + 2 * (v - K);
+            bad |= s4 > 255 || (b >= 0 && b <= I.n && Hs[b] > 255);
+        }
+        const bool anybad = __any_sync(FULL, bad);
+        if (lane == 0) ps.pkok = anybad ? 0 : 1;
+    }
+    __syncthreads();
+    if (ps.pkok) build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv, true);
+    else build_plan_seg<K, XG>(I, Ar, sm, L, ps, Xarg, mv, true);
 }
 
 // One lattice point (segment) of eval_fit: its pieces add POPC counts of the bit-sliced planes
@@ -1078,7 +1141,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     const uint2 *pieces = (const uint2 *)(sm + L.pieces);
     const int2 *bins = (const int2 *)(sm + L.bins);
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
-    const bool packed = I.m <= PACKED_MAX_M;
+    const bool packed = ps.pkok;
     EvalRange er;
     er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
@@ -1400,7 +1463,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr, A.I.pkw);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
     const bool batch = A.R > 0;
@@ -1646,7 +1709,7 @@ __global__ void __launch_bounds__(NT, 1) k_step_eval(SearchArgs A, int64_t *key_
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr, A.I.pkw);
     const int lane = threadIdx.x & 31;
     if (!WRITE_ALL && A.fs[FS_DONE]) {
         if (blockIdx.x == 0 && threadIdx.x == 0) *key_out = KEY_NONE;
@@ -1725,7 +1788,7 @@ __global__ void __launch_bounds__(NT, 1) k_debug_plan(SearchArgs A, int32_t *out
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ PlanScalars ps;
-    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr);
+    const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr, A.I.pkw);
     const uint32_t *Ar = load_state<K>(A, sm, L, ps);
     const int *segp = (const int *)(sm + L.seg);
     if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L));
@@ -1801,6 +1864,7 @@ struct lns_ctx {
     nccl_allreduce_fn nccl_allreduce = nullptr;
     int blocks_override = 0;
     int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
+    int no_pkw = 0;  // LNS_NO_PKW=1 at create: m > 255 always takes the segment plan (A/B measurement)
     // device-initiated exchange (lns_attach_peers)
     unsigned long long *d_xbuf = nullptr;            // own 64-word exchange buffer (its own allocation)
     unsigned long long **d_peers = nullptr;          // device array of the partitions' buffers
@@ -1993,17 +2057,15 @@ struct Geometry {
     int a_in_smem = 0;
     int x_global = 0;      // X does not fit in shared memory: per-CTA slots in global memory
     int pad = 0, XW = 0;   // padded placement (packed path, when X of 2W + 1 words fits)
+    int pkw = 0;           // m > 255: packed records allocated, the packed plan tried per iteration
     size_t smem_eval = 0;  // bytes for the stepped / eval kernels
 };
 
-lns_status check_k(lns_ctx *c, int k, Geometry &g)
+// Shared-memory geometry of the plan for k (pkw: with the packed-record region for m > 255).
+lns_status geometry(lns_ctx *c, int k, Geometry &g, int pkw)
 {
-    if (!c) return fail(LNS_EINVAL, "null context");
-    if (k < 1 || k > 3) return fail(LNS_EINVAL, "k must be 1, 2 or 3");
-    if (c->n < k) return fail(LNS_EINVAL, "n < k");
-    const int64_t Mk = comb_k(c->n, k);
-    if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
-    g.M = (uint32_t)Mk;
+    g.pkw = c->m > PACKED_MAX_M ? pkw : 0;
+    g.a_in_smem = 0; g.x_global = 0; g.smem_eval = 0;
     const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
     // preference: X and A in shared memory; X only; neither (X in global memory)
     // padded placement first (packed path only): X of 2W + 1 words, with or without A staged
@@ -2020,20 +2082,39 @@ lns_status check_k(lns_ctx *c, int k, Geometry &g)
         // segment-loop path: padded placement within the largest X (XW words, W < XW <= 2W + 1)
         // that fits next to the plan (A from global memory)
         for (int XWp = 2 * c->W + 1; XWp > c->W; XWp--) {
-            const Smem pwo = smem_layout(c->m, c->n, XWp, c->NWn, k, 0);
+            const Smem pwo = smem_layout(c->m, c->n, XWp, c->NWn, k, 0, 0, g.pkw);
             if (pwo.a_end <= budget) { g.pad = 1; g.XW = XWp; g.a_in_smem = 0; g.smem_eval = (size_t)pwo.a_end; break; }
         }
         if (g.pad) return LNS_OK;
     }
-    const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1);
-    const Smem without = smem_layout(c->m, c->n, c->W, c->NWn, k, 0);
-    const Smem xg = smem_layout(c->m, c->n, c->W, c->NWn, k, 0, 1);
+    const Smem with = smem_layout(c->m, c->n, c->W, c->NWn, k, 1, 0, g.pkw);
+    const Smem without = smem_layout(c->m, c->n, c->W, c->NWn, k, 0, 0, g.pkw);
+    const Smem xg = smem_layout(c->m, c->n, c->W, c->NWn, k, 0, 1, g.pkw);
     if (with.a_end <= budget) { g.a_in_smem = 1; g.smem_eval = (size_t)with.a_end; }
     else if (without.a_end <= budget) { g.a_in_smem = 0; g.smem_eval = (size_t)without.a_end; }
     else if (xg.a_end <= budget) { g.a_in_smem = 0; g.x_global = 1; g.smem_eval = (size_t)xg.a_end; }
     else return fail(LNS_ERANGE, "plan does not fit in shared memory (n or m too large)");
+    return LNS_OK;
+}
+
+lns_status check_k(lns_ctx *c, int k, Geometry &g)
+{
+    if (!c) return fail(LNS_EINVAL, "null context");
+    if (k < 1 || k > 3) return fail(LNS_EINVAL, "k must be 1, 2 or 3");
+    if (c->n < k) return fail(LNS_EINVAL, "n < k");
+    const int64_t Mk = comb_k(c->n, k);
+    if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
+    g.M = (uint32_t)Mk;
+    // m > 255: the packed-record region first, unless it pushes X out of shared
+    // memory where the segment plan alone would keep it there
+    lns_status s = geometry(c, k, g, (c->m > PACKED_MAX_M && !c->no_pkw) ? 1 : 0);
+    if (g.pkw && (s != LNS_OK || g.x_global)) {
+        Geometry g0 = g;
+        if (geometry(c, k, g0, 0) == LNS_OK && (s != LNS_OK || !g0.x_global)) { g = g0; s = LNS_OK; }
+    }
+    if (s != LNS_OK) return s;
     if (g.x_global) {  // one X slot per CTA of the largest grid any launch uses (eval_all: 8 x SMs)
-        lns_status s = grow(c->d_X, c->X_cap, (size_t)8 * c->numSMs * c->W * c->n);
+        s = grow(c->d_X, c->X_cap, (size_t)8 * c->numSMs * c->W * c->n);
         if (s != LNS_OK) return s;
     }
     return LNS_OK;
@@ -2055,6 +2136,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     SearchArgs A;
     A.I = dev_inst(c);
     A.I.XW = g.XW > 0 ? g.XW : c->W;
+    A.I.pkw = g.pkw;
     A.I.pad = 0;  // per launch: pad_for()
     A.M = g.M;
     slice_of(g.M, c->part, c->nparts, A.lo, A.hi);
@@ -2375,6 +2457,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     lns_ctx *c = new lns_ctx();
     c->device = device; c->m = m; c->n = n; c->W = W; c->NWn = NWn;
     { const char *e = getenv("LNS_NO_PAD"); c->no_pad = (e && e[0] == '1') ? 1 : 0; }
+    { const char *e = getenv("LNS_NO_PKW"); c->no_pkw = (e && e[0] == '1') ? 1 : 0; }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };

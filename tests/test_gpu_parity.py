@@ -243,6 +243,50 @@ def test_large_m_padded_placement_trajectory(L, orc, m, n, k, blocks, iters):
     assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
 
 
+def _clustered_instance(m, n, npool, noise, seed):
+    """Rows drawn from a small pool of +-1 rows (plus noise): many rows share a lattice point, so
+    some states exceed the byte window of the packed plan for m > 255 and others do not."""
+    rng = np.random.default_rng(seed)
+    pool = np.where(rng.random((npool, n)) < 0.5, -1, 1).astype(np.int8)
+    A = pool[rng.integers(0, npool, m)].copy()
+    A[rng.random((m, n)) < noise] *= -1
+    secret = np.where(rng.random(n) < 0.5, -1, 1).astype(np.int8)
+    y = A.astype(np.int64) @ secret
+    A[y < 0] *= -1
+    return A, np.abs(y).astype(np.int32)
+
+
+@pytest.mark.parametrize("k,iters,m,npool,noise", [(1, 150, 700, 10, 0.1), (2, 60, 550, 8, 0.12),
+                                                   (3, 25, 500, 8, 0.12)])
+@pytest.mark.parametrize("blocks", [1, 5])
+def test_large_m_packed_plan_guard_mixed_trajectory(L, orc, k, iters, m, npool, noise, blocks):
+    """m > 255: each iteration takes the packed byte-window plan when the
+    state's counts fit bytes and the segment plan otherwise. On these clustered instances the
+    guard (restated in tests/test_packed_model.bytes_fit) switches along the trajectory; the
+    whole trajectory must equal the oracle's."""
+    from test_packed_model import bytes_fit
+
+    n = 40
+    A, S = _clustered_instance(m, n, npool, noise, 100 + k)
+    V0 = pi.start_vector(n, 7 + k)
+    ten = pi.default_tenure(n, k)
+    otr, otf, oVo, ores = orc.tabu_run(A, S, k, V0, iters, ten, stop_on_zero=False)
+    V = V0.astype(np.int64).copy()
+    fits = []
+    for t in range(iters):
+        fits.append(bytes_fit(A.astype(np.int64), S, V, k))
+        for i in orc.flipsets(n, k, [otr[t]])[0]:
+            if i >= 0:
+                V[i] = -V[i]
+    assert 0 < sum(fits) < iters  # both plans are taken
+    with L.Instance(A, S) as I:
+        L.lns_config(I.ctx, blocks)
+        tr, tf, Vo, res = I.tabu_run(k, iters, -1, V0=V0, stop_on_zero=False)
+        assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+        for Vs in (V0, oVo):
+            assert np.array_equal(L.lns_eval_all(I.ctx, k, Vs).astype(np.int64), orc.eval_all(A, S, Vs, k))
+
+
 @pytest.mark.parametrize("G", [2, 3, 8])
 def test_partitioned_search_emulated_on_one_gpu(L, orc, G):
     """The multi-GPU protocol (PAPER.md:448-454 partitioning): G contexts each own a slice of the

@@ -243,3 +243,53 @@ def test_packed_model_absorbs_empty_points():
             V2[F] *= -1
             assert fitness(P, 3, F) == oracle.fitness(inst.A, inst.S, V2.astype(np.int8))
     assert seen > 0
+
+
+def bytes_fit(A, S, V, K):
+    """build_plan's guard for m > 255: every byte a walk window holds -- a walked
+    bin's own rows plus those of the K points below it in its walk -- is <= 255, and so is H_b of
+    every walked bin."""
+    m, n = A.shape
+    Y = A @ V
+    H = np.bincount(S, minlength=n + 1)
+    maxS = max(b for b in range(n + 1) if H[b] > 0)
+    vmin = int(Y.min())
+    U = (int(Y.max()) - vmin) // 2 + 1
+    cnt = [int(((Y - vmin) // 2 == u).sum()) for u in range(U)]
+    uneg = min(max((-2 * K - vmin + 1) >> 1, 0), U)
+    utop = min(max(((maxS + 2 * K - vmin) >> 1) + 1, uneg), U)
+    for v in range(uneg, utop + 2 * K):
+        s4 = sum(cnt[v - 2 * t] for t in range(K + 1) if uneg <= v - 2 * t < utop)
+        b = vmin + 2 * (v - K)
+        if s4 > 255 or (0 <= b <= n and H[b] > 255):
+            return False
+    return True
+
+
+@pytest.mark.parametrize("pad", [0, 1])
+def test_packed_model_large_m_when_bytes_fit(pad):
+    """m > 255: the byte-window arithmetic stays exact whenever the guard holds (random and
+    near-secret states of planted instances up to 1024 rows); a state with > 255 rows on one
+    lattice point fails the guard (the kernel then takes the segment plan)."""
+    rng = np.random.default_rng(23 + pad)
+    fit = 0
+    for trial in range(8):
+        m, n = [(300, int(rng.integers(20, 64))), (520, int(rng.integers(40, 64))),
+                (1024, int(rng.integers(200, 260)))][trial % 3]
+        K = int(rng.integers(1, 4))
+        inst = pi.planted_instance(m, n, int(rng.integers(1_000_000)))
+        A = inst.A.astype(np.int64)
+        V = np.where(rng.random(n) < 0.5, -1, 1).astype(np.int64) if trial % 2 else inst.secret.astype(np.int64)
+        if not bytes_fit(A, inst.S, V, K):
+            continue
+        fit += 1
+        P = build_plan(A, inst.S, V, K, pad)
+        for _ in range(6):
+            F = sorted(rng.choice(n, K, replace=False).tolist())
+            V2 = V.copy()
+            V2[F] *= -1
+            assert fitness(P, K, F) == oracle.fitness(inst.A, inst.S, V2.astype(np.int8)), (m, n, K, F)
+    assert fit >= 5
+    rows = np.tile(np.where(rng.random((1, 30)) < 0.5, -1, 1), (300, 1)).astype(np.int64)  # 300 equal rows
+    V = rows[0].copy()  # every row at Y = 30: one walked lattice point of 300 rows
+    assert not bytes_fit(rows, (rows @ V).astype(np.int32), V, 2)
