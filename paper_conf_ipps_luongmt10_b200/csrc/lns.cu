@@ -1356,14 +1356,16 @@ __device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, co
 // share of it against vbs = V_{t-1} and writes until[rank] = t for the ranks of this device's
 // slice (tabu at t, admissible again at t + 1: nothing to clear). CTA 0 stores V_{t-1} into its
 // slot first (it is not among the listed entries scanned at t). A group barrier (arrival counter
-// bar, monotonic, nb arrivals per pass) then publishes until[] before the evaluation reads it.
+// bar, monotonic, nb arrivals per pass; tb = this pass's number, one pass per iteration of the
+// group) then publishes until[] before the evaluation reads it.
 template <int K>
 __device__ void sol_tabu(const SearchArgs &A, const unsigned char *sm, const Smem &L, const uint32_t *vbs,
-                         uint32_t *ring, uint32_t *until, int64_t t, int bid, int nb, unsigned long long *bar,
-                         unsigned long long &tb)
+                         int gg, uint32_t *until, int64_t t, int bid, int nb, unsigned long long *bar,
+                         unsigned long long tb)
 {
     const int NW = A.I.NWn, n = A.I.n;
     const int64_t Lt = A.L;
+    uint32_t *ring = A.ring + (size_t)gg * (size_t)Lt * NW;
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
     __syncthreads();  // vbs = V_{t-1}: the previous move was applied by the plan
     const int64_t skip = (t - 1) % Lt;  // slot of V_{t-1} (held V_{t-1-L}, no longer listed)
@@ -1389,7 +1391,6 @@ __device__ void sol_tabu(const SearchArgs &A, const unsigned char *sm, const Sme
     if (nb > 1) {
         __syncthreads();
         if (threadIdx.x == 0) {
-            tb++;
             __threadfence();
             asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(bar) : "memory");
             const unsigned long long target = (unsigned long long)nb * tb;
@@ -1511,8 +1512,6 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         tri = ts;
     }
     unsigned long long tg = 0;  // iterations run by this group in this phase (exchange clock)
-    unsigned long long tb = 0;  // solution-list barrier passes (LNS_TABU_SOLUTIONS)
-    uint32_t *ring = A.sol_list ? A.ring + (size_t)gg * (size_t)A.L * A.I.NWn : nullptr;
     const int rbeg = batch ? A.phr0[phq] : 0, rend = batch ? A.phr0[phq] + A.phR[phq] : 1;
     for (int rs = rbeg + (batch ? g : 0); rs < rend; rs += G) {
         int64_t f, best_f, best_it, zero_it, t0;
@@ -1534,7 +1533,8 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (A.stop_on_zero && f == 0) break;
             if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
             else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr, mv);
-            if (A.sol_list) sol_tabu<K>(A, sm, L, vbs, ring, until, t, bid, nb, gslots + 24, tb);
+            // (the solution-list barrier is passed once per iteration, before the exchange: pass tg + 1)
+            if (A.sol_list) sol_tabu<K>(A, sm, L, vbs, gg, until, t, bid, nb, gslots + 24, tg + 1);
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
                                                   nullptr, tri, A.aspiration, (int)best_f)
