@@ -117,10 +117,11 @@ def neighborhood_size(n: int, k: int) -> int:
 
 
 def flipsets(n: int, k: int, ranks) -> np.ndarray:
-    """Flip sets (rows of 3, -1 padded) of ascending `ranks`, by walking the nested loops."""
+    """Flip sets (rows of max(3, k), -1 padded) of ascending `ranks`, by walking the nested loops
+    (k >= 4: the odometer generalisation of the same loops)."""
     ranks = np.ascontiguousarray(ranks, dtype=np.int64)
     assert np.all(np.diff(ranks) >= 0)
-    out = np.empty((len(ranks), 3), dtype=np.int32)
+    out = np.empty((len(ranks), max(3, k)), dtype=np.int32)
     rc = _load().oracle_flipsets(n, k, _p(ranks, _i64p), len(ranks), _p(out, _i32p))
     if rc != 0:
         raise ValueError("rank out of range")

@@ -18,8 +18,8 @@
  * Parity status: every function is pinned by tests/test_oracle.py:
  *   fitness      -- hand-computed golden values, f(V*) = 0 on planted instances, brute force
  *                   zero set == multiset equality, f >= 0, parity f = #negative rows (mod 2)
- *   rank order   -- itertools.combinations order, the paper's worked example (n = 6,
- *                   (2,3) -> 9), Appendix A-D formulas, C(n,k) counts
+ *   rank order   -- itertools.combinations order (k = 1..7), the paper's worked example
+ *                   (n = 6, (2,3) -> 9), Appendix A-D formulas, C(n,k) counts
  *   selection    -- brute-force argmin with lowest-rank tie-break, tabu invariants
  *   trajectory   -- stop-on-zero reaches a vector whose multiset equals S
  */
@@ -174,9 +174,39 @@ int64_t oracle_fitness_packed(const int8_t *A, int32_t m, int32_t n, const int32
  * Appendix A for k = 2 and of the "set of plans" of Appendix C for k = 3).
  * first_count[i1] = number of flip sets whose smallest index is i1, counted by a loop.
  * ------------------------------------------------------------------------------------- */
+#define ORACLE_KMAX 7
+
+/* k >= 4 ("k > 3 via the combinatorial number system"): the flip sets are
+ * still enumerated in lexicographic order by nested loops -- an odometer over i1 < i2 < ... < ik
+ * (the innermost index runs fastest; when it cannot advance, the next one out advances and the
+ * inner ones restart right after it) -- and the rank is still the loop counter. The number of
+ * flip sets whose smallest index is i1 is the number of (k-1)-subsets of {i1+1, ..., n-1},
+ * counted with Pascal's rule (subsets of a set of a elements: C(a, r) = C(a-1, r-1) + C(a-1, r)). */
+static int64_t subsets(int32_t a, int32_t r)
+{
+    int64_t row[ORACLE_KMAX + 1];
+    if (r < 0 || r > a) return 0;
+    for (int32_t j = 0; j <= r; j++) row[j] = (j == 0);
+    for (int32_t x = 1; x <= a; x++)
+        for (int32_t j = (x < r ? x : r); j >= 1; j--) row[j] += row[j - 1];
+    return row[r];
+}
+
+/* First flip set after idx[0..k-1] in lexicographic order, keeping idx[0..fixed-1]: 0 at the end. */
+static int odometer_next(int32_t *idx, int32_t k, int32_t n, int32_t fixed)
+{
+    int32_t j = k - 1;
+    while (j >= fixed && idx[j] == n - k + j) j--;
+    if (j < fixed) return 0;
+    idx[j]++;
+    for (int32_t q = j + 1; q < k; q++) idx[q] = idx[q - 1] + 1;
+    return 1;
+}
+
 static int64_t count_with_first(int32_t n, int32_t k, int32_t i1)
 {
     int64_t c = 0;
+    if (k >= 4) return subsets(n - 1 - i1, k - 1);
     if (k == 1) return 1;
     for (int32_t i2 = i1 + 1; i2 < n; i2++) {
         if (k == 2) c += 1;
@@ -197,6 +227,18 @@ int64_t oracle_neighborhood_size(int32_t n, int32_t k)
 int32_t oracle_flipsets(int32_t n, int32_t k, const int64_t *ranks, int64_t cnt, int32_t *out)
 {
     int64_t r = 0, q = 0;
+    if (k >= 4 && k <= ORACLE_KMAX && k <= n) { /* the odometer; rows of k indices */
+        int32_t idx[ORACLE_KMAX];
+        for (int32_t j = 0; j < k; j++) idx[j] = j;
+        do {
+            while (q < cnt && ranks[q] == r) {
+                for (int32_t j = 0; j < k; j++) out[(int64_t)k * q + j] = idx[j];
+                q++;
+            }
+            r++;
+        } while (q < cnt && odometer_next(idx, k, n, 0));
+        return q == cnt ? 0 : -1;
+    }
     if (k < 1 || k > 3) return -1;
     for (int32_t i1 = 0; i1 < n && q < cnt; i1++) {
         int32_t i2s = (k >= 2) ? i1 + 1 : 0, i2e = (k >= 2) ? n : 1;
@@ -295,6 +337,31 @@ static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k
                 q = lo;
                 if (q >= nsample || sample[q] >= base[i1 + 1]) continue;
             }
+            if (k >= 4) { /* odometer over i2 < ... < ik, i1 fixed */
+                int32_t idx[ORACLE_KMAX];
+                idx[0] = i1;
+                for (int32_t j = 1; j < k; j++) idx[j] = i1 + j;
+                if (idx[k - 1] >= n) continue;
+                do {
+                    if (mode == 2 && (q >= nsample || sample[q] != r)) { r++; continue; }
+                    int tabu = (mode == 1 && until && !(until[r] < t));
+                    if (tabu && aspire_below < 0) { r++; continue; }
+                    memcpy(vb, vb0, sizeof(uint64_t) * (size_t)P->nw);
+                    for (int32_t j = 0; j < k; j++) flip(vb, idx[j]);
+                    if (mode == 1 && sols && solset_contains(sols, vb)) {
+                        tabu = 1;
+                        if (aspire_below < 0) { r++; continue; }
+                    }
+                    int64_t f = fitness_packed(P, vb, Y, Hp);
+                    if (!(tabu && !(f < aspire_below))) {
+                        if (mode == 0) f_all[r] = f;
+                        else if (mode == 2) { while (q < nsample && sample[q] == r) { f_all[q] = f; q++; } }
+                        else if (f < mine.f || (f == mine.f && r < mine.r)) { mine.f = f; mine.r = r; }
+                    }
+                    r++;
+                } while (odometer_next(idx, k, n, 1));
+                continue;
+            }
             int32_t i2s = (k >= 2) ? i1 + 1 : 0, i2e = (k >= 2) ? n : 1;
             for (int32_t i2 = i2s; i2 < i2e; i2++) {
                 int32_t i3s = (k == 3) ? i2 + 1 : 0, i3e = (k == 3) ? n : 1;
@@ -335,7 +402,7 @@ static fr_t scan_neighbourhood(const packed_t *P, const uint64_t *vb0, int32_t k
 int32_t oracle_eval_all(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
                         int32_t k, int64_t *f_all, int32_t nthreads)
 {
-    if (k < 1 || k > 3 || n < k) return -1;
+    if (k < 1 || k > ORACLE_KMAX || n < k) return -1;
     packed_t P;
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
@@ -349,7 +416,7 @@ int32_t oracle_eval_all(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
 int32_t oracle_eval_ranks(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
                           int32_t k, const int64_t *ranks, int64_t cnt, int64_t *f_out, int32_t nthreads)
 {
-    if (k < 1 || k > 3 || n < k) return -1;
+    if (k < 1 || k > ORACLE_KMAX || n < k) return -1;
     packed_t P;
     pack_instance(A, m, n, S, &P);
     uint64_t *vb = malloc(sizeof(uint64_t) * (size_t)P.nw);
@@ -363,7 +430,7 @@ int32_t oracle_eval_ranks(const int8_t *A, int32_t m, int32_t n, const int32_t *
 int32_t oracle_eval_best(const int8_t *A, int32_t m, int32_t n, const int32_t *S, const int8_t *V,
                          int32_t k, const uint8_t *tabu, int64_t *best_f, int64_t *best_r, int32_t nthreads)
 {
-    if (k < 1 || k > 3 || n < k) return -1;
+    if (k < 1 || k > ORACLE_KMAX || n < k) return -1;
     int64_t M = oracle_neighborhood_size(n, k);
     int32_t *until = NULL;
     if (tabu) {
@@ -405,7 +472,7 @@ int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
      * L most recently visited solutions V_{t-L} .. V_{t-1} (V_0 = the start, V_{t-1} = the current
      * solution, which is never a neighbour); a neighbour is tabu iff it equals one of them. */
     const int aspiration = flags & 1, solutions = (flags & 2) != 0;
-    if (k < 1 || k > 3 || n < k || m < 1 || iters < 0 || L < 0) return -1;
+    if (k < 1 || k > ORACLE_KMAX || n < k || m < 1 || iters < 0 || L < 0) return -1;
     int64_t M = oracle_neighborhood_size(n, k);
     if (L >= M) return -2;
     if (solutions && L < 1) return -1;
@@ -438,7 +505,7 @@ int32_t oracle_tabu_run(const int8_t *A, int32_t m, int32_t n, const int32_t *S,
                                     aspiration ? best_f : -1, solutions ? &sols : NULL);
         if (b.r < 0) break; /* unreachable for L < M */
         /* apply: V <- V xor F_{r*}; flip set of r* found by walking the same nested loops */
-        int32_t F[3];
+        int32_t F[ORACLE_KMAX];
         oracle_flipsets(n, k, &b.r, 1, F);
         for (int32_t q = 0; q < k; q++) flip(vb, F[q]);
         f = b.f;

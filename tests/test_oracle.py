@@ -385,3 +385,45 @@ def test_tabu_solution_list_variant(orc, k, L, aspiration):
             Vc = _flip(Vc, fs)
             assert tuple(Vc) not in set(seen[max(0, len(seen) - L):])
             seen.append(tuple(Vc))
+
+
+# ---------------------------------------------------------------- k > 3
+@pytest.mark.parametrize("k", [4, 5, 6, 7])
+@pytest.mark.parametrize("n", [7, 8, 11, 16])
+def test_oracle_rank_order_k_above_3_is_lexicographic(orc, n, k):
+    """k >= 4: the odometer (nested loops generalised) enumerates flip sets in
+    itertools.combinations order and counts C(n, k) of them."""
+    if k > n:
+        return
+    M = comb(n, k)
+    assert orc.neighborhood_size(n, k) == M
+    got = orc.flipsets(n, k, np.arange(M))
+    assert np.array_equal(got, np.array(list(itertools.combinations(range(n), k)), dtype=np.int32))
+
+
+@pytest.mark.parametrize("k", [4, 5])
+def test_eval_all_k_above_3_matches_scalar_fitness(orc, k):
+    """new_fitness[rank] = f(V xor F_rank) for k = 4, 5 (scalar int8 fitness of the explicitly
+    flipped vector, ranks in itertools order), and the sampled / best variants agree."""
+    rng = np.random.default_rng(40 + k)
+    I = pi.planted_instance(13, 15, 91 + k)
+    V = np.where(rng.random(15) < 0.5, -1, 1).astype(np.int8)
+    fa = orc.eval_all(I.A, I.S, V, k)
+    assert len(fa) == comb(15, k)
+    for r, fs in enumerate(itertools.combinations(range(15), k)):
+        assert fa[r] == orc.fitness(I.A, I.S, _flip(V, fs))
+    ranks = np.unique(rng.integers(0, len(fa), 40))
+    assert np.array_equal(orc.eval_ranks(I.A, I.S, V, k, ranks), fa[ranks])
+    tabu = rng.random(len(fa)) < 0.3
+    bf, br = orc.eval_best(I.A, I.S, V, k, tabu)
+    masked = np.where(tabu, np.iinfo(np.int64).max, fa)
+    assert br == int(np.argmin(masked)) and bf == fa[br]
+
+
+@pytest.mark.parametrize("k,L", [(4, 0), (4, 30), (5, 100)])
+def test_tabu_trajectory_rules_k_above_3(orc, k, L):
+    I = pi.planted_instance(14, 16, 700 + k)
+    V0 = pi.start_vector(16, 9 + k)
+    tr, tf, Vo, res = orc.tabu_run(I.A, I.S, k, V0, 25, L, stop_on_zero=False)
+    V = _check_tabu_trace(orc, I.A, I.S, k, V0, L, tr, tf, res, False)
+    assert np.array_equal(V, Vo)
