@@ -42,7 +42,7 @@ extern "C" {
 
 typedef int32_t lns_status;
 #define LNS_OK 0
-#define LNS_EINVAL (-1)         /* bad argument (k not in {1,2,3}, n < k, A not +-1, S outside [0,n], Y != A V, ...) */
+#define LNS_EINVAL (-1)         /* bad argument (k not in 1..7 or the call not available for k, n < k, A not +-1, S outside [0,n], Y != A V, ...) */
 #define LNS_ERANGE (-2)         /* size limit exceeded (see Limits), or tenure >= C(n,k) */
 #define LNS_ENOMEM (-3)         /* device or host allocation failed */
 #define LNS_ECUDA (-4)          /* CUDA runtime error (message in lns_last_error) */
@@ -124,6 +124,10 @@ lns_status lns_eval_all(lns_ctx *ctx, int32_t k, const int8_t *V, int32_t *fitne
  *   slice of ranks and one NCCL u64-MIN all-reduce per iteration picks the global move; the
  *   trajectory is identical for any number of GPUs.  Synchronous.
  *   Errors: EINVAL, ERANGE (limits, tenure >= C(n,k)), ENOMEM, ECUDA, ENCCL. */
+/* k > 3 (PAPER.md:105-125 generalised; 4 <= k <= 7): lns_tabu_run (one
+ *   device, persistent kernel, rank tabu list with or without LNS_ASPIRATION), lns_eval_all and
+ *   lns_unrank only; m <= 255 (the byte window) else ERANGE; other calls and
+ *   flags with k > 3 return EINVAL. */
 lns_status lns_tabu_run(lns_ctx *ctx, int32_t k, int64_t iters, int64_t tenure, uint64_t seed,
                         const int8_t *V0, int32_t flags, int8_t *V_out, int64_t *trace_rank,
                         int64_t *trace_fit, lns_result *res, void *stream);
@@ -139,6 +143,7 @@ lns_status lns_tabu_run_batch(lns_ctx *ctx, int32_t k, int32_t R, int64_t iters,
                               lns_result *res, void *stream);
 
 /* lns_unrank -- flip sets of ranks (device kernel; used by tests of the rank order).
+ *   k = 4..7: out is count x k int32 (the generic-k unranking of the k > 3 kernel).
  *   ranks: (host|device) count int64 in [0, C(n,k)).  out: (host|device) count x 3 int32,
  *   unused slots -1.  Synchronous. Errors: EINVAL (rank out of range), ERANGE, ECUDA. */
 lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count, int32_t *out,
@@ -211,7 +216,7 @@ double lns_last_kernel_ms(lns_ctx *ctx);
  * the stepped API) and CTAs of lns_eval_all / lns_eval_neighborhood. Results never depend on it. */
 lns_status lns_config(lns_ctx *ctx, int32_t blocks);
 
-int64_t lns_neighborhood_size(int32_t n, int32_t k); /* C(n,k), or -1 if k not in {1,2,3} */
+int64_t lns_neighborhood_size(int32_t n, int32_t k); /* C(n,k), or -1 if k not in 1..7 */
 const char *lns_strerror(lns_status status);
 const char *lns_last_error(void);
 int32_t lns_version(void); /* major*10000 + minor*100 + patch */

@@ -295,7 +295,7 @@ def lns_unrank(n: int, k: int, ranks, out=None, stream=None):
     pr, kr = _ptr(ranks, np.int64)
     cnt = int(len(ranks))
     if out is None:
-        out = np.empty((cnt, 3), dtype=np.int32)
+        out = np.empty((cnt, max(3, k)), dtype=np.int32)  # k >= 4: count x k
     _check(load().lns_unrank(n, k, pr, cnt, _out_ptr(out, np.int32), _stream(stream)), "lns_unrank")
     return out
 

@@ -1846,6 +1846,361 @@ __global__ void k_bits_to_until(const uint32_t *bits, uint32_t *until, uint32_t 
         until[r] = bits ? (bits[r >> 5] >> (r & 31)) & 1u : 0u;
 }
 
+// ------------------------------------------------------------------------------------------
+// k = 4..7 ("k > 3 via the combinatorial number system"), m <= 255.
+// A compact variant of the same method: exact combinatorial unranking for any k (the complement
+// identity lex_rank(i_1 < .. < i_k) = M - 1 - sum_j C(n-1-i_j, k-j+1), u64 tables, binary
+// search per position), lexicographic successor stepping over each thread's contiguous run of
+// ranks, and the parity walks of §5.9 evaluated ROW by row: a walked row of lattice point u with
+// t = #{i in F : x_ji = 1} (one AND + POPC per column word F touches) adds 1 to byte t of a
+// 64-bit window (bins u, u+2, .., u+2k of its walk: k+1 <= 8 bytes, counts <= m <= 255); when a
+// point's rows are done its bin (byte 0) is complete: f += w_b h + |h - H_b|, and the window
+// shifts by one byte. Deep rows (Y < -2k) cost 60(2k - Y) - 240 t, rows above max(S) + 2k cost 1,
+// bins of [0, n] outside both walks cost H_b. One persistent cooperative kernel per search, the
+// same (f << 32 | r) key, warp/CTA argmin and counter exchange as k_search.
+// ------------------------------------------------------------------------------------------
+constexpr int KG_MAX = 7;
+constexpr int NTG = 512;  // threads per CTA of the generic-k kernel (k registers of indices/masks)
+
+struct GenArgs {
+    DevInst I;
+    int32_t K;
+    uint32_t M;
+    int64_t iters, L;
+    int32_t stop_on_zero, aspiration;
+    uint32_t *vb;
+    int32_t *Y;
+    int64_t *fs;
+    uint32_t *until;
+    int64_t *slots;
+    int64_t *trace_r, *trace_f;
+    int32_t *fit_out;  // non-null: write every rank's fitness (lns_eval_all), no search
+};
+
+struct GenSmem {
+    int Bs, Y, vb, cnt, pos, cur, bins, C, end;
+};
+
+__host__ __device__ inline GenSmem gen_layout(int m, int n, int NWn, int K)
+{
+    GenSmem s;
+    int o = 0;
+    s.Bs = o;   o = align16(o + 4 * m * NWn);          // sorted rows' sign bits x_jc
+    s.Y = o;    o = align16(o + 4 * m);
+    s.vb = o;   o = align16(o + 4 * NWn);
+    s.cnt = o;  o = align16(o + 4 * (n + 1));           // rows per lattice point u = (Y + n) / 2
+    s.pos = o;  o = align16(o + 4 * (n + 1));           // first sorted slot of point u
+    s.cur = o;  o = align16(o + 4 * (n + 1));
+    s.bins = o; o = align16(o + 8 * (n + 2 * K + 1));   // (H_b, w_b) of bin u' in [-K, n + K]
+    s.C = o;    o = align16(o + 8 * (n + 1) * (K + 1)); // C(x, e), x <= n, e <= K (u64)
+    s.end = o;
+    return s;
+}
+
+struct GenScalars {
+    int ua, np[2], ndeep, ntop, walk0[2];
+    int cbase;  // m - (H of the walked bins) + 60 sum_deep (2K - Y) + #top rows
+    unsigned long long key, gkey;
+};
+
+__device__ __forceinline__ void gen_unrank(uint32_t r, int n, int K, uint32_t M, const unsigned long long *C,
+                                           int *idx)
+{
+    unsigned long long R = (unsigned long long)(M - 1u - r);
+    int cprev = n;
+#pragma unroll
+    for (int j = 0; j < KG_MAX; j++) {
+        if (j < K) {
+            const int e = K - j;
+            int lo = e - 1, hi = cprev - 1;  // largest c in [lo, hi] with C(c, e) <= R (C(e-1, e) = 0)
+            while (lo < hi) {
+                const int mid = (lo + hi + 1) >> 1;
+                if (C[mid * (K + 1) + e] <= R) lo = mid; else hi = mid - 1;
+            }
+            R -= C[lo * (K + 1) + e];
+            idx[j] = n - 1 - lo;
+            cprev = lo;
+        }
+    }
+}
+
+// Lexicographic successor (the last index varies fastest; loops unrolled so idx stays in
+// registers). Only called when a successor exists.
+__device__ __forceinline__ void gen_succ(int n, int K, int *idx)
+{
+    int j = K - 1;  // rightmost index that can still advance
+#pragma unroll
+    for (int q = KG_MAX - 1; q > 0; q--)
+        if (q == j && idx[q] == n - K + q) j--;
+#pragma unroll
+    for (int q = 0; q < KG_MAX; q++) {
+        if (q == j) idx[q]++;
+        else if (q > 0 && q > j && q < K) idx[q] = idx[q - 1] + 1;
+    }
+}
+
+// The flip set as column-word masks: wq[j] = word of idx[j]; wm[j] = the bits of every index in
+// that word if j is the first index there, else 0 (indices ascend, so a word's indices are
+// consecutive). Static indexing only.
+__device__ __forceinline__ void gen_masks(const int *idx, int K, int *wq, uint32_t *wm)
+{
+#pragma unroll
+    for (int j = 0; j < KG_MAX; j++) {
+        wq[j] = j < K ? idx[j] >> 5 : 0;
+        wm[j] = 0;
+    }
+#pragma unroll
+    for (int j = 0; j < KG_MAX; j++) {
+        if (j < K && (j == 0 || wq[j] != wq[j > 0 ? j - 1 : 0])) {
+#pragma unroll
+            for (int q = j; q < KG_MAX; q++)
+                if (q < K && wq[q] == wq[j]) wm[j] |= 1u << (idx[q] & 31);
+        }
+    }
+}
+
+// t = #{i in F : x_ji = 1} for the sorted row brow.
+__device__ __forceinline__ int gen_t(const uint32_t *__restrict__ brow, const int *wq, const uint32_t *wm)
+{
+    int t = 0;
+#pragma unroll
+    for (int e = 0; e < KG_MAX; e++)
+        if (wm[e]) t += __popc(brow[wq[e]] & wm[e]);
+    return t;
+}
+
+// Plan of the current (Y, V): apply the pending move first (pending = K indices, or none).
+__device__ void gen_plan(const GenArgs &A, unsigned char *sm, const GenSmem &L, GenScalars &gs, const int *mvidx,
+                         bool pending)
+{
+    const int tid = threadIdx.x, m = A.I.m, n = A.I.n, NWn = A.I.NWn, K = A.K;
+    uint32_t *Bs = (uint32_t *)(sm + L.Bs);
+    int *Ys = (int *)(sm + L.Y), *cnt = (int *)(sm + L.cnt), *pos = (int *)(sm + L.pos), *cur = (int *)(sm + L.cur);
+    uint32_t *vbs = (uint32_t *)(sm + L.vb);
+    int2 *bins = (int2 *)(sm + L.bins);
+    const uint32_t *Ar = A.I.Arow;
+    for (int u = tid; u <= n; u += NTG) cnt[u] = 0;
+    if (pending) {  // Y'_j = Y_j - 2 sum_{i in F} B_ji = Y_j - 2K + 4 t_j
+        for (int j = tid; j < m; j += NTG) {
+            int t = 0;
+            for (int q = 0; q < K; q++) {
+                const int i = mvidx[q];
+                t += (int)(((__ldg(Ar + (size_t)j * NWn + (i >> 5)) ^ vbs[i >> 5]) >> (i & 31)) & 1u);
+            }
+            Ys[j] += 4 * t - 2 * K;
+        }
+        __syncthreads();
+        if (tid == 0)
+            for (int q = 0; q < K; q++) vbs[mvidx[q] >> 5] ^= 1u << (mvidx[q] & 31);
+    }
+    __syncthreads();
+    for (int j = tid; j < m; j += NTG) atomicAdd(&cnt[(Ys[j] + n) >> 1], 1);
+    __syncthreads();
+    if (tid == 0) {
+        // walked points: -2K <= Y = 2u - n <= maxS + 2K; placement deep | walk 0 | walk 1 | top
+        const int ua = max(0, (n - 2 * K + 1) >> 1), ub = min(n, (A.I.maxS + 2 * K + n) >> 1);
+        int p = 0, cdeep = 0;
+        for (int u = 0; u < min(ua, n + 1); u++) { pos[u] = p; p += cnt[u]; cdeep += cnt[u] * 60 * (2 * K - (2 * u - n)); }
+        gs.ndeep = p;
+        int hwalk = 0;
+        for (int q = 0; q < 2; q++) {
+            int np = 0;
+            for (int u = ua + q; u <= ub; u += 2) { pos[u] = p; p += cnt[u]; np++; }
+            gs.np[q] = np;
+            gs.walk0[q] = ua + q;
+            for (int P = 0; P < np + K; P++) {  // bins of walk positions 0 .. np + K - 1
+                const int b = 2 * (ua + q + 2 * P - K) - n;
+                if (np > 0 && b >= 0 && b <= n) hwalk += A.I.H[b];
+            }
+        }
+        const int pt = p;
+        for (int u = max(ub + 1, ua); u <= n; u++) { pos[u] = p; p += cnt[u]; }
+        gs.ntop = p - pt;
+        gs.ua = ua;
+        gs.cbase = m - hwalk + cdeep + gs.ntop;
+        gs.key = (unsigned long long)KEY_NONE;
+        gs.gkey = (unsigned long long)KEY_NONE;
+    }
+    for (int x = tid; x < n + 2 * K + 1; x += NTG) {
+        const int b = 2 * (x - K) - n;
+        bins[x] = make_int2((b >= 0 && b <= n) ? A.I.H[b] : 0, b < 0 ? 60 * (-b) - 1 : 0);
+    }
+    __syncthreads();
+    for (int u = tid; u <= n; u += NTG) cur[u] = pos[u];
+    __syncthreads();
+    for (int j = tid; j < m; j += NTG) {
+        const int p = atomicAdd(&cur[(Ys[j] + n) >> 1], 1);
+        for (int w = 0; w < NWn; w++) Bs[p * NWn + w] = __ldg(Ar + (size_t)j * NWn + w) ^ vbs[w];
+    }
+    __syncthreads();
+}
+
+// Fitness of the neighbour with flip-set words (wq, wm) from the plan.
+__device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *sm, const GenSmem &L,
+                                        const GenScalars &gs, const int *wq, const uint32_t *wm)
+{
+    const int NWn = A.I.NWn, K = A.K;
+    const uint32_t *Bs = (const uint32_t *)(sm + L.Bs);
+    const int *cnt = (const int *)(sm + L.cnt), *pos = (const int *)(sm + L.pos);
+    const int2 *bins = (const int2 *)(sm + L.bins);
+    int f = gs.cbase;
+    for (int p = 0; p < gs.ndeep; p++) f -= 240 * gen_t(Bs + p * NWn, wq, wm);
+    for (int q = 0; q < 2; q++) {
+        const int np = gs.np[q], u0 = gs.walk0[q];
+        if (np == 0) continue;
+        unsigned long long w = 0;
+        for (int P = 0; P < np + K; P++) {
+            const int u = u0 + 2 * P;
+            if (P < np) {
+                const int p0 = pos[u], p1 = p0 + cnt[u];
+                for (int p = p0; p < p1; p++) w += 1ull << (8 * gen_t(Bs + p * NWn, wq, wm));
+            }
+            const int h = (int)(w & 0xffu);
+            const int2 bn = bins[u];  // bin u' = u - K, stored at u' + K = u
+            f += bn.y * h + abs(h - bn.x);
+            w >>= 8;
+        }
+    }
+    return f;
+}
+
+__global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
+{
+    extern __shared__ __align__(16) unsigned char sm[];
+    __shared__ GenScalars gs;
+    __shared__ int s_mv[KG_MAX];
+    const GenSmem L = gen_layout(A.I.m, A.I.n, A.I.NWn, A.K);
+    const int tid = threadIdx.x, lane = tid & 31, K = A.K, n = A.I.n;
+    const int bid = blockIdx.x, nb = gridDim.x;
+    unsigned long long *C = (unsigned long long *)(sm + L.C);
+    for (int x = tid; x <= n; x += NTG) {  // C(x, e) by Pascal's rule along e (exact in u64 here)
+        unsigned long long c = 1;
+        for (int e = 0; e <= K; e++) {
+            C[x * (K + 1) + e] = (e <= x) ? c : 0ull;
+            c = (e < x) ? c * (unsigned long long)(x - e) / (unsigned long long)(e + 1) : 0ull;
+        }
+    }
+    int *Ys = (int *)(sm + L.Y);
+    uint32_t *vbs = (uint32_t *)(sm + L.vb);
+    for (int j = tid; j < A.I.m; j += NTG) Ys[j] = A.Y[j];
+    for (int w = tid; w < A.I.NWn; w += NTG) vbs[w] = A.vb[w];
+    __syncthreads();
+    // this thread's contiguous run of ranks
+    const uint64_t span = A.M, gt = (uint64_t)bid * NTG + tid, G = (uint64_t)nb * NTG;
+    const uint32_t lo = (uint32_t)(span * gt / G), hi = (uint32_t)(span * (gt + 1) / G);
+    if (A.fit_out) {
+        gen_plan(A, sm, L, gs, s_mv, false);
+        int idx[KG_MAX], wq[KG_MAX];
+        uint32_t wm[KG_MAX];
+        if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
+        for (uint32_t r = lo; r < hi; r++) {
+            gen_masks(idx, K, wq, wm);
+            A.fit_out[r] = gen_eval(A, sm, L, gs, wq, wm);
+            if (r + 1 < hi) gen_succ(n, K, idx);
+        }
+        return;
+    }
+    int64_t f = A.fs[FS_F], best_f = A.fs[FS_BEST], best_it = A.fs[FS_BESTIT], zero_it = A.fs[FS_ZERO];
+    const int64_t t0 = A.fs[FS_T];
+    int64_t t = t0 + 1;
+    bool failed = false, pending = false;
+    unsigned long long tg = 0;
+    unsigned long long *slots = (unsigned long long *)A.slots;
+    for (; t <= t0 + A.iters; t++) {
+        if (A.stop_on_zero && f == 0) break;
+        gen_plan(A, sm, L, gs, s_mv, pending);
+        unsigned long long best = (unsigned long long)KEY_NONE;
+        int idx[KG_MAX], wq[KG_MAX];
+        uint32_t wm[KG_MAX];
+        if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
+        for (uint32_t r = lo; r < hi; r++) {
+            const bool tabu = A.until[r] >= (uint32_t)t;
+            if (!tabu || A.aspiration) {
+                gen_masks(idx, K, wq, wm);
+                const int fr = gen_eval(A, sm, L, gs, wq, wm);
+                const unsigned long long key = ((unsigned long long)(uint32_t)fr << 32) | r;
+                if ((!tabu || fr < best_f) && key < best) best = key;
+            }
+            if (r + 1 < hi) gen_succ(n, K, idx);
+        }
+        best = warp_min_k(best);
+        if (lane == 0 && best != (unsigned long long)KEY_NONE) atomicMin(&gs.key, best);
+        __syncthreads();
+        unsigned long long key = gs.key;
+        tg++;
+        if (nb > 1) {  // the counter exchange of k_search
+            if (tid == 0) {
+                unsigned long long *slot = slots + 16 * (tg % 3), *ctr = slots + 48;
+                if (key != (unsigned long long)KEY_NONE)
+                    asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
+                asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
+                const unsigned long long target = (unsigned long long)nb * tg;
+                unsigned long long seen;
+                do {
+                    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+                } while (seen < target);
+                unsigned long long gk;
+                asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
+                gs.gkey = gk;
+                if (bid == 0)
+                    asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(slots + 16 * ((tg + 2) % 3)),
+                                 "l"((unsigned long long)KEY_NONE) : "memory");
+            }
+            __syncthreads();
+            key = gs.gkey;
+        }
+        if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
+        const uint32_t r = (uint32_t)(key & 0xffffffffu);
+        f = (int64_t)(key >> 32);
+        // the owner of rank r (the thread whose run holds it) sets until[r]: exactly one writer
+        if (r >= lo && r < hi) A.until[r] = (uint32_t)(t + A.L);
+        if (bid == 0 && tid == 0) {
+            if (A.trace_r) A.trace_r[t - 1] = r;
+            if (A.trace_f) A.trace_f[t - 1] = f;
+        }
+        if (f < best_f) { best_f = f; best_it = t; }
+        if (f == 0 && zero_it < 0) zero_it = t;
+        if (tid == 0) {
+            int mi[KG_MAX];
+            gen_unrank(r, n, K, A.M, C, mi);
+            for (int q = 0; q < K; q++) s_mv[q] = mi[q];
+        }
+        pending = true;
+        __syncthreads();
+    }
+    if (pending) gen_plan(A, sm, L, gs, s_mv, true);  // applies the last move (Y, V)
+    if (bid == 0) {
+        for (int j = tid; j < A.I.m; j += NTG) A.Y[j] = Ys[j];
+        for (int w = tid; w < A.I.NWn; w += NTG) A.vb[w] = vbs[w];
+        if (tid == 0) {
+            A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
+            A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
+            if (failed) A.fs[FS_ERR] = 2;
+        }
+    }
+}
+
+__global__ void k_unrank_gen(int n, int K, uint32_t M, const int64_t *ranks, int64_t count, int32_t *out, int32_t *bad)
+{
+    extern __shared__ __align__(16) unsigned char smc[];
+    unsigned long long *C = (unsigned long long *)smc;
+    for (int x = threadIdx.x; x <= n; x += blockDim.x) {
+        unsigned long long c = 1;
+        for (int e = 0; e <= K; e++) {
+            C[x * (K + 1) + e] = (e <= x) ? c : 0ull;
+            c = (e < x) ? c * (unsigned long long)(x - e) / (unsigned long long)(e + 1) : 0ull;
+        }
+    }
+    __syncthreads();
+    for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < count; i += (int64_t)gridDim.x * blockDim.x) {
+        const int64_t r = ranks[i];
+        if (r < 0 || r >= (int64_t)M) { *bad = 1; continue; }
+        int idx[KG_MAX];
+        gen_unrank((uint32_t)r, n, K, M, C, idx);
+        for (int q = 0; q < K; q++) out[i * K + q] = idx[q];
+    }
+}
+
 }  // namespace
 
 // ==========================================================================================
@@ -1921,7 +2276,14 @@ int64_t comb_k(int64_t n, int k)
     if (k == 1) return n;
     if (k == 2) return n * (n - 1) / 2;
     if (k == 3) return n * (n - 1) * (n - 2) / 6;
-    return -1;
+    if (k < 1 || k > KG_MAX) return -1;
+    if (n < k) return 0;
+    int64_t c = 1;  // C(n, k) = prod_{i < k} (n - i) / (i + 1), exact at every step; capped
+    for (int i = 0; i < k; i++) {
+        c = c * (n - i) / (i + 1);
+        if (c > ((int64_t)1 << 40)) return INT64_MAX;
+    }
+    return c;
 }
 
 DevInst dev_inst(const lns_ctx *c) { return DevInst{c->m, c->n, c->W, c->NWn, c->W, 0, c->d_Arow, c->d_H, c->maxS}; }
@@ -2100,7 +2462,9 @@ lns_status geometry(lns_ctx *c, int k, Geometry &g, int pkw)
 lns_status check_k(lns_ctx *c, int k, Geometry &g)
 {
     if (!c) return fail(LNS_EINVAL, "null context");
-    if (k < 1 || k > 3) return fail(LNS_EINVAL, "k must be 1, 2 or 3");
+    if (k < 1 || k > 3)
+        return fail(LNS_EINVAL, k <= KG_MAX ? "k = 4..7: lns_tabu_run, lns_eval_all and lns_unrank only"
+                                            : "k must be in 1..7");
     if (c->n < k) return fail(LNS_EINVAL, "n < k");
     const int64_t Mk = comb_k(c->n, k);
     if (Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
@@ -2362,6 +2726,108 @@ lns_status dispatch_step_apply(int k, const SearchArgs &A, const int64_t *key, c
     }
 }
 
+// k = 4..7 (the generic-k kernel k_gen): limits and shared memory.
+lns_status gen_check(lns_ctx *c, int k, uint32_t &M, size_t &smem)
+{
+    if (!c) return fail(LNS_EINVAL, "null context");
+    if (k < 4 || k > KG_MAX) return fail(LNS_EINVAL, "k must be in 1..7");
+    if (c->n < k) return fail(LNS_EINVAL, "n < k");
+    if (c->m > PACKED_MAX_M) return fail(LNS_ERANGE, "k > 3 needs m <= 255 (byte window)");
+    const int64_t Mk = comb_k(c->n, k);
+    if (Mk < 0 || Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
+    M = (uint32_t)Mk;
+    smem = (size_t)gen_layout(c->m, c->n, c->NWn, k).end;
+    if (smem > (size_t)(c->smemOptin - 1024)) return fail(LNS_ERANGE, "k > 3 plan does not fit in shared memory");
+    return LNS_OK;
+}
+
+GenArgs gen_args(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L, int flags)
+{
+    GenArgs A;
+    A.I = dev_inst(c);
+    A.K = k; A.M = M; A.iters = iters; A.L = L;
+    A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
+    A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
+    A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until; A.slots = c->d_slots;
+    A.trace_r = c->d_tr; A.trace_f = c->d_tf; A.fit_out = nullptr;
+    return A;
+}
+
+lns_status resolve_tenure(int64_t M, int64_t tenure, int64_t &L);
+
+// lns_tabu_run for k = 4..7: one persistent cooperative k_gen launch (single search, one device).
+lns_status gen_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, uint64_t seed, const int8_t *V0,
+                        int32_t flags, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit, lns_result *res,
+                        void *stream)
+{
+    uint32_t M;
+    size_t smem;
+    lns_status s = gen_check(c, k, M, smem);
+    if (s != LNS_OK) return s;
+    if (!res) return fail(LNS_EINVAL, "res is required");
+    if (iters < 0 || iters >= (int64_t)INT32_MAX) return fail(LNS_EINVAL, "iters must be in [0, 2^31)");
+    if ((flags & (LNS_FORCE_STEPPED | LNS_TABU_SOLUTIONS)) || c->comm || c->nparts > 1 || c->npeers > 0)
+        return fail(LNS_EINVAL, "k > 3: one device, persistent kernel, rank tabu list (optionally aspiration) only");
+    int64_t L;
+    if ((s = resolve_tenure(M, tenure, L)) != LNS_OK) return s;
+    if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    Geometry g;
+    g.M = M;
+    if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
+    if (iters > 0) {
+        CK(allow_smem((const void *)k_gen, (int)smem));
+        int occ = 0;
+        CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
+        if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
+        int nb = (int)std::min<int64_t>(std::min(c->numSMs, MAX_SLOTS), std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
+        if (c->blocks_override > 0) nb = std::min(c->blocks_override, c->numSMs);
+        k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
+        GenArgs A = gen_args(c, k, M, iters, L, flags);
+        void *args[] = {&A};
+        CK(cudaEventRecord(c->ev0, st));
+        CK(cudaLaunchCooperativeKernel((void *)k_gen, dim3(nb), dim3(NTG), args, smem, st));
+        CK(cudaEventRecord(c->ev1, st));
+    }
+    s = search_finish(c, V_out, trace_rank, trace_fit, res, st);
+    float ms = 0;
+    if (iters > 0 && cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
+    cudaGetLastError();
+    return s;
+}
+
+// lns_eval_all for k = 4..7.
+lns_status gen_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness_out, void *stream)
+{
+    uint32_t M;
+    size_t smem;
+    lns_status s = gen_check(c, k, M, smem);
+    if (s != LNS_OK) return s;
+    if (!V || !fitness_out) return fail(LNS_EINVAL, "null argument");
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    if ((s = grow(c->d_fit, c->fit_cap, M)) != LNS_OK) return s;
+    CK(cudaMemcpyAsync(c->d_V, V, c->n, cudaMemcpyDefault, st));
+    k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, nullptr, c->d_fs);
+    CK(allow_smem((const void *)k_gen, (int)smem));
+    GenArgs A = gen_args(c, k, M, 0, 0, 0);
+    A.fit_out = c->d_fit;
+    int nb = (int)std::min<int64_t>(4LL * c->numSMs, std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
+    if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs);
+    CK(cudaEventRecord(c->ev0, st));
+    k_gen<<<nb, NTG, smem, st>>>(A);
+    CK(cudaGetLastError());
+    CK(cudaEventRecord(c->ev1, st));
+    int64_t fs[FS_N];
+    CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
+    CK(cudaMemcpyAsync(fitness_out, c->d_fit, 4 * (size_t)M, cudaMemcpyDefault, st));
+    CK(cudaStreamSynchronize(st));
+    float ms = 0; cudaEventElapsedTime(&ms, c->ev0, c->ev1); c->last_ms = ms;
+    if (fs[FS_ERR]) return fail(LNS_EINVAL, "V must be +-1");
+    return LNS_OK;
+}
+
 lns_status resolve_tenure(int64_t M, int64_t tenure, int64_t &L)
 {
     L = tenure < 0 ? M / 6 : tenure;
@@ -2422,7 +2888,7 @@ void lns_pool_stats(int64_t *cached_bytes, int64_t *live_bytes)
 
 int64_t lns_neighborhood_size(int32_t n, int32_t k)
 {
-    if (k < 1 || k > 3) return -1;
+    if (k < 1 || k > KG_MAX) return -1;
     return n < k ? 0 : comb_k(n, k);
 }
 
@@ -2655,6 +3121,7 @@ lns_status lns_eval_neighborhood(lns_ctx *c, int32_t k, const int8_t *V, const i
 
 lns_status lns_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness_out, void *stream)
 {
+    if (k >= 4) return gen_eval_all(c, k, V, fitness_out, stream);
     Geometry g;
     lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
@@ -2731,6 +3198,7 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
                         int32_t flags, int8_t *V_out, int64_t *trace_rank, int64_t *trace_fit, lns_result *res,
                         void *stream)
 {
+    if (k >= 4) return gen_tabu_run(c, k, iters, tenure, seed, V0, flags, V_out, trace_rank, trace_fit, res, stream);
     Geometry g;
     lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;
@@ -2950,6 +3418,32 @@ lns_status lns_debug_plan(lns_ctx *c, int32_t k, const int8_t *V, int32_t *out_h
 
 lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count, int32_t *out, void *stream)
 {
+    if (k >= 4 && k <= KG_MAX && n >= k) {  // generic-k unranking (k_gen's), count x k entries
+        if (count < 0 || (count > 0 && (!ranks || !out))) return fail(LNS_EINVAL, "bad buffers");
+        const int64_t Mk = comb_k(n, k);
+        if (Mk < 0 || Mk >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "C(n,k) >= 2^32-1");
+        if (count == 0) return LNS_OK;
+        cudaStream_t st = (cudaStream_t)stream;
+        int64_t *d_r = nullptr;
+        int32_t *d_o = nullptr, *d_bad = nullptr;
+        if (cudaMalloc(&d_r, count * 8) != cudaSuccess || cudaMalloc(&d_o, count * 4 * k) != cudaSuccess ||
+            cudaMalloc(&d_bad, 4) != cudaSuccess) {
+            cudaFree(d_r); cudaFree(d_o); cudaGetLastError();
+            return fail(LNS_ENOMEM, "cudaMalloc failed");
+        }
+        int bad = 0;
+        cudaMemcpyAsync(d_r, ranks, count * 8, cudaMemcpyDefault, st);
+        cudaMemsetAsync(d_bad, 0, 4, st);
+        const int blocks = (int)std::min<int64_t>((count + 255) / 256, 4096);
+        k_unrank_gen<<<blocks, 256, 8 * (size_t)(n + 1) * (k + 1), st>>>(n, k, (uint32_t)Mk, d_r, count, d_o, d_bad);
+        cudaMemcpyAsync(out, d_o, count * 4 * k, cudaMemcpyDefault, st);
+        cudaMemcpyAsync(&bad, d_bad, 4, cudaMemcpyDeviceToHost, st);
+        const cudaError_t e = cudaStreamSynchronize(st);
+        cudaFree(d_r); cudaFree(d_o); cudaFree(d_bad);
+        if (e != cudaSuccess) return fail(LNS_ECUDA, cudaGetErrorString(e));
+        if (bad) return fail(LNS_EINVAL, "rank out of range");
+        return LNS_OK;
+    }
     if (k < 1 || k > 3 || n < k) return fail(LNS_EINVAL, "bad n/k");
     if (count < 0 || (count > 0 && (!ranks || !out))) return fail(LNS_EINVAL, "bad buffers");
     const int64_t Mk = comb_k(n, k);

@@ -51,7 +51,9 @@ def test_host_only_entry_points():
     for n in (1, 3, 21, 117, 1024, 2954):
         for k in (1, 2, 3):
             assert L.lns_neighborhood_size(n, k) == comb(n, k)
-    assert L.lns_neighborhood_size(10, 4) == -1
+    for n, k in ((10, 4), (500, 4), (80, 7)):  # k > 3 (the generic-k path)
+        assert L.lns_neighborhood_size(n, k) == comb(n, k)
+    assert L.lns_neighborhood_size(10, 8) == -1
     assert L.lns_strerror(L.LNS_ENOADMISSIBLE) == "no admissible neighbour"
     cached, live = L.lns_pool_stats()  # host-only: the device-memory cache's counters
     assert cached >= 0 and live >= 0

@@ -679,3 +679,71 @@ def test_compute_sanitizer_clean(L, tool):
     assert "sanitize probe done" in out.stdout, tail
     log = out.stdout + out.stderr
     assert "ERROR SUMMARY: 0 errors" in log or "SUMMARY: 0 hazards displayed (0 errors" in log, tail
+
+
+# ------------------------------------------------------------------ k > 3
+@pytest.mark.parametrize("k", [4, 5, 6, 7])
+def test_unrank_k_above_3_exhaustive(L, orc, k):
+    for n in (k, k + 1, 13, 30 if k < 7 else 24):
+        M = comb(n, k)
+        r = np.arange(M, dtype=np.int64)
+        assert np.array_equal(L.lns_unrank(n, k, r), orc.flipsets(n, k, r))
+
+
+@pytest.mark.parametrize("n,k", [(500, 4), (200, 5), (120, 6), (80, 7)])
+def test_unrank_k_above_3_sampled_large(L, n, k):
+    """Large n: sampled ranks (both ends included) map to strictly increasing index tuples whose
+    lexicographic rank, restated with math.comb, is the rank itself."""
+    M = comb(n, k)
+    rng = np.random.default_rng(n + k)
+    r = np.unique(np.concatenate([[0, 1, M - 2, M - 1], rng.integers(0, M, 3000)])).astype(np.int64)
+    F = L.lns_unrank(n, k, r)
+    assert np.all(np.diff(F, axis=1) > 0) and F.min() >= 0 and F.max() < n
+    for q in range(0, len(r), 97):
+        lex = M - 1 - sum(comb(n - 1 - int(F[q, j]), k - j) for j in range(k))
+        assert lex == r[q]
+
+
+@pytest.mark.parametrize("m,n,k", [(41, 35, 4), (70, 40, 4), (33, 23, 5), (100, 20, 6), (255, 18, 7)])
+def test_eval_all_k_above_3_matches_oracle(L, orc, m, n, k):
+    """Every neighbour's fitness for k = 4..7 (random, near-secret, all-negative and secret
+    states: deep rows, rows above the top cut, empty lattice points, m up to 255)."""
+    inst = pi.planted_instance(m, n, 4000 + m + k)
+    rng = np.random.default_rng(m * n + k)
+    with L.Instance(inst.A, inst.S) as I:
+        for V in _states(inst, rng, count=1):
+            got = L.lns_eval_all(I.ctx, k, V).astype(np.int64)
+            assert np.array_equal(got, orc.eval_all(inst.A, inst.S, V, k))
+
+
+@pytest.mark.parametrize("k,ten,iters,blocks", [(4, -1, 30, 0), (4, 5, 40, 3), (5, 0, 20, 1), (6, 50, 12, 0)])
+@pytest.mark.parametrize("aspiration", [False, True])
+def test_trajectory_k_above_3_bit_exact(L, orc, k, ten, iters, blocks, aspiration):
+    inst = pi.planted_instance(45, 29, 5000 + k)
+    V0 = pi.start_vector(29, 30 + k)
+    t_or = pi.default_tenure(29, k) if ten < 0 else ten
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0, iters, t_or, stop_on_zero=False, aspiration=aspiration)
+    with L.Instance(inst.A, inst.S) as I:
+        L.lns_config(I.ctx, blocks)
+        tr, tf, Vo, res = I.tabu_run(k, iters, ten, V0=V0, stop_on_zero=False,
+                                     flags=L.LNS_ASPIRATION if aspiration else 0)
+    assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+
+
+def test_k_above_3_limits(L):
+    inst = pi.planted_instance(300, 20, 9)
+    small = pi.planted_instance(20, 12, 9)
+    with L.Instance(inst.A, inst.S) as I:
+        with pytest.raises(L.LnsError) as ei:
+            I.tabu_run(4, 3, -1, seed=1)
+        assert ei.value.status == L.LNS_ERANGE  # m > 255
+    with L.Instance(small.A, small.S) as I:
+        for call in (lambda: L.lns_tabu_run_batch(I.ctx, 4, 2, 3, -1, 0, None, 0),
+                     lambda: I.tabu_run(8, 3, -1, seed=1),
+                     lambda: I.tabu_run(4, 3, -1, seed=1, flags=L.LNS_FORCE_STEPPED),
+                     lambda: I.tabu_run(4, 3, 2, seed=1, flags=L.LNS_TABU_SOLUTIONS)):
+            with pytest.raises(L.LnsError) as ei:
+                call()
+            assert ei.value.status == L.LNS_EINVAL
+        res = I.tabu_run(4, 5, -1, seed=1, stop_on_zero=False)[3]
+        assert res["iters_done"] == 5
