@@ -2220,6 +2220,7 @@ struct lns_ctx {
     int blocks_override = 0;
     int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
     int no_pkw = 0;  // LNS_NO_PKW=1 at create: m > 255 always takes the segment plan (A/B measurement)
+    int force_pkw = 0;  // LNS_FORCE_PKW=1 at create: m > 255 tries the packed plan for any slice size
     // device-initiated exchange (lns_attach_peers)
     unsigned long long *d_xbuf = nullptr;            // own 64-word exchange buffer (its own allocation)
     unsigned long long **d_peers = nullptr;          // device array of the partitions' buffers
@@ -2420,6 +2421,7 @@ struct Geometry {
     int x_global = 0;      // X does not fit in shared memory: per-CTA slots in global memory
     int pad = 0, XW = 0;   // padded placement (packed path, when X of 2W + 1 words fits)
     int pkw = 0;           // m > 255: packed records allocated, the packed plan tried per iteration
+    int pkw_force = 0;     // LNS_FORCE_PKW=1 at create: try it for any slice size (tests)
     size_t smem_eval = 0;  // bytes for the stepped / eval kernels
 };
 
@@ -2477,6 +2479,7 @@ lns_status check_k(lns_ctx *c, int k, Geometry &g)
         if (geometry(c, k, g0, 0) == LNS_OK && (s != LNS_OK || !g0.x_global)) { g = g0; s = LNS_OK; }
     }
     if (s != LNS_OK) return s;
+    g.pkw_force = c->force_pkw;
     if (g.x_global) {  // one X slot per CTA of the largest grid any launch uses (eval_all: 8 x SMs)
         s = grow(c->d_X, c->X_cap, (size_t)8 * c->numSMs * c->W * c->n);
         if (s != LNS_OK) return s;
@@ -2613,6 +2616,13 @@ cudaError_t allow_smem(const void *fn, int bytes)
 
 // Padded placement pays off when a CTA evaluates many neighbours per plan (it adds a serial warp
 // pass to every plan build): the same slice test as the contiguous-run evaluation path.
+// m > 255: the packed plan (§5.11) pays off when a CTA evaluates many neighbours per plan (its
+// build adds a barrier and a serial placement); otherwise the segment plan is used throughout.
+inline int pkw_for(const Geometry &g, uint32_t span, int nb)
+{
+    return (g.pkw && (g.pkw_force || span / (uint32_t)std::max(nb, 1) >= 2u * NT)) ? 1 : 0;
+}
+
 inline int pad_for(const Geometry &g, uint32_t span, int nb)
 {
     return (g.pad && span / (uint32_t)std::max(nb, 1) >= 4u * NT) ? 1 : 0;
@@ -2631,6 +2641,7 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     const int nb = nb_force > 0 ? nb_force : search_blocks(c, A.hi - A.lo, 1);
     if (A.npeers > 0) A.nb_total = (int64_t)nb * A.npeers;
     A.I.pad = pad_for(g, A.hi - A.lo, nb);
+    A.I.pkw = pkw_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
     k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
@@ -2650,6 +2661,7 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int grid, i
     const int budget = c->smemOptin - 1024;
     CK(allow_smem((const void *)k_search<K>, budget));
     A.I.pad = pad_for(g, A.hi - A.lo, nb_min);
+    A.I.pkw = pkw_for(g, A.hi - A.lo, nb_min);
     const size_t smem = cache_geometry(A, g, nb_min, budget);
     if (!A.until_smem) {  // one global until[] per group of every phase
         lns_status s = grow(c->d_until, c->until_cap, (size_t)ngroups * g.M);
@@ -2683,9 +2695,11 @@ lns_status launch_step_eval(lns_ctx *c, const SearchArgs &A, const Geometry &g, 
         nb = (int)std::min<int64_t>(std::max<int64_t>(1, (A.hi - A.lo) / 1024), 4LL * c->numSMs * occ);
         if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs * occ);
         a.I.pad = pad_for(g, A.hi - A.lo, nb);
+        a.I.pkw = pkw_for(g, A.hi - A.lo, nb);
         k_step_eval<K, true><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     } else {
         a.I.pad = pad_for(g, A.hi - A.lo, nb);
+        a.I.pkw = pkw_for(g, A.hi - A.lo, nb);
         k_step_eval<K, false><<<nb, NT, g.smem_eval, st>>>(a, key_out, fit_out);
     }
     CK(cudaGetLastError());
@@ -2924,6 +2938,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     c->device = device; c->m = m; c->n = n; c->W = W; c->NWn = NWn;
     { const char *e = getenv("LNS_NO_PAD"); c->no_pad = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_NO_PKW"); c->no_pkw = (e && e[0] == '1') ? 1 : 0; }
+    { const char *e = getenv("LNS_FORCE_PKW"); c->force_pkw = (e && e[0] == '1') ? 1 : 0; }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };

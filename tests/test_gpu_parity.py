@@ -259,7 +259,7 @@ def _clustered_instance(m, n, npool, noise, seed):
 @pytest.mark.parametrize("k,iters,m,npool,noise", [(1, 150, 700, 10, 0.1), (2, 60, 550, 8, 0.12),
                                                    (3, 25, 500, 8, 0.12)])
 @pytest.mark.parametrize("blocks", [1, 5])
-def test_large_m_packed_plan_guard_mixed_trajectory(L, orc, k, iters, m, npool, noise, blocks):
+def test_large_m_packed_plan_guard_mixed_trajectory(L, orc, k, iters, m, npool, noise, blocks, monkeypatch):
     """m > 255: each iteration takes the packed byte-window plan when the
     state's counts fit bytes and the segment plan otherwise. On these clustered instances the
     guard (restated in tests/test_packed_model.bytes_fit) switches along the trajectory; the
@@ -279,6 +279,7 @@ def test_large_m_packed_plan_guard_mixed_trajectory(L, orc, k, iters, m, npool, 
             if i >= 0:
                 V[i] = -V[i]
     assert 0 < sum(fits) < iters  # both plans are taken
+    monkeypatch.setenv("LNS_FORCE_PKW", "1")  # small slices too (read at create)
     with L.Instance(A, S) as I:
         L.lns_config(I.ctx, blocks)
         tr, tf, Vo, res = I.tabu_run(k, iters, -1, V0=V0, stop_on_zero=False)
@@ -538,6 +539,24 @@ def test_eval_all_large_slices(L, orc, m, n, k):
             got = L.lns_eval_all(ctx, k, V)
             want = orc.eval_all(inst.A, inst.S, V, k)
             assert np.array_equal(got.astype(np.int64), want)
+    finally:
+        L.lns_destroy(ctx)
+
+
+@pytest.mark.parametrize("m,n,k", [(300, 50, 3), (260, 40, 2), (520, 64, 1), (1024, 200, 2), (700, 90, 3)])
+@pytest.mark.parametrize("plan", ["LNS_FORCE_PKW", "LNS_NO_PKW"])
+def test_eval_all_large_m_both_plans(L, orc, m, n, k, plan, monkeypatch):
+    """m > 255: every fitness with the packed plan tried on every slice
+    (LNS_FORCE_PKW; states whose counts fit bytes take it) and with the segment plan only
+    (LNS_NO_PKW), against the oracle."""
+    monkeypatch.setenv(plan, "1")
+    inst = pi.planted_instance(m, n, 8100 + m + n + k)
+    rng = np.random.default_rng(m + n + k)
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        for V in _states(inst, rng, count=1):
+            got = L.lns_eval_all(ctx, k, V)
+            assert np.array_equal(got.astype(np.int64), orc.eval_all(inst.A, inst.S, V, k))
     finally:
         L.lns_destroy(ctx)
 
