@@ -1851,11 +1851,11 @@ __global__ void k_bits_to_until(const uint32_t *bits, uint32_t *until, uint32_t 
 // A compact variant of the same method: exact combinatorial unranking for any k (the complement
 // identity lex_rank(i_1 < .. < i_k) = M - 1 - sum_j C(n-1-i_j, k-j+1), u64 tables, binary
 // search per position), lexicographic successor stepping over each thread's contiguous run of
-// ranks, and the parity walks of §5.9 evaluated ROW by row: a walked row of lattice point u with
-// t = #{i in F : x_ji = 1} (one AND + POPC per column word F touches) adds 1 to byte t of a
-// 64-bit window (bins u, u+2, .., u+2k of its walk: k+1 <= 8 bytes, counts <= m <= 255); when a
-// point's rows are done its bin (byte 0) is complete: f += w_b h + |h - H_b|, and the window
-// shifts by one byte. Deep rows (Y < -2k) cost 60(2k - Y) - 240 t, rows above max(S) + 2k cost 1,
+// ranks, and the parity walks of §5.9 over (point, row word) pieces: the k columns of a row word
+// are summed into three bit planes of t = #{i in F : x_ji = 1}, and a piece adds
+// sum_rows 256^t (k masked plane-product POPCs) to a 64-bit window (bins u, u+2, .., u+2k of its
+// walk: k+1 <= 8 bytes, counts <= m <= 255); when a point's last piece is done its bin (byte 0)
+// is complete: f += w_b h + |h - H_b|, and the window shifts by one byte. Deep rows (Y < -2k) cost 60(2k - Y) - 240 t, rows above max(S) + 2k cost 1,
 // bins of [0, n] outside both walks cost H_b. One persistent cooperative kernel per search, the
 // same (f << 32 | r) key, warp/CTA argmin and counter exchange as k_search.
 // ------------------------------------------------------------------------------------------
@@ -1878,7 +1878,7 @@ struct GenArgs {
 };
 
 struct GenSmem {
-    int Bs, Y, vb, cnt, pos, cur, bins, C, end;
+    int Bs, Y, vb, cnt, pos, cur, bins, C, X, pc, end;
 };
 
 __host__ __device__ inline GenSmem gen_layout(int m, int n, int NWn, int K)
@@ -1893,12 +1893,16 @@ __host__ __device__ inline GenSmem gen_layout(int m, int n, int NWn, int K)
     s.cur = o;  o = align16(o + 4 * (n + 1));
     s.bins = o; o = align16(o + 8 * (n + 2 * K + 1));   // (H_b, w_b) of bin u' in [-K, n + K]
     s.C = o;    o = align16(o + 8 * (n + 1) * (K + 1)); // C(x, e), x <= n, e <= K (u64)
+    const int W = (m + 31) >> 5;
+    s.X = o;    o = align16(o + 4 * W * n);             // X[w][c]: column c's bits of sorted rows 32w..
+    s.pc = o;   o = align16(o + 8 * 2 * (n + 3 + 2 * W)); // pieces of both walks (uint2)
     s.end = o;
     return s;
 }
 
 struct GenScalars {
     int ua, np[2], ndeep, ntop, walk0[2];
+    int pc0[2], pc1[2];  // pieces of walk q: [pc0[q], pc1[q])
     int cbase;  // m - (H of the walked bins) + 60 sum_deep (2K - Y) + #top rows
     unsigned long long key, gkey;
 };
@@ -1937,36 +1941,6 @@ __device__ __forceinline__ void gen_succ(int n, int K, int *idx)
         if (q == j) idx[q]++;
         else if (q > 0 && q > j && q < K) idx[q] = idx[q - 1] + 1;
     }
-}
-
-// The flip set as column-word masks: wq[j] = word of idx[j]; wm[j] = the bits of every index in
-// that word if j is the first index there, else 0 (indices ascend, so a word's indices are
-// consecutive). Static indexing only.
-__device__ __forceinline__ void gen_masks(const int *idx, int K, int *wq, uint32_t *wm)
-{
-#pragma unroll
-    for (int j = 0; j < KG_MAX; j++) {
-        wq[j] = j < K ? idx[j] >> 5 : 0;
-        wm[j] = 0;
-    }
-#pragma unroll
-    for (int j = 0; j < KG_MAX; j++) {
-        if (j < K && (j == 0 || wq[j] != wq[j > 0 ? j - 1 : 0])) {
-#pragma unroll
-            for (int q = j; q < KG_MAX; q++)
-                if (q < K && wq[q] == wq[j]) wm[j] |= 1u << (idx[q] & 31);
-        }
-    }
-}
-
-// t = #{i in F : x_ji = 1} for the sorted row brow.
-__device__ __forceinline__ int gen_t(const uint32_t *__restrict__ brow, const int *wq, const uint32_t *wm)
-{
-    int t = 0;
-#pragma unroll
-    for (int e = 0; e < KG_MAX; e++)
-        if (wm[e]) t += __popc(brow[wq[e]] & wm[e]);
-    return t;
 }
 
 // Plan of the current (Y, V): apply the pending move first (pending = K indices, or none).
@@ -2033,32 +2007,105 @@ __device__ void gen_plan(const GenArgs &A, unsigned char *sm, const GenSmem &L, 
         for (int w = 0; w < NWn; w++) Bs[p * NWn + w] = __ldg(Ar + (size_t)j * NWn + w) ^ vbs[w];
     }
     __syncthreads();
+    // X[w][c] = column c's bits over sorted rows 32w .. 32w+31 (row-major Bs transposed), and the
+    // pieces of each walk: (mask, word | last << 15 | popc(mask) << 16) per (point, row word), an
+    // empty point one zero piece that only completes its bin
+    uint32_t *X = (uint32_t *)(sm + L.X);
+    const int W = (m + 31) >> 5;
+    for (int e = tid; e < W * n; e += NTG) {
+        const int w = e / n, c = e - w * n;
+        uint32_t x = 0;
+        for (int l = 0; l < 32 && 32 * w + l < m; l++)
+            x |= ((Bs[(32 * w + l) * NWn + (c >> 5)] >> (c & 31)) & 1u) << l;
+        X[e] = x;
+    }
+    if (tid == 0) {
+        uint2 *pc = (uint2 *)(sm + L.pc);
+        int np_ = 0;
+        for (int q = 0; q < 2; q++) {
+            gs.pc0[q] = np_;
+            int lastw = 0;
+            for (int P = 0; P < gs.np[q]; P++) {
+                const int u = gs.walk0[q] + 2 * P, st = pos[u], en = st + cnt[u];
+                if (en == st) { pc[np_++] = make_uint2(0u, (uint32_t)lastw | (1u << 15)); continue; }
+                for (int w = st >> 5; w <= (en - 1) >> 5; w++) {
+                    const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
+                    const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
+                    pc[np_++] = make_uint2(mask, (uint32_t)w | ((w == (en - 1) >> 5) ? 1u << 15 : 0u) |
+                                                     ((uint32_t)__popc(mask) << 16));
+                    lastw = w;
+                }
+            }
+            gs.pc1[q] = np_;
+        }
+    }
+    __syncthreads();
 }
 
-// Fitness of the neighbour with flip-set words (wq, wm) from the plan.
-__device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *sm, const GenSmem &L,
-                                        const GenScalars &gs, const int *wq, const uint32_t *wm)
+// Bit-sliced planes of t = #{i in F : x_i = 1} over one row word (t <= 7: three planes).
+__device__ __forceinline__ void gen_planes(const uint32_t *__restrict__ xw, const int *idx, int K, uint32_t &b0,
+                                           uint32_t &b1, uint32_t &b2)
 {
-    const int NWn = A.I.NWn, K = A.K;
-    const uint32_t *Bs = (const uint32_t *)(sm + L.Bs);
-    const int *cnt = (const int *)(sm + L.cnt), *pos = (const int *)(sm + L.pos);
+    b0 = 0; b1 = 0; b2 = 0;
+#pragma unroll
+    for (int j = 0; j < KG_MAX; j++) {
+        if (j < K) {
+            const uint32_t x = xw[idx[j]];
+            const uint32_t c0 = b0 & x;
+            b0 ^= x;
+            b2 |= b1 & c0;
+            b1 ^= c0;
+        }
+    }
+}
+
+// Fitness of the neighbour idx[0..K) from the plan. Per piece (the rows of one lattice point in
+// one row word, mask m) the walk window gains sum_rows 256^t = popc(m) + sum (256^t - 1), and with
+// t = b0 + 2 b1 + 4 b2: 256^t - 1 = (1 + 255 b0)(1 + 65535 b1)(1 + (2^32 - 1) b2) - 1, i.e. seven
+// masked plane products (those K cannot reach vanish: K = 4 needs 4 POPCs, 5: 5, 6: 6, 7: 7).
+__device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *sm, const GenSmem &L,
+                                        const GenScalars &gs, const int *idx)
+{
+    const int K = A.K, n = A.I.n;
+    const uint32_t *X = (const uint32_t *)(sm + L.X);
+    const uint2 *pc = (const uint2 *)(sm + L.pc);
     const int2 *bins = (const int2 *)(sm + L.bins);
     int f = gs.cbase;
-    for (int p = 0; p < gs.ndeep; p++) f -= 240 * gen_t(Bs + p * NWn, wq, wm);
+    uint32_t b0, b1, b2;
+    for (int w = 0, nd = gs.ndeep; 32 * w < nd; w++) {  // deep rows: -240 sum t
+        gen_planes(X + w * n, idx, K, b0, b1, b2);
+        const uint32_t dm = (nd - 32 * w >= 32) ? FULL : ((1u << (nd - 32 * w)) - 1u);
+        f -= 240 * (__popc(b0 & dm) + 2 * __popc(b1 & dm) + 4 * __popc(b2 & dm));
+    }
     for (int q = 0; q < 2; q++) {
-        const int np = gs.np[q], u0 = gs.walk0[q];
-        if (np == 0) continue;
-        unsigned long long w = 0;
-        for (int P = 0; P < np + K; P++) {
-            const int u = u0 + 2 * P;
-            if (P < np) {
-                const int p0 = pos[u], p1 = p0 + cnt[u];
-                for (int p = p0; p < p1; p++) w += 1ull << (8 * gen_t(Bs + p * NWn, wq, wm));
+        if (gs.np[q] == 0) continue;
+        unsigned long long win = 0;
+        int curw = -1, u = gs.walk0[q];
+        for (int e = gs.pc0[q]; e < gs.pc1[q]; e++) {
+            const uint2 pr = pc[e];
+            const int w = (int)(pr.y & 0x7fffu);
+            if (w != curw) { gen_planes(X + w * n, idx, K, b0, b1, b2); curw = w; }
+            const uint32_t m = pr.x;
+            unsigned long long d = (unsigned long long)(pr.y >> 16);
+            d += 255ull * __popc(b0 & m) + 65535ull * __popc(b1 & m) + 16711425ull * __popc(b0 & b1 & m);
+            if (K >= 4) d += 4294967295ull * __popc(b2 & m);
+            if (K >= 5) d += 1095216660225ull * __popc(b0 & b2 & m);     // 255 (2^32 - 1)
+            if (K >= 6) d += 281470681677825ull * __popc(b1 & b2 & m);  // 65535 (2^32 - 1)
+            if (K >= 7) d += 71775023827845375ull * __popc(b0 & b1 & b2 & m);  // 255 * 65535 (2^32 - 1)
+            win += d;
+            if (pr.y & (1u << 15)) {  // the point's last piece: its bin is complete
+                const int h = (int)(win & 0xffu);
+                const int2 bn = bins[u];  // bin u' = u - K, stored at u' + K = u
+                f += bn.y * h + abs(h - bn.x);
+                win >>= 8;
+                u += 2;
             }
-            const int h = (int)(w & 0xffu);
-            const int2 bn = bins[u];  // bin u' = u - K, stored at u' + K = u
+        }
+        for (int P = 0; P < K; P++, u += 2) {  // trailing bins: rows carried past the last point
+            const int h = (int)(win & 0xffu);
+            const int2 bn = bins[u];
             f += bn.y * h + abs(h - bn.x);
-            w >>= 8;
+            win >>= 8;
         }
     }
     return f;
@@ -2090,12 +2137,10 @@ __global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
     const uint32_t lo = (uint32_t)(span * gt / G), hi = (uint32_t)(span * (gt + 1) / G);
     if (A.fit_out) {
         gen_plan(A, sm, L, gs, s_mv, false);
-        int idx[KG_MAX], wq[KG_MAX];
-        uint32_t wm[KG_MAX];
+        int idx[KG_MAX];
         if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
         for (uint32_t r = lo; r < hi; r++) {
-            gen_masks(idx, K, wq, wm);
-            A.fit_out[r] = gen_eval(A, sm, L, gs, wq, wm);
+            A.fit_out[r] = gen_eval(A, sm, L, gs, idx);
             if (r + 1 < hi) gen_succ(n, K, idx);
         }
         return;
@@ -2110,14 +2155,12 @@ __global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
         if (A.stop_on_zero && f == 0) break;
         gen_plan(A, sm, L, gs, s_mv, pending);
         unsigned long long best = (unsigned long long)KEY_NONE;
-        int idx[KG_MAX], wq[KG_MAX];
-        uint32_t wm[KG_MAX];
+        int idx[KG_MAX];
         if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
         for (uint32_t r = lo; r < hi; r++) {
             const bool tabu = A.until[r] >= (uint32_t)t;
             if (!tabu || A.aspiration) {
-                gen_masks(idx, K, wq, wm);
-                const int fr = gen_eval(A, sm, L, gs, wq, wm);
+                const int fr = gen_eval(A, sm, L, gs, idx);
                 const unsigned long long key = ((unsigned long long)(uint32_t)fr << 32) | r;
                 if ((!tabu || fr < best_f) && key < best) best = key;
             }
