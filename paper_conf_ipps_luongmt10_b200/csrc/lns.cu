@@ -1875,6 +1875,12 @@ struct GenArgs {
     int64_t *slots;
     int64_t *trace_r, *trace_f;
     int32_t *fit_out;  // non-null: write every rank's fitness (lns_eval_all), no search
+    // batched restarts (R > 0): G groups of nbg CTAs; until[] of M entries and 64 exchange slots
+    // per group; restart r from V0s + r n, results into res + r FS_N and vouts + r NWn
+    int32_t R, G, nbg;
+    const int8_t *V0s;
+    int64_t *res;
+    uint32_t *vouts;
 };
 
 struct GenSmem {
@@ -2116,9 +2122,14 @@ __global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ GenScalars gs;
     __shared__ int s_mv[KG_MAX];
+    __shared__ int s_pen, s_hd;
     const GenSmem L = gen_layout(A.I.m, A.I.n, A.I.NWn, A.K);
-    const int tid = threadIdx.x, lane = tid & 31, K = A.K, n = A.I.n;
-    const int bid = blockIdx.x, nb = gridDim.x;
+    const int tid = threadIdx.x, lane = tid & 31, K = A.K, n = A.I.n, m = A.I.m, NWn = A.I.NWn;
+    // batched restarts (A.R > 0): group g = CTAs [g nbg, (g+1) nbg) runs restarts g, g + G, ...
+    const bool batch = A.R > 0;
+    const int nbg = batch ? A.nbg : (int)gridDim.x;
+    const int g = (int)blockIdx.x / nbg, bid = (int)blockIdx.x - g * nbg;
+    if (batch && g >= A.G) return;
     unsigned long long *C = (unsigned long long *)(sm + L.C);
     for (int x = tid; x <= n; x += NTG) {  // C(x, e) by Pascal's rule along e (exact in u64 here)
         unsigned long long c = 1;
@@ -2129,12 +2140,14 @@ __global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
     }
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
-    for (int j = tid; j < A.I.m; j += NTG) Ys[j] = A.Y[j];
-    for (int w = tid; w < A.I.NWn; w += NTG) vbs[w] = A.vb[w];
+    if (!batch) {
+        for (int j = tid; j < m; j += NTG) Ys[j] = A.Y[j];
+        for (int w = tid; w < NWn; w += NTG) vbs[w] = A.vb[w];
+    }
     __syncthreads();
-    // this thread's contiguous run of ranks
-    const uint64_t span = A.M, gt = (uint64_t)bid * NTG + tid, G = (uint64_t)nb * NTG;
-    const uint32_t lo = (uint32_t)(span * gt / G), hi = (uint32_t)(span * (gt + 1) / G);
+    // this thread's contiguous run of ranks (within its group)
+    const uint64_t span = A.M, gt = (uint64_t)bid * NTG + tid, Gt = (uint64_t)nbg * NTG;
+    const uint32_t lo = (uint32_t)(span * gt / Gt), hi = (uint32_t)(span * (gt + 1) / Gt);
     if (A.fit_out) {
         gen_plan(A, sm, L, gs, s_mv, false);
         int idx[KG_MAX];
@@ -2145,81 +2158,127 @@ __global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
         }
         return;
     }
-    int64_t f = A.fs[FS_F], best_f = A.fs[FS_BEST], best_it = A.fs[FS_BESTIT], zero_it = A.fs[FS_ZERO];
-    const int64_t t0 = A.fs[FS_T];
-    int64_t t = t0 + 1;
-    bool failed = false, pending = false;
-    unsigned long long tg = 0;
-    unsigned long long *slots = (unsigned long long *)A.slots;
-    for (; t <= t0 + A.iters; t++) {
-        if (A.stop_on_zero && f == 0) break;
-        gen_plan(A, sm, L, gs, s_mv, pending);
-        unsigned long long best = (unsigned long long)KEY_NONE;
-        int idx[KG_MAX];
-        if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
-        for (uint32_t r = lo; r < hi; r++) {
-            const bool tabu = A.until[r] >= (uint32_t)t;
-            if (!tabu || A.aspiration) {
-                const int fr = gen_eval(A, sm, L, gs, idx);
-                const unsigned long long key = ((unsigned long long)(uint32_t)fr << 32) | r;
-                if ((!tabu || fr < best_f) && key < best) best = key;
-            }
-            if (r + 1 < hi) gen_succ(n, K, idx);
-        }
-        best = warp_min_k(best);
-        if (lane == 0 && best != (unsigned long long)KEY_NONE) atomicMin(&gs.key, best);
-        __syncthreads();
-        unsigned long long key = gs.key;
-        tg++;
-        if (nb > 1) {  // the counter exchange of k_search
-            if (tid == 0) {
-                unsigned long long *slot = slots + 16 * (tg % 3), *ctr = slots + 48;
-                if (key != (unsigned long long)KEY_NONE)
-                    asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
-                asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
-                const unsigned long long target = (unsigned long long)nb * tg;
-                unsigned long long seen;
-                do {
-                    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
-                } while (seen < target);
-                unsigned long long gk;
-                asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
-                gs.gkey = gk;
-                if (bid == 0)
-                    asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(slots + 16 * ((tg + 2) % 3)),
-                                 "l"((unsigned long long)KEY_NONE) : "memory");
-            }
+    uint32_t *until = A.until + (batch ? (size_t)g * A.M : 0);
+    unsigned long long *slots = (unsigned long long *)A.slots + 64 * (size_t)g;
+    unsigned long long tg = 0;  // exchanges of this group (monotonic across its restarts)
+    for (int rs = batch ? g : 0; rs < (batch ? A.R : 1); rs += (batch ? A.G : 1)) {
+        int64_t f, best_f, best_it, zero_it, t0;
+        if (batch) {
+            // restart rs from V0s[rs]: V bits, Y = A V, f from scratch
+            int *hist = (int *)(sm + L.cnt);
+            for (int w = tid; w < NWn; w += NTG) vbs[w] = 0u;
+            for (int b = tid; b <= n; b += NTG) hist[b] = 0;
+            if (tid == 0) { s_pen = 0; s_hd = 0; }
             __syncthreads();
-            key = gs.gkey;
+            const int8_t *V0 = A.V0s + (size_t)rs * n;
+            for (int i = tid; i < n; i += NTG)
+                if (V0[i] < 0) atomicOr(&vbs[i >> 5], 1u << (i & 31));
+            __syncthreads();
+            int pen = 0;
+            for (int j = tid; j < m; j += NTG) {
+                int d = 0;
+                for (int w = 0; w < NWn; w++) d += __popc(__ldg(A.I.Arow + (size_t)j * NWn + w) ^ vbs[w]);
+                const int y = n - 2 * d;
+                Ys[j] = y;
+                if (y < 0) pen += -2 * y;
+                else atomicAdd(&hist[y], 1);
+            }
+            atomicAdd(&s_pen, pen);
+            __syncthreads();
+            int hd = 0;
+            for (int b = tid; b <= n; b += NTG) hd += abs(A.I.H[b] - hist[b]);
+            atomicAdd(&s_hd, hd);
+            for (uint32_t r = lo; r < hi; r++) until[r] = 0u;  // this thread's ranks only
+            __syncthreads();
+            f = 30 * (int64_t)s_pen + s_hd;
+            best_f = f; best_it = 0; zero_it = (f == 0) ? 0 : -1; t0 = 0;
+        } else {
+            f = A.fs[FS_F]; best_f = A.fs[FS_BEST]; best_it = A.fs[FS_BESTIT]; zero_it = A.fs[FS_ZERO];
+            t0 = A.fs[FS_T];
         }
-        if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
-        const uint32_t r = (uint32_t)(key & 0xffffffffu);
-        f = (int64_t)(key >> 32);
-        // the owner of rank r (the thread whose run holds it) sets until[r]: exactly one writer
-        if (r >= lo && r < hi) A.until[r] = (uint32_t)(t + A.L);
-        if (bid == 0 && tid == 0) {
-            if (A.trace_r) A.trace_r[t - 1] = r;
-            if (A.trace_f) A.trace_f[t - 1] = f;
+        int64_t t = t0 + 1;
+        bool failed = false, pending = false;
+        for (; t <= t0 + A.iters; t++) {
+            if (A.stop_on_zero && f == 0) break;
+            gen_plan(A, sm, L, gs, s_mv, pending);
+            unsigned long long best = (unsigned long long)KEY_NONE;
+            int idx[KG_MAX];
+            if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
+            for (uint32_t r = lo; r < hi; r++) {
+                const bool tabu = until[r] >= (uint32_t)t;
+                if (!tabu || A.aspiration) {
+                    const int fr = gen_eval(A, sm, L, gs, idx);
+                    const unsigned long long key = ((unsigned long long)(uint32_t)fr << 32) | r;
+                    if ((!tabu || fr < best_f) && key < best) best = key;
+                }
+                if (r + 1 < hi) gen_succ(n, K, idx);
+            }
+            best = warp_min_k(best);
+            if (lane == 0 && best != (unsigned long long)KEY_NONE) atomicMin(&gs.key, best);
+            __syncthreads();
+            unsigned long long key = gs.key;
+            tg++;
+            if (nbg > 1) {  // the counter exchange of k_search, per group
+                if (tid == 0) {
+                    unsigned long long *slot = slots + 16 * (tg % 3), *ctr = slots + 48;
+                    if (key != (unsigned long long)KEY_NONE)
+                        asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
+                    asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
+                    const unsigned long long target = (unsigned long long)nbg * tg;
+                    unsigned long long seen;
+                    do {
+                        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+                    } while (seen < target);
+                    unsigned long long gk;
+                    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
+                    gs.gkey = gk;
+                    if (bid == 0)
+                        asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(slots + 16 * ((tg + 2) % 3)),
+                                     "l"((unsigned long long)KEY_NONE) : "memory");
+                }
+                __syncthreads();
+                key = gs.gkey;
+            }
+            if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
+            const uint32_t r = (uint32_t)(key & 0xffffffffu);
+            f = (int64_t)(key >> 32);
+            // the owner of rank r (the thread whose run holds it) sets until[r]: exactly one writer
+            if (r >= lo && r < hi) until[r] = (uint32_t)(t + A.L);
+            if (!batch && bid == 0 && tid == 0) {
+                if (A.trace_r) A.trace_r[t - 1] = r;
+                if (A.trace_f) A.trace_f[t - 1] = f;
+            }
+            if (f < best_f) { best_f = f; best_it = t; }
+            if (f == 0 && zero_it < 0) zero_it = t;
+            if (tid == 0) {
+                int mi[KG_MAX];
+                gen_unrank(r, n, K, A.M, C, mi);
+                for (int q = 0; q < K; q++) s_mv[q] = mi[q];
+            }
+            pending = true;
+            __syncthreads();
         }
-        if (f < best_f) { best_f = f; best_it = t; }
-        if (f == 0 && zero_it < 0) zero_it = t;
-        if (tid == 0) {
-            int mi[KG_MAX];
-            gen_unrank(r, n, K, A.M, C, mi);
-            for (int q = 0; q < K; q++) s_mv[q] = mi[q];
+        if (pending) gen_plan(A, sm, L, gs, s_mv, true);  // applies the last move (Y, V)
+        if (bid == 0) {
+            if (batch) {
+                for (int w = tid; w < NWn; w += NTG) A.vouts[(size_t)rs * NWn + w] = vbs[w];
+                if (tid == 0) {
+                    int64_t *o = A.res + (size_t)rs * FS_N;
+                    o[FS_F] = f; o[FS_T] = t - 1; o[FS_BEST] = best_f; o[FS_BESTIT] = best_it;
+                    o[FS_ZERO] = zero_it; o[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
+                    o[FS_ERR] = failed ? 2 : 0;
+                }
+            } else {
+                for (int j = tid; j < m; j += NTG) A.Y[j] = Ys[j];
+                for (int w = tid; w < NWn; w += NTG) A.vb[w] = vbs[w];
+                if (tid == 0) {
+                    A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
+                    A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
+                    if (failed) A.fs[FS_ERR] = 2;
+                }
+            }
         }
-        pending = true;
-        __syncthreads();
-    }
-    if (pending) gen_plan(A, sm, L, gs, s_mv, true);  // applies the last move (Y, V)
-    if (bid == 0) {
-        for (int j = tid; j < A.I.m; j += NTG) A.Y[j] = Ys[j];
-        for (int w = tid; w < A.I.NWn; w += NTG) A.vb[w] = vbs[w];
-        if (tid == 0) {
-            A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
-            A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
-            if (failed) A.fs[FS_ERR] = 2;
-        }
+        __syncthreads();  // vbs / Ys are reused by the next restart
     }
 }
 
@@ -2807,6 +2866,7 @@ GenArgs gen_args(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L, int fl
     A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until; A.slots = c->d_slots;
     A.trace_r = c->d_tr; A.trace_f = c->d_tf; A.fit_out = nullptr;
+    A.R = 0; A.G = 1; A.nbg = 1; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
     return A;
 }
 
@@ -2852,6 +2912,83 @@ lns_status gen_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     if (iters > 0 && cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
     cudaGetLastError();
     return s;
+}
+
+// lns_tabu_run_batch for k = 4..7: R restarts on G groups of nbg CTAs (one cooperative k_gen).
+lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, int64_t tenure, uint64_t seed,
+                              const int8_t *V0, int32_t flags, int8_t *V_out, lns_result *res, void *stream)
+{
+    uint32_t M;
+    size_t smem;
+    lns_status s = gen_check(c, k, M, smem);
+    if (s != LNS_OK) return s;
+    if (!res || R < 0) return fail(LNS_EINVAL, "bad argument");
+    if (iters < 0 || iters >= (int64_t)INT32_MAX) return fail(LNS_EINVAL, "iters must be in [0, 2^31)");
+    if (flags & (LNS_FORCE_STEPPED | LNS_TABU_SOLUTIONS))
+        return fail(LNS_EINVAL, "k > 3: rank tabu list (optionally aspiration) only");
+    int64_t L;
+    if ((s = resolve_tenure(M, tenure, L)) != LNS_OK) return s;
+    if (iters + L >= (int64_t)UINT32_MAX) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    if (R == 0) return LNS_OK;
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    const int n = c->n, SMs = c->numSMs;
+    std::vector<int8_t> hv((size_t)R * n);
+    if (V0) {
+        CK(cudaMemcpy(hv.data(), V0, hv.size(), cudaMemcpyDefault));
+        for (int8_t v : hv)
+            if (v != 1 && v != -1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
+    } else {
+        for (int r = 0; r < R; r++) {
+            uint64_t sr = seed + (uint64_t)r;
+            vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
+        }
+    }
+    // groups: one round of R searches on SMs / R CTAs each when R <= SMs, else SMs single-CTA
+    // groups; an until[] of M entries per group (8 GiB at most)
+    int nbg = c->blocks_override > 0 ? std::min(c->blocks_override, SMs) : std::max(1, SMs / std::max(1, R));
+    int G = std::min(R, std::max(1, SMs / nbg));
+    G = (int)std::min<int64_t>(G, std::max<int64_t>(1, (8LL << 30) / (4LL * M)));
+    if ((s = grow(c->d_V0s, c->v0s_cap, hv.size())) != LNS_OK) return s;
+    if ((s = grow(c->d_res, c->res_cap, (size_t)R * FS_N)) != LNS_OK) return s;
+    if ((s = grow(c->d_vouts, c->vouts_cap, (size_t)R * c->NWn)) != LNS_OK) return s;
+    if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)G * 64)) != LNS_OK) return s;
+    if ((s = grow(c->d_until, c->until_cap, (size_t)G * M)) != LNS_OK) return s;
+    CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
+    CK(allow_smem((const void *)k_gen, (int)smem));
+    int occ = 0;
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
+    if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
+    k_init_slots<<<(64 * G + 255) / 256, 256, 0, st>>>(c->d_gslots, G);
+    GenArgs A = gen_args(c, k, M, iters, L, flags);
+    A.R = R; A.G = G; A.nbg = nbg; A.V0s = c->d_V0s; A.res = c->d_res; A.vouts = c->d_vouts;
+    A.until = c->d_until; A.slots = c->d_gslots; A.trace_r = nullptr; A.trace_f = nullptr;
+    void *args[] = {&A};
+    CK(cudaEventRecord(c->ev0, st));
+    CK(cudaLaunchCooperativeKernel((void *)k_gen, dim3(G * nbg), dim3(NTG), args, smem, st));
+    CK(cudaEventRecord(c->ev1, st));
+    std::vector<int64_t> hres((size_t)R * FS_N);
+    std::vector<uint32_t> hvo((size_t)R * c->NWn);
+    CK(cudaMemcpyAsync(hres.data(), c->d_res, hres.size() * 8, cudaMemcpyDeviceToHost, st));
+    CK(cudaMemcpyAsync(hvo.data(), c->d_vouts, hvo.size() * 4, cudaMemcpyDeviceToHost, st));
+    CK(cudaStreamSynchronize(st));
+    float ms = 0;
+    if (cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
+    for (int r = 0; r < R; r++) {
+        const int64_t *o = hres.data() + (size_t)r * FS_N;
+        if (o[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
+        res[r].iters_done = o[FS_T]; res[r].final_f = o[FS_F]; res[r].best_f = o[FS_BEST];
+        res[r].best_iter = o[FS_BESTIT]; res[r].first_zero_iter = o[FS_ZERO];
+        res[r].solved = o[FS_BEST] == 0; res[r].reserved = 0;
+    }
+    if (V_out) {
+        std::vector<int8_t> ho((size_t)R * n);
+        for (int r = 0; r < R; r++)
+            for (int i = 0; i < n; i++)
+                ho[(size_t)r * n + i] = ((hvo[(size_t)r * c->NWn + i / 32] >> (i % 32)) & 1) ? -1 : 1;
+        CK(cudaMemcpy(V_out, ho.data(), ho.size(), cudaMemcpyDefault));
+    }
+    return LNS_OK;
 }
 
 // lns_eval_all for k = 4..7.
@@ -3315,6 +3452,7 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
 lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, int64_t tenure, uint64_t seed,
                               const int8_t *V0, int32_t flags, int8_t *V_out, lns_result *res, void *stream)
 {
+    if (k >= 4) return gen_tabu_run_batch(c, k, R, iters, tenure, seed, V0, flags, V_out, res, stream);
     Geometry g;
     lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;

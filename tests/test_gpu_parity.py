@@ -757,7 +757,7 @@ def test_k_above_3_limits(L):
             I.tabu_run(4, 3, -1, seed=1)
         assert ei.value.status == L.LNS_ERANGE  # m > 255
     with L.Instance(small.A, small.S) as I:
-        for call in (lambda: L.lns_tabu_run_batch(I.ctx, 4, 2, 3, -1, 0, None, 0),
+        for call in (lambda: L.lns_tabu_run_batch(I.ctx, 4, 2, 3, 2, 0, None, L.LNS_TABU_SOLUTIONS),
                      lambda: I.tabu_run(8, 3, -1, seed=1),
                      lambda: I.tabu_run(4, 3, -1, seed=1, flags=L.LNS_FORCE_STEPPED),
                      lambda: I.tabu_run(4, 3, 2, seed=1, flags=L.LNS_TABU_SOLUTIONS)):
@@ -766,3 +766,22 @@ def test_k_above_3_limits(L):
             assert ei.value.status == L.LNS_EINVAL
         res = I.tabu_run(4, 5, -1, seed=1, stop_on_zero=False)[3]
         assert res["iters_done"] == 5
+
+
+@pytest.mark.parametrize("k,R,iters,blocks,aspiration", [(4, 5, 25, 0, False), (4, 9, 15, 2, True), (5, 3, 10, 0, False),
+                                                         (4, 200, 6, 0, False)])
+def test_batch_k_above_3_matches_single_runs(L, orc, k, R, iters, blocks, aspiration):
+    """lns_tabu_run_batch for k >= 4: groups of CTAs run whole restarts (in-kernel restart init,
+    per-group exchange and until[]); R > SMs takes several restarts per group."""
+    inst = pi.planted_instance(37, 26, 5100 + k)
+    rng = np.random.default_rng(R + k)
+    V0 = np.where(rng.random((R, 26)) < 0.5, -1, 1).astype(np.int8)
+    fl = L.LNS_ASPIRATION if aspiration else 0
+    with L.Instance(inst.A, inst.S) as I:
+        L.lns_config(I.ctx, blocks)
+        Vo = np.empty((R, 26), np.int8)
+        batch = L.lns_tabu_run_batch(I.ctx, k, R, iters, -1, 0, V0, fl, Vo)
+    for r in sorted(set(range(0, R, max(1, R // 8))) | {R - 1}):
+        _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0[r], iters, pi.default_tenure(26, k),
+                                       stop_on_zero=False, aspiration=aspiration)
+        assert batch[r] == ores and np.array_equal(Vo[r], oVo), r
