@@ -27,6 +27,7 @@ try:
     L.lns_tabu_run_batch(ctx, 1, 2, 8, 2, 7, None, L.LNS_TABU_SOLUTIONS)
     L.lns_tabu_run(ctx, 4, 4, -1, 1, None, 0)  # k > 3: k_gen, several CTAs
     L.lns_eval_all(ctx, 5, V)
+    L.lns_tabu_run_batch(ctx, 4, 3, 3, -1, 2, None, 0)  # k > 3 batched restarts
 finally:
     L.lns_destroy(ctx)
 big = pi.planted_instance(260, 40, 5)  # m > 255: segment-loop path, padded placement
