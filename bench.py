@@ -19,6 +19,7 @@ to rank r mod N (no per-iteration collective; the total job is fixed -> strong s
 over ranks), inputs resident in HBM. ``e2e`` = the same job through the C ABI with HOST buffers
 (instance upload, start vectors, final vectors and results back inside the timed region).
 ``single_search`` = one search at a time (latency view: all SMs on one search, 2,000 iterations).
+``c5_single_search`` = BASELINE configs[4] (1024 x 1024, 3-Hamming), one search, 5 iterations.
 ``roofline`` = the search kernel's integer throughput against the issue-rate peak.
 ``cpu_baseline`` = the CPU oracle on this host on a bounded sample. ``--impl reference`` times
 that oracle alone as the reference arm (this paper has no code).
@@ -48,6 +49,7 @@ CFG = "C4"
 RUNS = 50        # independent searches per step
 ITERS = 400      # iterations per search per step
 SINGLE_ITERS = 2000
+C5_ITERS = 5     # C5 iterations timed beside the headline (9.5 ms each)
 L2_FLUSH_BYTES = 512 << 20  # > 126 MB L2
 
 
@@ -210,6 +212,7 @@ def main():
     ap.add_argument("--runs", type=int, default=RUNS)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-single", action="store_true")
+    ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)
     args = ap.parse_args()
     rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
@@ -342,6 +345,25 @@ def main():
                   "us_per_iteration": 1e3 * best / SINGLE_ITERS, "iters": SINGLE_ITERS,
                   "note": "one search on all SMs (persistent kernel, one exchange per iteration)"}
 
+    # ---- C5 (BASELINE configs[4], 1024 x 1024, 3-Hamming, 1.78e8 neighbours per iteration): one
+    #      search on all SMs, a few iterations (N = 1 only; context beside the headline)
+    c5 = None
+    if world == 1 and not args.no_c5:
+        inst5 = pi.config_instance("C5")
+        M5 = L.lns_neighborhood_size(inst5.n, 3)
+        with L.Instance(inst5.A, inst5.S) as I5:
+            L.lns_tabu_run(I5.ctx, 3, 1, -1, pi.config_seed("C5"), None, 0)
+            ms5 = []
+            for _ in range(2):
+                flush.fill_(0)
+                torch.cuda.synchronize()
+                L.lns_tabu_run(I5.ctx, 3, C5_ITERS, -1, pi.config_seed("C5"), None, 0)
+                ms5.append(L.lns_last_kernel_ms(I5.ctx))
+        b5 = min(ms5)
+        c5 = {"neighbors_per_s": C5_ITERS * M5 / (b5 / 1e3), "tabu_iters_per_s": C5_ITERS / (b5 / 1e3),
+              "ms_per_iteration": b5 / C5_ITERS, "iters": C5_ITERS,
+              "note": "C5 single search from the config seed (packed plan for m > 255, DESIGN.md §5.11); device time of the launch"}
+
     # ---- roofline: the search kernel (one launch per step)
     pk, src = peaks()
     mhz = float(pk.get("sm_max_mhz", 1965.0))
@@ -406,6 +428,7 @@ def main():
             "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
             "single_search": single,
+            "c5_single_search": c5,
             # our kernels per timed step: k_init_slots + the persistent k_search
             "gpu_launches": args.steps * 2,
             "clocks": clocks,
