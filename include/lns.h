@@ -5,7 +5,8 @@
  *
  * The hot path: full evaluation of the k-Hamming neighbourhood (k = 1, 2, 3;
  * sizes n, C(n,2), C(n,3)) of the current +-1 solution V, selection of the
- * best non-tabu neighbour, and the move, inside a tabu search.
+ * best non-tabu neighbour, and the move, inside a tabu search. Variant
+ * k = 4..7 (the same method, generic-k kernel; see the note above lns_tabu_run).
  *
  * Conventions shared by every entry point
  *  - Problem (Definition 1): A is an m x n matrix with entries +-1, stored
