@@ -2323,6 +2323,8 @@ struct lns_ctx {
     int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
     int no_pkw = 0;  // LNS_NO_PKW=1 at create: m > 255 always takes the segment plan (A/B measurement)
     int force_pkw = 0;  // LNS_FORCE_PKW=1 at create: m > 255 tries the packed plan for any slice size
+    int no_graph = 0;   // LNS_NO_GRAPH=1 at create: the stepped loop launches directly (A/B measurement)
+    cudaStream_t cap_stream = nullptr;  // private stream for capturing the stepped loop's graph
     // device-initiated exchange (lns_attach_peers)
     unsigned long long *d_xbuf = nullptr;            // own 64-word exchange buffer (its own allocation)
     unsigned long long **d_peers = nullptr;          // device array of the partitions' buffers
@@ -3119,6 +3121,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     { const char *e = getenv("LNS_NO_PAD"); c->no_pad = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_NO_PKW"); c->no_pkw = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_FORCE_PKW"); c->force_pkw = (e && e[0] == '1') ? 1 : 0; }
+    { const char *e = getenv("LNS_NO_GRAPH"); c->no_graph = (e && e[0] == '1') ? 1 : 0; }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };
@@ -3155,6 +3158,7 @@ void lns_destroy(lns_ctx *c)
     cudaFree(c->d_xbuf); cudaFree(c->d_peers);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
+    if (c->cap_stream) cudaStreamDestroy(c->cap_stream);
     delete c;
 }
 
@@ -3425,21 +3429,60 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         if (c->nparts > 1 && !c->comm)
             return fail(LNS_EINVAL, "partitioned run needs a communicator or attached peers (or use the stepped API)");
         int64_t *kb = c->d_slots + SLOT_OUT;
-        CK(cudaEventRecord(c->ev0, st));
-        for (int64_t t = 0; t < iters; t++) {
-            if ((s = dispatch_step_eval(c, k, A, g, kb, nullptr, false, st)) != LNS_OK) return s;
+        // one iteration: partial key of this slice, NCCL u64 MIN across the communicator, move
+        auto one = [&](cudaStream_t q) -> lns_status {
+            lns_status e = dispatch_step_eval(c, k, A, g, kb, nullptr, false, q);
+            if (e != LNS_OK) return e;
             if (c->comm) {
-                const int rc = c->nccl_allreduce(kb, kb, 1, /*ncclUint64*/ 5, /*ncclMin*/ 3, c->comm, st);
+                const int rc = c->nccl_allreduce(kb, kb, 1, /*ncclUint64*/ 5, /*ncclMin*/ 3, c->comm, q);
                 if (rc != 0) return fail(LNS_ENCCL, "ncclAllReduce failed");
             }
-            if ((s = dispatch_step_apply(k, A, kb, st)) != LNS_OK) return s;
-            if ((flags & LNS_STOP_ON_ZERO) && (t % 64) == 63) {
+            return dispatch_step_apply(k, A, kb, q);
+        };
+        // The loop is launch-bound for small neighbourhoods: after one direct iteration (it sets
+        // the kernels' attributes) CH iterations are captured once into a CUDA graph on a private
+        // stream (the kernels read the iteration from device state, so the graph replays as is)
+        // and the graph is replayed on `st`; the remainder runs directly. LNS_NO_GRAPH=1 at create
+        // keeps every launch direct.
+        constexpr int64_t CH = 64;
+        cudaGraphExec_t ge = nullptr;
+        CK(cudaEventRecord(c->ev0, st));
+        int64_t t = 0;
+        if (iters > 0) {
+            if ((s = one(st)) != LNS_OK) return s;
+            t = 1;
+        }
+        if (!c->no_graph && iters - t >= CH) {
+            if (!c->cap_stream) CK(cudaStreamCreateWithFlags(&c->cap_stream, cudaStreamNonBlocking));
+            cudaGraph_t gr = nullptr;
+            CK(cudaStreamBeginCapture(c->cap_stream, cudaStreamCaptureModeThreadLocal));
+            lns_status ce = LNS_OK;
+            for (int64_t q = 0; q < CH && ce == LNS_OK; q++) ce = one(c->cap_stream);
+            const cudaError_t ee = cudaStreamEndCapture(c->cap_stream, &gr);
+            if (ce != LNS_OK) { if (gr) cudaGraphDestroy(gr); return ce; }
+            CK(ee);
+            const cudaError_t ie = cudaGraphInstantiate(&ge, gr, 0);
+            cudaGraphDestroy(gr);
+            CK(ie);
+        }
+        while (t < iters) {
+            const int64_t t_prev = t;
+            if (ge && iters - t >= CH) {
+                const cudaError_t le = cudaGraphLaunch(ge, st);
+                if (le != cudaSuccess) { cudaGraphExecDestroy(ge); return fail(LNS_ECUDA, cudaGetErrorString(le)); }
+                t += CH;
+            } else {
+                if ((s = one(st)) != LNS_OK) { if (ge) cudaGraphExecDestroy(ge); return s; }
+                t++;
+            }
+            if ((flags & LNS_STOP_ON_ZERO) && (t / 64) != (t_prev / 64)) {
                 int64_t done;
                 CK(cudaMemcpyAsync(&done, c->d_fs + FS_DONE, 8, cudaMemcpyDeviceToHost, st));
                 CK(cudaStreamSynchronize(st));
                 if (done) break;
             }
         }
+        if (ge) cudaGraphExecDestroy(ge);
         CK(cudaEventRecord(c->ev1, st));
     }
     s = search_finish(c, V_out, trace_rank, trace_fit, res, st);

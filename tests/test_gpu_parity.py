@@ -785,3 +785,54 @@ def test_batch_k_above_3_matches_single_runs(L, orc, k, R, iters, blocks, aspira
         _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, k, V0[r], iters, pi.default_tenure(26, k),
                                        stop_on_zero=False, aspiration=aspiration)
         assert batch[r] == ores and np.array_equal(Vo[r], oVo), r
+
+
+def _nccl_world1_comm():
+    """A one-rank NCCL communicator created through the libnccl torch ships (ctypes:
+    ncclGetUniqueId + ncclCommInitRank), for the production lns_attach_comm path."""
+    import ctypes
+    import glob
+    import os
+
+    import nvidia
+
+    libs = glob.glob(os.path.join(list(nvidia.__path__)[0], "nccl", "lib", "libnccl.so*"))
+    if not libs:
+        pytest.skip("libnccl not found")
+    class UniqueId(ctypes.Structure):  # ncclUniqueId: 128 bytes, passed by value
+        _fields_ = [("internal", ctypes.c_char * 128)]
+
+    nccl = ctypes.CDLL(libs[0], mode=ctypes.RTLD_GLOBAL)
+    uid = UniqueId()
+    assert nccl.ncclGetUniqueId(ctypes.byref(uid)) == 0
+    comm = ctypes.c_void_p()
+    nccl.ncclCommInitRank.argtypes = [ctypes.POINTER(ctypes.c_void_p), ctypes.c_int, UniqueId, ctypes.c_int]
+    assert nccl.ncclCommInitRank(ctypes.byref(comm), 1, uid, 0) == 0
+    return nccl, comm
+
+
+@pytest.mark.parametrize("cfg,iters", [("C2", 300), ("C3", 140)])
+def test_nccl_attached_stepped_loop_with_graphs(L, orc, cfg, iters, monkeypatch):
+    """lns_attach_comm with a real NCCL communicator (world 1): the stepped loop of lns_tabu_run
+    (eval launch, ncclAllReduce u64 MIN, apply launch per iteration) captured into CUDA graphs of
+    64 iterations and replayed, plus direct iterations; and the same with LNS_NO_GRAPH=1. Both
+    give the oracle trajectory."""
+    import torch
+
+    torch.cuda.init()
+    nccl, comm = _nccl_world1_comm()
+    c = pi.CONFIGS[cfg]
+    inst = pi.config_instance(cfg)
+    V0 = pi.start_vector(inst.n, 5)
+    otr, otf, oVo, ores = orc.tabu_run(inst.A, inst.S, c["k"], V0, iters, pi.default_tenure(inst.n, c["k"]),
+                                       stop_on_zero=False)
+    try:
+        for nog in ("0", "1"):
+            monkeypatch.setenv("LNS_NO_GRAPH", nog)
+            with L.Instance(inst.A, inst.S) as I:
+                L.lns_attach_comm(I.ctx, comm.value, 0, 1)
+                tr, tf, Vo, res = I.tabu_run(c["k"], iters, -1, V0=V0, stop_on_zero=False)
+                L.lns_attach_comm(I.ctx, None, 0, 1)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
+    finally:
+        nccl.ncclCommDestroy(comm)
