@@ -1861,6 +1861,9 @@ __global__ void k_bits_to_until(const uint32_t *bits, uint32_t *until, uint32_t 
 // ------------------------------------------------------------------------------------------
 constexpr int KG_MAX = 7;
 constexpr int NTG = 512;  // threads per CTA of the generic-k kernel (k registers of indices/masks)
+#ifndef KGEN_OCC
+#define KGEN_OCC 2  // CTAs per SM (64 registers per thread): 2 hide latency better than 1 (+20%)
+#endif
 
 struct GenArgs {
     DevInst I;
@@ -2117,7 +2120,7 @@ __device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *s
     return f;
 }
 
-__global__ void __launch_bounds__(NTG, 1) k_gen(GenArgs A)
+__global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
     __shared__ GenScalars gs;
@@ -2900,8 +2903,8 @@ lns_status gen_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         int occ = 0;
         CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
         if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
-        int nb = (int)std::min<int64_t>(std::min(c->numSMs, MAX_SLOTS), std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
-        if (c->blocks_override > 0) nb = std::min(c->blocks_override, c->numSMs);
+        int nb = (int)std::min<int64_t>(std::min(c->numSMs * occ, MAX_SLOTS), std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
+        if (c->blocks_override > 0) nb = std::min(c->blocks_override, c->numSMs * occ);
         k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
         GenArgs A = gen_args(c, k, M, iters, L, flags);
         void *args[] = {&A};
@@ -2946,10 +2949,15 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
             vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
         }
     }
-    // groups: one round of R searches on SMs / R CTAs each when R <= SMs, else SMs single-CTA
-    // groups; an until[] of M entries per group (8 GiB at most)
-    int nbg = c->blocks_override > 0 ? std::min(c->blocks_override, SMs) : std::max(1, SMs / std::max(1, R));
-    int G = std::min(R, std::max(1, SMs / nbg));
+    CK(allow_smem((const void *)k_gen, (int)smem));
+    int occ = 0;
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
+    if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
+    // groups: one round of R searches on S / R CTAs each when R <= S (S = SMs x resident CTAs),
+    // else S single-CTA groups; an until[] of M entries per group (8 GiB at most)
+    const int S = SMs * occ;
+    int nbg = c->blocks_override > 0 ? std::min(c->blocks_override, S) : std::max(1, S / std::max(1, R));
+    int G = std::min(R, std::max(1, S / nbg));
     G = (int)std::min<int64_t>(G, std::max<int64_t>(1, (8LL << 30) / (4LL * M)));
     if ((s = grow(c->d_V0s, c->v0s_cap, hv.size())) != LNS_OK) return s;
     if ((s = grow(c->d_res, c->res_cap, (size_t)R * FS_N)) != LNS_OK) return s;
@@ -2957,10 +2965,6 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)G * 64)) != LNS_OK) return s;
     if ((s = grow(c->d_until, c->until_cap, (size_t)G * M)) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
-    CK(allow_smem((const void *)k_gen, (int)smem));
-    int occ = 0;
-    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
-    if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
     k_init_slots<<<(64 * G + 255) / 256, 256, 0, st>>>(c->d_gslots, G);
     GenArgs A = gen_args(c, k, M, iters, L, flags);
     A.R = R; A.G = G; A.nbg = nbg; A.V0s = c->d_V0s; A.res = c->d_res; A.vouts = c->d_vouts;
