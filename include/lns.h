@@ -127,7 +127,8 @@ lns_status lns_eval_all(lns_ctx *ctx, int32_t k, const int8_t *V, int32_t *fitne
  *   Errors: EINVAL, ERANGE (limits, tenure >= C(n,k)), ENOMEM, ECUDA, ENCCL. */
 /* k > 3 (PAPER.md:105-125 generalised; 4 <= k <= 7): lns_tabu_run (one
  *   device, persistent kernel, rank tabu list with or without LNS_ASPIRATION),
- *   lns_tabu_run_batch (the same per restart), lns_eval_all and lns_unrank only; m <= 255 (the byte window) else ERANGE; other calls and
+ *   lns_tabu_run_batch (the same per restart), lns_eval_neighborhood (no partition),
+ *   lns_eval_all and lns_unrank only; m <= 255 (the byte window) else ERANGE; other calls and
  *   flags with k > 3 return EINVAL. */
 lns_status lns_tabu_run(lns_ctx *ctx, int32_t k, int64_t iters, int64_t tenure, uint64_t seed,
                         const int8_t *V0, int32_t flags, int8_t *V_out, int64_t *trace_rank,

@@ -1878,6 +1878,7 @@ struct GenArgs {
     int64_t *slots;
     int64_t *trace_r, *trace_f;
     int32_t *fit_out;  // non-null: write every rank's fitness (lns_eval_all), no search
+    unsigned long long *best_out;  // non-null: MIN of the admissible keys (until[r] = 0) into it (eval_neighborhood)
     // batched restarts (R > 0): G groups of nbg CTAs; until[] of M entries and 64 exchange slots
     // per group; restart r from V0s + r n, results into res + r FS_N and vouts + r NWn
     int32_t R, G, nbg;
@@ -2151,13 +2152,22 @@ __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
     // this thread's contiguous run of ranks (within its group)
     const uint64_t span = A.M, gt = (uint64_t)bid * NTG + tid, Gt = (uint64_t)nbg * NTG;
     const uint32_t lo = (uint32_t)(span * gt / Gt), hi = (uint32_t)(span * (gt + 1) / Gt);
-    if (A.fit_out) {
+    if (A.fit_out || A.best_out) {
         gen_plan(A, sm, L, gs, s_mv, false);
         int idx[KG_MAX];
+        unsigned long long best = (unsigned long long)KEY_NONE;
         if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
         for (uint32_t r = lo; r < hi; r++) {
-            A.fit_out[r] = gen_eval(A, sm, L, gs, idx);
+            if (A.fit_out) A.fit_out[r] = gen_eval(A, sm, L, gs, idx);
+            else if (A.until[r] == 0u) {
+                const unsigned long long key = ((unsigned long long)(uint32_t)gen_eval(A, sm, L, gs, idx) << 32) | r;
+                if (key < best) best = key;
+            }
             if (r + 1 < hi) gen_succ(n, K, idx);
+        }
+        if (A.best_out) {
+            best = warp_min_k(best);
+            if (lane == 0 && best != (unsigned long long)KEY_NONE) atomicMin(A.best_out, best);
         }
         return;
     }
@@ -2870,7 +2880,7 @@ GenArgs gen_args(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L, int fl
     A.stop_on_zero = (flags & LNS_STOP_ON_ZERO) ? 1 : 0;
     A.aspiration = (flags & LNS_ASPIRATION) ? 1 : 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until; A.slots = c->d_slots;
-    A.trace_r = c->d_tr; A.trace_f = c->d_tf; A.fit_out = nullptr;
+    A.trace_r = c->d_tr; A.trace_f = c->d_tf; A.fit_out = nullptr; A.best_out = nullptr;
     A.R = 0; A.G = 1; A.nbg = 1; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
     return A;
 }
@@ -2994,6 +3004,51 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
                 ho[(size_t)r * n + i] = ((hvo[(size_t)r * c->NWn + i / 32] >> (i % 32)) & 1) ? -1 : 1;
         CK(cudaMemcpy(V_out, ho.data(), ho.size(), cudaMemcpyDefault));
     }
+    return LNS_OK;
+}
+
+// lns_eval_neighborhood for k = 4..7: k_gen over every rank, admissible keys MIN-reduced.
+lns_status gen_eval_best(lns_ctx *c, int32_t k, const int8_t *V, const int32_t *Y, const uint32_t *tabu_bits,
+                         int64_t *best_fitness, int64_t *best_rank, void *stream)
+{
+    uint32_t M;
+    size_t smem;
+    lns_status s = gen_check(c, k, M, smem);
+    if (s != LNS_OK) return s;
+    if (!V || !Y || !best_fitness || !best_rank) return fail(LNS_EINVAL, "null argument");
+    if (c->nparts > 1 || c->comm || c->npeers > 0) return fail(LNS_EINVAL, "k > 3: no partitions");
+    DeviceGuard dg(c->device);
+    cudaStream_t st = (cudaStream_t)stream;
+    const size_t tw = (M + 31) / 32;
+    if ((s = grow(c->d_until, c->until_cap, M)) != LNS_OK) return s;
+    if (tabu_bits) {
+        if ((s = grow(c->d_bits, c->bits_cap, tw)) != LNS_OK) return s;
+        CK(cudaMemcpyAsync(c->d_bits, tabu_bits, tw * 4, cudaMemcpyDefault, st));
+    }
+    k_bits_to_until<<<std::min<uint32_t>(4096, (M + 255) / 256), 256, 0, st>>>(tabu_bits ? c->d_bits : nullptr,
+                                                                              c->d_until, M);
+    CK(cudaMemcpyAsync(c->d_V, V, c->n, cudaMemcpyDefault, st));
+    CK(cudaMemcpyAsync(c->d_Yin, Y, 4 * (size_t)c->m, cudaMemcpyDefault, st));
+    k_fill_i64<<<1, 32, 0, st>>>(c->d_slots + SLOT_OUT, KEY_NONE, 1);
+    k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, c->d_Yin, c->d_fs);
+    CK(allow_smem((const void *)k_gen, (int)smem));
+    GenArgs A = gen_args(c, k, M, 0, 0, 0);
+    A.best_out = (unsigned long long *)(c->d_slots + SLOT_OUT);
+    int nb = (int)std::min<int64_t>(4LL * c->numSMs, std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
+    if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs);
+    CK(cudaEventRecord(c->ev0, st));
+    k_gen<<<nb, NTG, smem, st>>>(A);
+    CK(cudaGetLastError());
+    CK(cudaEventRecord(c->ev1, st));
+    int64_t key, fs[FS_N];
+    CK(cudaMemcpyAsync(&key, c->d_slots + SLOT_OUT, 8, cudaMemcpyDeviceToHost, st));
+    CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
+    CK(cudaStreamSynchronize(st));
+    float ms = 0; cudaEventElapsedTime(&ms, c->ev0, c->ev1); c->last_ms = ms;
+    if (fs[FS_ERR]) return fail(LNS_EINVAL, "V must be +-1 and Y must equal A V");
+    if (key == KEY_NONE) { *best_fitness = -1; *best_rank = -1; return fail(LNS_ENOADMISSIBLE, "all ranks tabu"); }
+    *best_fitness = key >> 32;
+    *best_rank = key & 0xffffffffLL;
     return LNS_OK;
 }
 
@@ -3286,6 +3341,7 @@ lns_status lns_attach_peers_ipc(lns_ctx *c, int32_t part, int32_t nparts, const 
 lns_status lns_eval_neighborhood(lns_ctx *c, int32_t k, const int8_t *V, const int32_t *Y, const uint32_t *tabu_bits,
                                  int64_t *best_fitness, int64_t *best_rank, void *stream)
 {
+    if (k >= 4) return gen_eval_best(c, k, V, Y, tabu_bits, best_fitness, best_rank, stream);
     Geometry g;
     lns_status s = check_k(c, k, g);
     if (s != LNS_OK) return s;

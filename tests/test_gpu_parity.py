@@ -137,7 +137,10 @@ def test_eval_neighborhood_errors(L):
             L.lns_eval_neighborhood(ctx, 1, V, Y + 2)
         assert e.value.status == L.LNS_EINVAL
         with pytest.raises(L.LnsError) as e:
-            L.lns_eval_neighborhood(ctx, 4, V, Y)
+            L.lns_eval_neighborhood(ctx, 8, V, Y)  # k in 1..7
+        assert e.value.status == L.LNS_EINVAL
+        with pytest.raises(L.LnsError) as e:
+            L.lns_eval_neighborhood(ctx, 4, V, Y + 2)  # the k > 3 path checks Y = A V too
         assert e.value.status == L.LNS_EINVAL
         allbits = np.full(1, 0xFFFFFFFF, np.uint32)
         with pytest.raises(L.LnsError) as e:
@@ -836,3 +839,26 @@ def test_nccl_attached_stepped_loop_with_graphs(L, orc, cfg, iters, monkeypatch)
             assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(Vo, oVo)
     finally:
         nccl.ncclCommDestroy(comm)
+
+
+@pytest.mark.parametrize("m,n,k", [(41, 30, 4), (60, 22, 5)])
+def test_eval_neighborhood_k_above_3_best_with_tabu(L, orc, m, n, k):
+    """lns_eval_neighborhood for k >= 4: best admissible (f, rank) with 0 / 50 % / all-but-one tabu,
+    and ENOADMISSIBLE when every rank is tabu."""
+    inst = pi.planted_instance(m, n, 5300 + n + k)
+    rng = np.random.default_rng(n + k)
+    M = comb(n, k)
+    with L.Instance(inst.A, inst.S) as I:
+        for V in _states(inst, rng, count=1):
+            Y = (inst.A.astype(np.int32) @ V.astype(np.int32)).astype(np.int32)
+            for frac in (0.0, 0.5, 1.0):
+                tabu = rng.random(M) < frac
+                if frac == 1.0:
+                    tabu[rng.integers(M)] = False
+                bits = np.packbits(tabu, bitorder="little")
+                bits = np.concatenate([bits, np.zeros((-len(bits)) % 4, np.uint8)]).view(np.uint32)
+                assert L.lns_eval_neighborhood(I.ctx, k, V, Y, bits) == orc.eval_best(inst.A, inst.S, V, k, tabu)
+        allbits = np.full((M + 31) // 32, 0xFFFFFFFF, np.uint32)
+        with pytest.raises(L.LnsError) as ei:
+            L.lns_eval_neighborhood(I.ctx, k, V, Y, allbits)
+        assert ei.value.status == L.LNS_ENOADMISSIBLE
