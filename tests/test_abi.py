@@ -71,3 +71,38 @@ def test_no_cpu_fallback_without_gpu():
 
     with pytest.raises(L.LnsError):
         L.lns_create(np.ones((2, 3), np.int8), np.array([3, 3], np.int32))
+
+
+def _build_c_example(tmp_path):
+    import os
+    import shutil
+    import subprocess
+
+    import paper_conf_ipps_luongmt10_b200 as L
+
+    cc = shutil.which("cc") or shutil.which("gcc")
+    if not cc:
+        pytest.skip("no C compiler")
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    libdir = os.path.dirname(L._build.LIB)
+    L.load()  # builds liblns.so if missing
+    exe = str(tmp_path / "tabu_c")
+    subprocess.check_call([cc, "-O2", "-Wall", "-Werror", "-I", os.path.join(root, "include"),
+                           os.path.join(root, "examples", "tabu_c.c"), "-L", libdir, "-llns",
+                           f"-Wl,-rpath,{libdir}", "-o", exe])
+    return exe
+
+
+def test_c_example_builds_against_the_header_and_fails_loudly_without_gpu(tmp_path):
+    """The boundary is a plain C ABI: examples/tabu_c.c (no Python, no torch) compiles against
+    include/lns.h and links liblns.so; without a usable GPU its first call fails with a CUDA error
+    (no CPU fallback)."""
+    import subprocess
+
+    import torch
+
+    exe = _build_c_example(tmp_path)
+    if torch.cuda.is_available():
+        return
+    out = subprocess.run([exe, "21", "21", "1", "10"], capture_output=True, text=True, timeout=120)
+    assert out.returncode == 1 and "CUDA error" in out.stderr, out.stderr

@@ -862,3 +862,15 @@ def test_eval_neighborhood_k_above_3_best_with_tabu(L, orc, m, n, k):
         with pytest.raises(L.LnsError) as ei:
             L.lns_eval_neighborhood(I.ctx, k, V, Y, allbits)
         assert ei.value.status == L.LNS_ENOADMISSIBLE
+
+
+def test_c_example_runs_on_the_gpu(L, tmp_path):
+    """examples/tabu_c.c -- the C ABI from plain C, host buffers only: eval, tabu run, batch."""
+    import subprocess
+
+    from test_abi import _build_c_example
+
+    exe = _build_c_example(tmp_path)
+    for args in (["101", "117", "3", "200"], ["73", "73", "2", "300"], ["41", "30", "4", "20"]):
+        out = subprocess.run([exe, *args], capture_output=True, text=True, timeout=300)
+        assert out.returncode == 0 and out.stdout.strip().endswith("ok"), out.stdout + out.stderr
