@@ -568,7 +568,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     PH(1);
     // C. place rows; emit the records (one thread per walked point); bin constants; deep constant.
     //    pstart[w] = shared address of the first record in row word w
-    const int vmin = ps.vmin, U = ps.U, NB = ps.NB, uf = ps.ufirst, uneg = ps.uneg, utop = ps.utop;
+    const int vmin = ps.vmin, NB = ps.NB, uf = ps.ufirst, uneg = ps.uneg, utop = ps.utop;
     const uint32_t pk0 = (uint32_t)__cvta_generic_to_shared(pk);
     for (int j = tid; j < m; j += NT) {
         const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
@@ -1468,7 +1468,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
     const bool batch = A.R > 0;
-    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int lane = threadIdx.x & 31;
     const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
     __shared__ unsigned long long *s_peers[MAX_PEERS];
     __shared__ int s_xto;
