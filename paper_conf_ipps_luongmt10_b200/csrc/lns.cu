@@ -337,17 +337,16 @@ __device__ __forceinline__ void range_publish(int mn, int mx, PlanScalars &ps)
 // Plan step D: X[w][c], per (row word, column word) pair, lane l loads sorted row 32w+l's sign
 // bits of columns 32cw..32cw+31 (rowAt[p] = -1 marks a hole) and a 5-round shuffle transpose turns
 // rows into columns; zero cnt[] for the next plan.
-__device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L,
-                                               const PlanScalars &ps, uint32_t *X, int Uc)
+// The transpose of warps w0, w0 + 1, .., w0 + nw - 1 (no barrier).
+__device__ __forceinline__ void plan_transpose_warps(const DevInst &I, const uint32_t *Ar, unsigned char *sm,
+                                                     const Smem &L, const PlanScalars &ps, uint32_t *X, int w0, int nw)
 {
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const int m = I.m, n = I.n, NWn = I.NWn;
     const uint32_t *vbs = (const uint32_t *)(sm + L.vb);
     const int *rowAt = (const int *)(sm + L.rowAt);
-    int *cnt = (int *)(sm + L.cnt);
-    for (int u = tid; u < Uc; u += NT) cnt[u] = 0;
     const int Wp = ps.Wp;
-    for (int pr = warp; pr < Wp * NWn; pr += NWARP) {
+    for (int pr = warp - w0; pr < Wp * NWn; pr += nw) {
         const int w = pr / NWn, cw = pr - w * NWn;
         const int p = 32 * w + lane;
         const int j = I.pad ? rowAt[p] : (p < m ? rowAt[p] : -1);
@@ -362,6 +361,14 @@ __device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t 
         const int c = 32 * cw + lane;
         if (c < n) X[w * n + c] = x;
     }
+}
+
+__device__ __forceinline__ void plan_transpose(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L,
+                                               const PlanScalars &ps, uint32_t *X, int Uc)
+{
+    int *cnt = (int *)(sm + L.cnt);
+    for (int u = threadIdx.x; u < Uc; u += NT) cnt[u] = 0;
+    plan_transpose_warps(I, Ar, sm, L, ps, X, 0, NWARP);
     __syncthreads();
     PH(3);
 }
@@ -574,63 +581,69 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
         rowAt[p] = j;
     }
-    for (int v = uneg + tid; v < utop; v += NT) {
-        const int st = seg[v], Lv = cnt[uf + v], en = st + Lv;
-        int p = pofs[v];
-        if (p < 0) continue;  // absorbed by its predecessor
-        const int b = vmin + 2 * (v - K);
-        uint32_t Hfin = ((b >= 0 && b <= n) ? (uint32_t)Hs[b] << 8 : 0u) | 8u;
-        uint32_t wfin = 0x4404u | ((b < 0 ? (uint32_t)(60 * (-b) - 1) : 0u) << 16);
-        uint32_t src = v + 8 < utop ? (uint32_t)cnt[uf + v + 8] : 0u;
-        if (v + 2 < utop && pofs[v + 2] < 0) {
-            // two bins: v and the absorbed v + 2 (both weights 0): h_v -> byte 1, h_v+2 -> byte 2 of
-            // hb, H in bytes 1, 2 of z, shift 16 (the SAD adds 16 = 8 per bin), and the rows of the
-            // points v + 8, v + 10 enter as the new bytes 2, 3
-            const int b2 = b + 4;
-            Hfin = (b2 <= n ? (uint32_t)Hs[b2] << 16 : 0u) | (b <= n ? (uint32_t)Hs[b] << 8 : 0u) | 16u;
-            wfin = 0x4104u;
-            src |= (v + 10 < utop ? (uint32_t)cnt[uf + v + 10] : 0u) << 8;
-        }
-        if (Lv == 0) {  // empty point: one zero record (in the previous row word) that completes its bin
-            const int w = max(0, (st - 1) >> 5);
-            pk[p] = make_uint4(0u, src, Hfin, wfin);
-            atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
-            if (v - uneg < 2) ps.pkw0[v - uneg] = w;
-            continue;
-        }
-        const int w0 = st >> 5, w1 = (en - 1) >> 5;
-        if (v - uneg < 2) ps.pkw0[v - uneg] = w0;
-        for (int w = w0; w <= w1; w++, p++) {
-            const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
-            const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
-            pk[p] = w == w1 ? make_uint4(mask, src, Hfin, wfin) : make_uint4(mask, 0u, 0u, 0x4444u);
-            atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
-        }
-    }
-    for (int v = tid; v < uneg; v += NT)  // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form)
-        if (cnt[uf + v] > 0)
-            atomicAdd((unsigned *)&ps.cneg, (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v))));
-    const int z0 = ps.pkz[0], z1 = ps.pkz[1];
-    for (int beta = tid; beta < NB; beta += NT) {
-        const int b = vmin + 2 * (beta - K);
-        const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
-        bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
-        // walked bins: [first point, last point + 2K] of the walk of beta's parity
-        const int zp = ((beta - uneg) & 1) ? z1 : z0;
-        if (Hb && beta >= uneg && zp >= 0 && beta <= zp + 2 * K) atomicAdd(&ps.hwalk, Hb);
-    }
-    __syncthreads();
+    __syncthreads();  // rows placed: step D (X, warps 1..) overlaps the rest of C (warp 0)
     PH(2);
-    if (tid < 2) {  // the walks' ready-to-use addresses and constants (read by pk_walk)
-        const int q = tid, wd = ps.pkw0[q];
-        const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
-        const uint32_t xb = XG ? (uint32_t)(wd * n) : (uint32_t)__cvta_generic_to_shared(X + wd * n);
-        ps.pkwk[q] = make_uint4(xb, pk0 + 16u * pb, pk0 + 16u * pe,
-                                (uint32_t)__cvta_generic_to_shared(pstart + wd + 1));
-        ps.pkwt[q] = make_uint4(ps.pkwin[q], ps.pkhtr[q], (uint32_t)ps.pktrl[q], (uint32_t)ps.pkz[q]);
+    if (warp != 0) {
+        plan_transpose_warps(I, Ar, sm, L, ps, X, 1, NWARP - 1);
+    } else {
+        for (int v = uneg + lane; v < utop; v += 32) {
+            const int st = seg[v], Lv = cnt[uf + v], en = st + Lv;
+            int p = pofs[v];
+            if (p < 0) continue;  // absorbed by its predecessor
+            const int b = vmin + 2 * (v - K);
+            uint32_t Hfin = ((b >= 0 && b <= n) ? (uint32_t)Hs[b] << 8 : 0u) | 8u;
+            uint32_t wfin = 0x4404u | ((b < 0 ? (uint32_t)(60 * (-b) - 1) : 0u) << 16);
+            uint32_t src = v + 8 < utop ? (uint32_t)cnt[uf + v + 8] : 0u;
+            if (v + 2 < utop && pofs[v + 2] < 0) {
+                // two bins: v and the absorbed v + 2 (both weights 0): h_v -> byte 1, h_v+2 -> byte 2 of
+                // hb, H in bytes 1, 2 of z, shift 16 (the SAD adds 16 = 8 per bin), and the rows of the
+                // points v + 8, v + 10 enter as the new bytes 2, 3
+                const int b2 = b + 4;
+                Hfin = (b2 <= n ? (uint32_t)Hs[b2] << 16 : 0u) | (b <= n ? (uint32_t)Hs[b] << 8 : 0u) | 16u;
+                wfin = 0x4104u;
+                src |= (v + 10 < utop ? (uint32_t)cnt[uf + v + 10] : 0u) << 8;
+            }
+            if (Lv == 0) {  // empty point: one zero record (in the previous row word) that completes its bin
+                const int w = max(0, (st - 1) >> 5);
+                pk[p] = make_uint4(0u, src, Hfin, wfin);
+                atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
+                if (v - uneg < 2) ps.pkw0[v - uneg] = w;
+                continue;
+            }
+            const int w0 = st >> 5, w1 = (en - 1) >> 5;
+            if (v - uneg < 2) ps.pkw0[v - uneg] = w0;
+            for (int w = w0; w <= w1; w++, p++) {
+                const int lo = max(st, 32 * w) - 32 * w, hi = min(en, 32 * w + 32) - 32 * w;
+                const uint32_t mask = (hi == 32 ? FULL : ((1u << hi) - 1u)) & (FULL << lo);
+                pk[p] = w == w1 ? make_uint4(mask, src, Hfin, wfin) : make_uint4(mask, 0u, 0u, 0x4444u);
+                atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
+            }
+        }
+        for (int v = lane; v < uneg; v += 32)  // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form)
+            if (cnt[uf + v] > 0)
+                atomicAdd((unsigned *)&ps.cneg, (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v))));
+        const int z0 = ps.pkz[0], z1 = ps.pkz[1];
+        for (int beta = lane; beta < NB; beta += 32) {
+            const int b = vmin + 2 * (beta - K);
+            const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
+            bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
+            // walked bins: [first point, last point + 2K] of the walk of beta's parity
+            const int zp = ((beta - uneg) & 1) ? z1 : z0;
+            if (Hb && beta >= uneg && zp >= 0 && beta <= zp + 2 * K) atomicAdd(&ps.hwalk, Hb);
+        }
+        __syncwarp();  // the last readers of cnt[] and the writers of pkw0 are in this warp
+        for (int u = lane; u < Uc; u += 32) cnt[u] = 0;  // zero for the next plan
+        if (lane < 2) {  // the walks' ready-to-use addresses and constants (read by pk_walk)
+            const int q = tid, wd = ps.pkw0[q];
+            const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
+            const uint32_t xb = XG ? (uint32_t)(wd * n) : (uint32_t)__cvta_generic_to_shared(X + wd * n);
+            ps.pkwk[q] = make_uint4(xb, pk0 + 16u * pb, pk0 + 16u * pe,
+                                    (uint32_t)__cvta_generic_to_shared(pstart + wd + 1));
+            ps.pkwt[q] = make_uint4(ps.pkwin[q], ps.pkhtr[q], (uint32_t)ps.pktrl[q], (uint32_t)ps.pkz[q]);
+        }
     }
-    // D. X (its closing barrier also publishes pkwk / pkwt)
-    plan_transpose(I, Ar, sm, L, ps, X, Uc);
+    __syncthreads();  // X (warps 1..), records, bins, pkwk / pkwt are published
+    PH(3);
 }
 
 // ------------------------------------------------------------------------------------------
