@@ -2086,10 +2086,12 @@ __device__ __forceinline__ void gen_planes(const uint32_t *__restrict__ xw, cons
 // one row word, mask m) the walk window gains sum_rows 256^t = popc(m) + sum (256^t - 1), and with
 // t = b0 + 2 b1 + 4 b2: 256^t - 1 = (1 + 255 b0)(1 + 65535 b1)(1 + (2^32 - 1) b2) - 1, i.e. seven
 // masked plane products (those K cannot reach vanish: K = 4 needs 4 POPCs, 5: 5, 6: 6, 7: 7).
+template <int KT>
 __device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *sm, const GenSmem &L,
                                         const GenScalars &gs, const int *idx)
 {
-    const int K = A.K, n = A.I.n;
+    constexpr int K = KT;
+    const int n = A.I.n;
     const uint32_t *X = (const uint32_t *)(sm + L.X);
     const uint2 *pc = (const uint2 *)(sm + L.pc);
     const int2 *bins = (const int2 *)(sm + L.bins);
@@ -2134,6 +2136,8 @@ __device__ __forceinline__ int gen_eval(const GenArgs &A, const unsigned char *s
     return f;
 }
 
+// One instantiation per k (4..7): the plane loops and the product terms fold at compile time.
+template <int KT>
 __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
@@ -2141,7 +2145,8 @@ __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
     __shared__ int s_mv[KG_MAX];
     __shared__ int s_pen, s_hd;
     const GenSmem L = gen_layout(A.I.m, A.I.n, A.I.NWn, A.K);
-    const int tid = threadIdx.x, lane = tid & 31, K = A.K, n = A.I.n, m = A.I.m, NWn = A.I.NWn;
+    constexpr int K = KT;
+    const int tid = threadIdx.x, lane = tid & 31, n = A.I.n, m = A.I.m, NWn = A.I.NWn;
     // batched restarts (A.R > 0): group g = CTAs [g nbg, (g+1) nbg) runs restarts g, g + G, ...
     const bool batch = A.R > 0;
     const int nbg = batch ? A.nbg : (int)gridDim.x;
@@ -2171,9 +2176,9 @@ __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
         unsigned long long best = (unsigned long long)KEY_NONE;
         if (lo < hi) gen_unrank(lo, n, K, A.M, C, idx);
         for (uint32_t r = lo; r < hi; r++) {
-            if (A.fit_out) A.fit_out[r] = gen_eval(A, sm, L, gs, idx);
+            if (A.fit_out) A.fit_out[r] = gen_eval<KT>(A, sm, L, gs, idx);
             else if (A.until[r] == 0u) {
-                const unsigned long long key = ((unsigned long long)(uint32_t)gen_eval(A, sm, L, gs, idx) << 32) | r;
+                const unsigned long long key = ((unsigned long long)(uint32_t)gen_eval<KT>(A, sm, L, gs, idx) << 32) | r;
                 if (key < best) best = key;
             }
             if (r + 1 < hi) gen_succ(n, K, idx);
@@ -2233,7 +2238,7 @@ __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
             for (uint32_t r = lo; r < hi; r++) {
                 const bool tabu = until[r] >= (uint32_t)t;
                 if (!tabu || A.aspiration) {
-                    const int fr = gen_eval(A, sm, L, gs, idx);
+                    const int fr = gen_eval<KT>(A, sm, L, gs, idx);
                     const unsigned long long key = ((unsigned long long)(uint32_t)fr << 32) | r;
                     if ((!tabu || fr < best_f) && key < best) best = key;
                 }
@@ -2870,7 +2875,29 @@ lns_status dispatch_step_apply(int k, const SearchArgs &A, const int64_t *key, c
     }
 }
 
-// k = 4..7 (the generic-k kernel k_gen): limits and shared memory.
+// k = 4..7 (the generic-k kernel k_gen): the instantiation, limits and shared memory.
+const void *kgen_fn(int k)
+{
+    switch (k) {
+    case 4: return (const void *)k_gen<4>;
+    case 5: return (const void *)k_gen<5>;
+    case 6: return (const void *)k_gen<6>;
+    default: return (const void *)k_gen<7>;
+    }
+}
+
+cudaError_t kgen_launch(int k, int nb, size_t smem, cudaStream_t st, const GenArgs &A)
+{
+    switch (k) {
+    case 4: k_gen<4><<<nb, NTG, smem, st>>>(A); break;
+    case 5: k_gen<5><<<nb, NTG, smem, st>>>(A); break;
+    case 6: k_gen<6><<<nb, NTG, smem, st>>>(A); break;
+    default: k_gen<7><<<nb, NTG, smem, st>>>(A); break;
+    }
+    return cudaGetLastError();
+}
+
+// k = 4..7: limits and shared memory.
 lns_status gen_check(lns_ctx *c, int k, uint32_t &M, size_t &smem)
 {
     if (!c) return fail(LNS_EINVAL, "null context");
@@ -2922,9 +2949,9 @@ lns_status gen_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     g.M = M;
     if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
     if (iters > 0) {
-        CK(allow_smem((const void *)k_gen, (int)smem));
+        CK(allow_smem(kgen_fn(k), (int)smem));
         int occ = 0;
-        CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
+        CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kgen_fn(k), NTG, smem));
         if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
         int nb = (int)std::min<int64_t>(std::min(c->numSMs * occ, MAX_SLOTS), std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
         if (c->blocks_override > 0) nb = std::min(c->blocks_override, c->numSMs * occ);
@@ -2932,7 +2959,7 @@ lns_status gen_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         GenArgs A = gen_args(c, k, M, iters, L, flags);
         void *args[] = {&A};
         CK(cudaEventRecord(c->ev0, st));
-        CK(cudaLaunchCooperativeKernel((void *)k_gen, dim3(nb), dim3(NTG), args, smem, st));
+        CK(cudaLaunchCooperativeKernel((void *)kgen_fn(k), dim3(nb), dim3(NTG), args, smem, st));
         CK(cudaEventRecord(c->ev1, st));
     }
     s = search_finish(c, V_out, trace_rank, trace_fit, res, st);
@@ -2972,9 +2999,9 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
             vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
         }
     }
-    CK(allow_smem((const void *)k_gen, (int)smem));
+    CK(allow_smem(kgen_fn(k), (int)smem));
     int occ = 0;
-    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_gen, NTG, smem));
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kgen_fn(k), NTG, smem));
     if (occ < 1) return fail(LNS_ERANGE, "k > 3 kernel does not fit on an SM");
     // groups: one round of R searches on S / R CTAs each when R <= S (S = SMs x resident CTAs),
     // else S single-CTA groups; an until[] of M entries per group (8 GiB at most)
@@ -2994,7 +3021,7 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     A.until = c->d_until; A.slots = c->d_gslots; A.trace_r = nullptr; A.trace_f = nullptr;
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
-    CK(cudaLaunchCooperativeKernel((void *)k_gen, dim3(G * nbg), dim3(NTG), args, smem, st));
+    CK(cudaLaunchCooperativeKernel((void *)kgen_fn(k), dim3(G * nbg), dim3(NTG), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     std::vector<int64_t> hres((size_t)R * FS_N);
     std::vector<uint32_t> hvo((size_t)R * c->NWn);
@@ -3044,14 +3071,13 @@ lns_status gen_eval_best(lns_ctx *c, int32_t k, const int8_t *V, const int32_t *
     CK(cudaMemcpyAsync(c->d_Yin, Y, 4 * (size_t)c->m, cudaMemcpyDefault, st));
     k_fill_i64<<<1, 32, 0, st>>>(c->d_slots + SLOT_OUT, KEY_NONE, 1);
     k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, c->d_Yin, c->d_fs);
-    CK(allow_smem((const void *)k_gen, (int)smem));
+    CK(allow_smem(kgen_fn(k), (int)smem));
     GenArgs A = gen_args(c, k, M, 0, 0, 0);
     A.best_out = (unsigned long long *)(c->d_slots + SLOT_OUT);
     int nb = (int)std::min<int64_t>(4LL * c->numSMs, std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
     if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs);
     CK(cudaEventRecord(c->ev0, st));
-    k_gen<<<nb, NTG, smem, st>>>(A);
-    CK(cudaGetLastError());
+    CK(kgen_launch(k, nb, smem, st, A));
     CK(cudaEventRecord(c->ev1, st));
     int64_t key, fs[FS_N];
     CK(cudaMemcpyAsync(&key, c->d_slots + SLOT_OUT, 8, cudaMemcpyDeviceToHost, st));
@@ -3078,14 +3104,13 @@ lns_status gen_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness
     if ((s = grow(c->d_fit, c->fit_cap, M)) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V, V, c->n, cudaMemcpyDefault, st));
     k_init<<<1, NT, 0, st>>>(dev_inst(c), c->d_V, c->d_vb, c->d_Y, nullptr, c->d_fs);
-    CK(allow_smem((const void *)k_gen, (int)smem));
+    CK(allow_smem(kgen_fn(k), (int)smem));
     GenArgs A = gen_args(c, k, M, 0, 0, 0);
     A.fit_out = c->d_fit;
     int nb = (int)std::min<int64_t>(4LL * c->numSMs, std::max<int64_t>(1, (int64_t)M / (4 * NTG)));
     if (c->blocks_override > 0) nb = std::min(c->blocks_override, 4 * c->numSMs);
     CK(cudaEventRecord(c->ev0, st));
-    k_gen<<<nb, NTG, smem, st>>>(A);
-    CK(cudaGetLastError());
+    CK(kgen_launch(k, nb, smem, st, A));
     CK(cudaEventRecord(c->ev1, st));
     int64_t fs[FS_N];
     CK(cudaMemcpyAsync(fs, c->d_fs, sizeof(fs), cudaMemcpyDeviceToHost, st));
