@@ -236,6 +236,46 @@ int32_t lns_version(void); /* major*10000 + minor*100 + patch */
 void lns_pool_trim(void);
 void lns_pool_stats(int64_t *cached_bytes, int64_t *live_bytes);
 
+/* ---------------------------------------------------------------------------------------------
+ * Second binary fitness: UBQP (SURVEY.md §8(f) f4 "a pluggable binary fitness").
+ * The paper states its neighbourhood mappings "for binary problems" and
+ * validates them on the PPP only. Here the same k-Hamming tabu search (neighbourhood
+ * PAPER.md:105-125, lexicographic ranks R6, until[] tabu list R3 with default tenure
+ * floor(C(n,k)/6), least fitness / lowest rank R5, no aspiration R4) minimises
+ *     f(x) = x^T Q x = sum_i sum_j Q_ij x_i x_j,   x in {0,1}^n,  Q symmetric int32.
+ * k in {1, 2, 3}. Vectors are uint8 0/1 (NOT the +-1 int8 of the PPP calls).
+ * ------------------------------------------------------------------------------------------- */
+typedef struct lns_bqp lns_bqp;
+
+/* lns_bqp_create -- upload Q ((host|device) n x n int32 row-major, symmetric) to `device`; the
+ *   caller keeps Q. *out receives a context owned by the library until lns_bqp_destroy.
+ *   Errors: EINVAL (n < 1, Q not symmetric, bad device), ERANGE (n > 4096, or sum |Q_ij| >= 2^29:
+ *   the kernels compute fitnesses exactly in int32), ENOMEM, ECUDA. */
+lns_status lns_bqp_create(const int32_t *Q, int32_t n, int32_t device, lns_bqp **out);
+
+/* lns_bqp_destroy -- free everything the context owns (NULL is a no-op). */
+void lns_bqp_destroy(lns_bqp *ctx);
+
+/* lns_bqp_eval_all -- f(x xor F_r) of every neighbour r of x, by lexicographic rank.
+ *   x: (host|device) n uint8 0/1.  fitness_out: (host|device) C(n,k) int32.  Synchronous
+ *   (ordered after `stream`). Errors: EINVAL (k not 1..3, n < k, x not 0/1), ERANGE
+ *   (C(n,k) >= 2^32 - 1), ENOMEM, ECUDA. */
+lns_status lns_bqp_eval_all(lns_bqp *ctx, int32_t k, const uint8_t *x, int32_t *fitness_out, void *stream);
+
+/* lns_bqp_tabu_run -- `iters` iterations of the tabu search from x0 ((host|device) n uint8 0/1),
+ *   tenure < 0 -> floor(C(n,k)/6). Outputs (each may be NULL except res; host or device):
+ *   x_out n uint8, trace_rank / trace_fit `iters` int64 (accepted rank and fitness per
+ *   iteration), res[4] (host) = {iterations done, final f, best f, first iteration reaching best
+ *   f (0 = x0)}. Synchronous (ordered after `stream`; the library runs on a private stream
+ *   and replays the per-iteration eval + apply launches from a CUDA graph).
+ *   Errors: EINVAL, ERANGE (tenure >= C(n,k), iters + tenure >= 2^32), ENOMEM, ECUDA. */
+lns_status lns_bqp_tabu_run(lns_bqp *ctx, int32_t k, int64_t iters, int64_t tenure, const uint8_t *x0,
+                            uint8_t *x_out, int64_t *trace_rank, int64_t *trace_fit, int64_t *res,
+                            void *stream);
+
+/* lns_bqp_last_kernel_ms -- device time (CUDA events) of the last eval_all / tabu_run (-1: NULL). */
+double lns_bqp_last_kernel_ms(const lns_bqp *ctx);
+
 #ifdef __cplusplus
 }
 #endif

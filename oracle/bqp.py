@@ -64,7 +64,7 @@ def eval_all(Q, x, k: int) -> np.ndarray:
     Xp = np.repeat(x[None, :], len(F), axis=0)
     rows = np.arange(len(F))[:, None]
     Xp[rows, F] ^= 1
-    return np.einsum("ri,ij,rj->r", Xp, Q, Xp)
+    return np.sum((Xp @ Q) * Xp, axis=1)  # row r: x_r'^T Q x_r'
 
 
 def tabu_run(Q, x0, k: int, iters: int, tenure: int = -1):

@@ -82,6 +82,11 @@ _SIGS = {
     "lns_version": (_i32, []),
     "lns_pool_trim": (None, []),
     "lns_pool_stats": (None, [ctypes.POINTER(_i64), ctypes.POINTER(_i64)]),
+    "lns_bqp_create": (_i32, [_vp, _i32, _i32, ctypes.POINTER(_vp)]),
+    "lns_bqp_destroy": (None, [_vp]),
+    "lns_bqp_eval_all": (_i32, [_vp, _i32, _vp, _vp, _vp]),
+    "lns_bqp_tabu_run": (_i32, [_vp, _i32, _i64, _i64, _vp, _vp, _vp, _vp, _vp, _vp]),
+    "lns_bqp_last_kernel_ms": (ctypes.c_double, [_vp]),
 }
 
 
@@ -127,7 +132,8 @@ def _ptr(x, dtype) -> tuple[Optional[int], Any]:
     except ImportError:  # pragma: no cover
         torch = None
     if torch is not None and isinstance(x, torch.Tensor):
-        tdt = {np.int8: torch.int8, np.int32: torch.int32, np.int64: torch.int64, np.uint32: torch.int32}[dtype]
+        tdt = {np.int8: torch.int8, np.uint8: torch.uint8, np.int32: torch.int32, np.int64: torch.int64,
+               np.uint32: torch.int32}[dtype]
         t = x.contiguous()
         if t.dtype != tdt:
             t = t.to(tdt)
@@ -146,7 +152,7 @@ def _out_ptr(x, dtype):
     import torch
 
     assert isinstance(x, torch.Tensor) and x.is_contiguous()
-    want = {np.int8: torch.int8, np.int32: torch.int32, np.int64: torch.int64}[dtype]
+    want = {np.int8: torch.int8, np.uint8: torch.uint8, np.int32: torch.int32, np.int64: torch.int64}[dtype]
     assert x.dtype == want, f"output tensor must be {want}"
     return x.data_ptr()
 
@@ -355,3 +361,52 @@ class Instance:
         res = lns_tabu_run(self.ctx, k, iters, tenure, seed, V0, fl, Vo, tr, tf, stream)
         it = res["iters_done"]
         return (tr[:it] if trace else None), (tf[:it] if trace else None), Vo, res
+
+
+# --------------------------------------------------------------------------- UBQP
+BQP_RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter")
+
+
+def lns_bqp_create(Q, device: int = 0) -> int:
+    """Upload a symmetric int32 n x n matrix Q (f(x) = x^T Q x, x in {0,1}^n); returns the handle."""
+    n = int(tuple(Q.shape)[0])
+    pq, kq = _ptr(Q, np.int32)
+    out = _vp()
+    _check(load().lns_bqp_create(pq, n, device, ctypes.byref(out)), "lns_bqp_create")
+    return out.value
+
+
+def lns_bqp_destroy(ctx: int) -> None:
+    load().lns_bqp_destroy(ctx)
+
+
+def lns_bqp_eval_all(ctx: int, k: int, x, out=None, stream=None):
+    """f(x xor F_r) for every rank r (int32); `out` may be a device tensor."""
+    if out is None:
+        out = np.empty(lns_neighborhood_size(len(x), k), dtype=np.int32)
+    px, kx = _ptr(x, np.uint8)
+    _check(load().lns_bqp_eval_all(ctx, k, px, _out_ptr(out, np.int32), _stream(stream)), "lns_bqp_eval_all")
+    return out
+
+
+def lns_bqp_tabu_run(ctx: int, k: int, iters: int, tenure: int = -1, x0=None, x_out=None,
+                     trace: bool = True, stream=None):
+    """(trace_rank, trace_fit, x_out, result dict) of `iters` tabu iterations from x0 (uint8 0/1)."""
+    n = len(x0)
+    px, kx = _ptr(x0, np.uint8)
+    if x_out is None:
+        x_out = np.empty(n, dtype=np.uint8)
+    tr = np.empty(max(iters, 1), dtype=np.int64) if trace else None
+    tf = np.empty(max(iters, 1), dtype=np.int64) if trace else None
+    res = np.zeros(4, dtype=np.int64)
+    _check(load().lns_bqp_tabu_run(ctx, k, iters, tenure, px, _out_ptr(x_out, np.uint8),
+                                   None if tr is None else tr.ctypes.data,
+                                   None if tf is None else tf.ctypes.data, res.ctypes.data, _stream(stream)),
+           "lns_bqp_tabu_run")
+    d = dict(zip(BQP_RESULT_FIELDS, (int(v) for v in res)))
+    it = d["iters_done"]
+    return (None if tr is None else tr[:it].copy()), (None if tf is None else tf[:it].copy()), x_out, d
+
+
+def lns_bqp_last_kernel_ms(ctx: int) -> float:
+    return float(load().lns_bqp_last_kernel_ms(ctx))

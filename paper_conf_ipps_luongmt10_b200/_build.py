@@ -8,6 +8,7 @@ import sys
 PKG = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(PKG)
 SRC = [os.path.join(PKG, "csrc", "lns.cu")]
+DEPS = [os.path.join(PKG, "csrc", "bqp.cuh")]  # included by lns.cu
 HDR = [os.path.join(ROOT, "include", "lns.h")]
 LIB = os.path.join(PKG, "liblns.so")
 
@@ -29,7 +30,7 @@ def stale() -> bool:
     if not os.path.exists(LIB):
         return True
     t = os.path.getmtime(LIB)
-    return any(os.path.getmtime(p) > t for p in SRC + HDR)
+    return any(os.path.getmtime(p) > t for p in SRC + DEPS + HDR)
 
 
 LIB_PROF = os.path.join(PKG, "liblns_prof.so")  # -DLNS_PHASE_TIMING variant for tools/profiling

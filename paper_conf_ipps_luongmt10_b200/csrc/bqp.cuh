@@ -1,0 +1,411 @@
+// bqp.cuh -- the k-Hamming tabu search on a second binary fitness: UBQP, f(x) = x^T Q x over
+// x in {0,1}^n (SURVEY.md §8(f) f4 "a pluggable binary fitness"). Included at
+// the end of lns.cu (same translation unit: shares fail / CK / DeviceGuard / pool_alloc).
+//
+// The paper's mappings are stated "for binary problems"; only the
+// fitness changes. The neighbourhood, rank order (reading R6), tabu list (R3), selection (R5) and
+// key packing are those of the PPP path. Incremental evaluation (derived in DESIGN.md §5.13):
+// with g = Q x and d_i = 1 - 2 x_i, flipping F changes f by
+//     sum_{i in F} h_i + 2 sum_{i<j in F} d_i d_j Q_ij,   h_i = 2 d_i g_i + Q_ii,
+// so a neighbour costs k table reads and C(k,2) reads of Q (rows of the flip set, L1/L2
+// resident); the move updates g with k rows of Q (g_j += sum_{i in F} d_i Q_ij).
+namespace {
+
+constexpr int BQ_NT = 256;      // eval CTA
+constexpr int BQ_AT = 1024;     // init / apply CTA
+constexpr int BQ_N_MAX = 4096;
+enum { BS_F = 0, BS_T, BS_BEST, BS_BESTIT, BS_ERR, BS_N };  // state (int64); ERR: 1 bad x, 2 no move
+
+__device__ __forceinline__ uint64_t bq_comb(uint64_t x, int e)
+{
+    return e == 1 ? x : e == 2 ? x * (x - 1) / 2 : x * (x - 1) * (x - 2) / 6;  // 0 for x < e
+}
+
+// Lexicographic unranking (reading R6) by the combinatorial number system:
+// M - 1 - r = sum_e C(n-1-i_{K-e}, e); each term is the largest C(z, e) <= remainder (binary search).
+template <int K>
+__device__ __forceinline__ void bq_unrank(uint64_t r, int n, uint64_t M, int *idx)
+{
+    uint64_t R = M - 1 - r;
+    int top = n - 1;
+#pragma unroll
+    for (int e = K; e >= 1; e--) {
+        int lo = e - 1, hi = top;  // C(lo, e) = 0 <= R
+        while (lo < hi) {
+            const int mid = (lo + hi + 1) >> 1;
+            if (bq_comb((uint64_t)mid, e) <= R) lo = mid; else hi = mid - 1;
+        }
+        idx[K - e] = n - 1 - lo;
+        R -= bq_comb((uint64_t)lo, e);
+        top = lo - 1;
+    }
+}
+
+template <int K>
+__device__ __forceinline__ void bq_succ(int n, int *idx)
+{
+    int i = K - 1;
+    while (i > 0 && idx[i] == n - K + i) i--;
+    idx[i]++;
+#pragma unroll
+    for (int j = 1; j < K; j++)
+        if (j > i) idx[j] = idx[j - 1] + 1;
+}
+
+__device__ __forceinline__ unsigned long long bq_key(int32_t f, uint32_t r)
+{
+    return ((unsigned long long)((uint32_t)f ^ 0x80000000u) << 32) | r;  // order-preserving
+}
+
+// g = Q x, f = x^T g, state reset; x entries must be 0 or 1.
+__global__ void __launch_bounds__(BQ_AT) k_bqp_init(const int32_t *__restrict__ Q, int n,
+                                                    const uint8_t *__restrict__ x, int32_t *__restrict__ g,
+                                                    int64_t *st)
+{
+    __shared__ unsigned long long s_f;
+    __shared__ int s_bad;
+    if (threadIdx.x == 0) { s_f = 0; s_bad = 0; }
+    __syncthreads();
+    long long part = 0;
+    for (int j = threadIdx.x; j < n; j += blockDim.x) {
+        int acc = 0;
+        for (int i = 0; i < n; i++) acc += x[i] ? Q[(size_t)i * n + j] : 0;  // Q symmetric: column j
+        g[j] = acc;
+        if (x[j] > 1) s_bad = 1;
+        part += x[j] ? (long long)acc : 0;
+    }
+    atomicAdd(&s_f, (unsigned long long)part);
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        const int64_t f = (int64_t)s_f;
+        st[BS_F] = f; st[BS_T] = 0; st[BS_BEST] = f; st[BS_BESTIT] = 0; st[BS_ERR] = s_bad ? 1 : 0;
+    }
+}
+
+// Every neighbour of iteration t = st[T] + 1: fitness (fit_out, optional) and the least admissible
+// key (until[r] < t; until == nullptr: all admissible) MIN-reduced into *key.
+template <int K>
+__global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ Q, int n, uint64_t M,
+                                                    const uint8_t *__restrict__ x, const int32_t *__restrict__ g,
+                                                    const int64_t *__restrict__ st, const uint32_t *__restrict__ until,
+                                                    int32_t *__restrict__ fit_out, unsigned long long *key)
+{
+    extern __shared__ int32_t s_h[];  // h_i = 2 d_i g_i + Q_ii, then d_i (n + n ints)
+    int32_t *s_d = s_h + n;
+    __shared__ unsigned long long s_key;
+    if (st[BS_ERR]) return;  // uniform over the grid
+    for (int i = threadIdx.x; i < n; i += blockDim.x) {
+        const int d = 1 - 2 * (int)x[i];
+        s_d[i] = d;
+        s_h[i] = 2 * d * g[i] + Q[(size_t)i * n + i];
+    }
+    if (threadIdx.x == 0) s_key = (unsigned long long)KEY_NONE;
+    __syncthreads();
+    const int32_t f0 = (int32_t)st[BS_F];
+    const uint32_t t = (uint32_t)(st[BS_T] + 1);
+    const uint64_t T = (uint64_t)gridDim.x * blockDim.x;
+    const uint64_t per = (M + T - 1) / T;
+    const uint64_t lo = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) * per;
+    const uint64_t hi = min(M, lo + per);
+    unsigned long long best = (unsigned long long)KEY_NONE;
+    if (lo < hi) {
+        int idx[K];
+        bq_unrank<K>(lo, n, M, idx);
+        for (uint64_t r = lo; r < hi; r++) {
+            // modular (u32) sums: every partial term fits int32 and so does f0 + delta
+            // (|f| <= sum |Q_ij| < 2^29), so the wrapped total is exact
+            uint32_t delta = (uint32_t)s_h[idx[0]];
+            if (K >= 2) {
+                const int d01 = s_d[idx[0]] * s_d[idx[1]];
+                delta += (uint32_t)s_h[idx[1]] + (uint32_t)(2 * d01 * Q[(size_t)idx[0] * n + idx[1]]);
+            }
+            if (K == 3) {
+                const int d02 = s_d[idx[0]] * s_d[idx[2]], d12 = s_d[idx[1]] * s_d[idx[2]];
+                delta += (uint32_t)s_h[idx[2]] + (uint32_t)(2 * d02 * Q[(size_t)idx[0] * n + idx[2]]) +
+                         (uint32_t)(2 * d12 * Q[(size_t)idx[1] * n + idx[2]]);
+            }
+            const int32_t fr = (int32_t)((uint32_t)f0 + delta);
+            if (fit_out) fit_out[r] = fr;
+            if (!until || until[r] < t) best = min(best, bq_key(fr, (uint32_t)r));
+            if (r + 1 < hi) bq_succ<K>(n, idx);
+        }
+    }
+    best = warp_min_k(best);
+    if ((threadIdx.x & 31) == 0 && best != (unsigned long long)KEY_NONE) atomicMin(&s_key, best);
+    __syncthreads();
+    if (threadIdx.x == 0 && s_key != (unsigned long long)KEY_NONE) atomicMin(key, s_key);
+}
+
+// Apply the winning move of iteration t = st[T] + 1: x ^= F, g += sum_{i in F} d_i Q_i., until[r] =
+// t + L, trace, best; *key reset for the next iteration. One CTA.
+template <int K>
+__global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__ Q, int n, uint64_t M,
+                                                     uint8_t *x, int32_t *g, int64_t *st, uint32_t *until,
+                                                     int64_t L, unsigned long long *key, int64_t *trace_r,
+                                                     int64_t *trace_f)
+{
+    if (st[BS_ERR]) return;
+    const unsigned long long kv = *key;
+    if (kv == (unsigned long long)KEY_NONE) {
+        if (threadIdx.x == 0) st[BS_ERR] = 2;
+        return;
+    }
+    const uint32_t r = (uint32_t)(kv & 0xffffffffu);
+    const int32_t f = (int32_t)((uint32_t)(kv >> 32) ^ 0x80000000u);
+    int idx[K], d[K];
+    bq_unrank<K>(r, n, M, idx);
+#pragma unroll
+    for (int q = 0; q < K; q++) d[q] = 1 - 2 * (int)x[idx[q]];
+    for (int j = threadIdx.x; j < n; j += blockDim.x) {
+        int acc = g[j];
+#pragma unroll
+        for (int q = 0; q < K; q++) acc += d[q] * Q[(size_t)idx[q] * n + j];
+        g[j] = acc;
+    }
+    __syncthreads();  // every thread has read x[F] before it flips
+    if (threadIdx.x == 0) {
+#pragma unroll
+        for (int q = 0; q < K; q++) x[idx[q]] ^= 1;
+        const int64_t t = st[BS_T] + 1;
+        until[r] = (uint32_t)(t + L);
+        if (trace_r) { trace_r[t - 1] = r; trace_f[t - 1] = f; }
+        st[BS_F] = f; st[BS_T] = t;
+        if (f < st[BS_BEST]) { st[BS_BEST] = f; st[BS_BESTIT] = t; }
+        *key = (unsigned long long)KEY_NONE;
+    }
+}
+
+}  // namespace
+
+struct lns_bqp {
+    int device = 0, n = 0, nsm = 148;
+    int32_t *d_Q = nullptr, *d_g = nullptr, *d_fit = nullptr;
+    uint8_t *d_x = nullptr;
+    int64_t *d_st = nullptr, *d_tr = nullptr, *d_tf = nullptr;
+    uint32_t *d_until = nullptr;
+    unsigned long long *d_key = nullptr;
+    size_t fit_cap = 0, until_cap = 0, tr_cap = 0;
+    cudaStream_t st = nullptr;
+    cudaEvent_t ev0 = nullptr, ev1 = nullptr, evu = nullptr;
+    float last_ms = 0;
+};
+
+namespace {
+
+lns_status bqp_check_k(const lns_bqp *c, int32_t k, uint64_t &M)
+{
+    if (!c) return fail(LNS_EINVAL, "null context");
+    if (k < 1 || k > 3) return fail(LNS_EINVAL, "UBQP: k must be 1, 2 or 3");
+    if (c->n < k) return fail(LNS_EINVAL, "n < k");
+    M = (uint64_t)comb_k(c->n, k);
+    if (M >= 0xffffffffull) return fail(LNS_ERANGE, "C(n,k) >= 2^32 - 1");
+    return LNS_OK;
+}
+
+int bqp_blocks(const lns_bqp *c, uint64_t M)
+{
+    const uint64_t want = (M + BQ_NT - 1) / BQ_NT;
+    return (int)std::max<uint64_t>(1, std::min<uint64_t>(want, (uint64_t)c->nsm * 8));
+}
+
+lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, const uint32_t *until, int32_t *fit)
+{
+    const int nb = bqp_blocks(c, M);
+    const size_t sm = 2 * sizeof(int32_t) * (size_t)c->n;
+    switch (k) {
+    case 1: k_bqp_eval<1><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
+    case 2: k_bqp_eval<2><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
+    default: k_bqp_eval<3><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
+    }
+    CK(cudaGetLastError());
+    return LNS_OK;
+}
+
+lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, int64_t L, bool trace)
+{
+    int64_t *tr = trace ? c->d_tr : nullptr, *tf = trace ? c->d_tf : nullptr;
+    switch (k) {
+    case 1: k_bqp_apply<1><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
+    case 2: k_bqp_apply<2><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
+    default: k_bqp_apply<3><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
+    }
+    CK(cudaGetLastError());
+    return LNS_OK;
+}
+
+// Order the private stream after the caller's stream (inputs the caller wrote there).
+lns_status bqp_enter(lns_bqp *c, void *stream)
+{
+    CK(cudaEventRecord(c->evu, (cudaStream_t)stream));
+    CK(cudaStreamWaitEvent(c->st, c->evu, 0));
+    return LNS_OK;
+}
+
+lns_status bqp_start(lns_bqp *c, const uint8_t *x)
+{
+    CK(cudaMemcpyAsync(c->d_x, x, (size_t)c->n, cudaMemcpyDefault, c->st));
+    k_bqp_init<<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, c->d_x, c->d_g, c->d_st);
+    CK(cudaGetLastError());
+    const unsigned long long none = (unsigned long long)KEY_NONE;
+    CK(cudaMemcpyAsync(c->d_key, &none, sizeof(none), cudaMemcpyHostToDevice, c->st));
+    return LNS_OK;
+}
+
+}  // namespace
+
+extern "C" {
+
+lns_status lns_bqp_create(const int32_t *Q, int32_t n, int32_t device, lns_bqp **out)
+{
+    if (!out || !Q) return fail(LNS_EINVAL, "null argument");
+    *out = nullptr;
+    if (n < 1) return fail(LNS_EINVAL, "n must be >= 1");
+    if (n > BQ_N_MAX) return fail(LNS_ERANGE, "n > 4096");
+    int ndev = 0;
+    CK(cudaGetDeviceCount(&ndev));
+    if (device < 0 || device >= ndev) return fail(LNS_EINVAL, "bad device index");
+    std::vector<int32_t> hQ((size_t)n * n);  // Q may live on the host or on a device (UVA copy)
+    CK(cudaMemcpy(hQ.data(), Q, sizeof(int32_t) * hQ.size(), cudaMemcpyDefault));
+    Q = hQ.data();
+    int64_t absum = 0;
+    for (int64_t i = 0; i < n; i++)
+        for (int64_t j = 0; j < n; j++) {
+            const int32_t q = Q[i * n + j];
+            if (q != Q[j * n + i]) return fail(LNS_EINVAL, "Q must be symmetric");
+            absum += q < 0 ? -(int64_t)q : (int64_t)q;
+        }
+    // |f(x)|, |f(x')|, |g_i| and |Q_ii| are bounded by S = sum |Q_ij| < 2^29, so h_i (< 3 S),
+    // the 2 Q_ij pair terms and every fitness fit int32 (the eval kernel sums them mod 2^32)
+    if (absum >= ((int64_t)1 << 29)) return fail(LNS_ERANGE, "sum |Q_ij| >= 2^29");
+    DeviceGuard dg(device);
+    lns_bqp *c = new lns_bqp();
+    c->device = device;
+    c->n = n;
+    cudaDeviceGetAttribute(&c->nsm, cudaDevAttrMultiProcessorCount, device);
+    bool ok = pool_alloc(&c->d_Q, sizeof(int32_t) * (size_t)n * n) == cudaSuccess &&
+              pool_alloc(&c->d_g, sizeof(int32_t) * (size_t)n) == cudaSuccess &&
+              pool_alloc(&c->d_x, (size_t)n) == cudaSuccess &&
+              pool_alloc(&c->d_st, sizeof(int64_t) * BS_N) == cudaSuccess &&
+              pool_alloc(&c->d_key, sizeof(unsigned long long)) == cudaSuccess;
+    if (!ok) { lns_bqp_destroy(c); return fail(LNS_ENOMEM, "cudaMalloc failed"); }
+    if (cudaStreamCreateWithFlags(&c->st, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreate(&c->ev0) != cudaSuccess || cudaEventCreate(&c->ev1) != cudaSuccess ||
+        cudaEventCreateWithFlags(&c->evu, cudaEventDisableTiming) != cudaSuccess) {
+        lns_bqp_destroy(c);
+        return fail(LNS_ECUDA, "stream / event creation failed");
+    }
+    if (cudaMemcpy(c->d_Q, Q, sizeof(int32_t) * (size_t)n * n, cudaMemcpyDefault) != cudaSuccess) {
+        lns_bqp_destroy(c);
+        return fail(LNS_ECUDA, "copy of Q failed");
+    }
+    *out = c;
+    return LNS_OK;
+}
+
+void lns_bqp_destroy(lns_bqp *c)
+{
+    if (!c) return;
+    DeviceGuard dg(c->device);
+    if (c->st) cudaStreamSynchronize(c->st);
+    pool_free(c->d_Q); pool_free(c->d_g); pool_free(c->d_x); pool_free(c->d_st); pool_free(c->d_key);
+    pool_free(c->d_fit); pool_free(c->d_until); pool_free(c->d_tr); pool_free(c->d_tf);
+    if (c->ev0) cudaEventDestroy(c->ev0);
+    if (c->ev1) cudaEventDestroy(c->ev1);
+    if (c->evu) cudaEventDestroy(c->evu);
+    if (c->st) cudaStreamDestroy(c->st);
+    delete c;
+}
+
+lns_status lns_bqp_eval_all(lns_bqp *c, int32_t k, const uint8_t *x, int32_t *fitness_out, void *stream)
+{
+    uint64_t M;
+    lns_status s = bqp_check_k(c, k, M);
+    if (s != LNS_OK) return s;
+    if (!x || !fitness_out) return fail(LNS_EINVAL, "null argument");
+    DeviceGuard dg(c->device);
+    if ((s = grow(c->d_fit, c->fit_cap, M)) != LNS_OK) return s;
+    if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
+    if ((s = bqp_start(c, x)) != LNS_OK) return s;
+    CK(cudaEventRecord(c->ev0, c->st));
+    if ((s = bqp_launch_eval(c, k, M, nullptr, c->d_fit)) != LNS_OK) return s;
+    CK(cudaEventRecord(c->ev1, c->st));
+    int64_t hs[BS_N];
+    CK(cudaMemcpyAsync(hs, c->d_st, sizeof(hs), cudaMemcpyDeviceToHost, c->st));
+    CK(cudaMemcpyAsync(fitness_out, c->d_fit, sizeof(int32_t) * M, cudaMemcpyDefault, c->st));
+    CK(cudaStreamSynchronize(c->st));
+    cudaEventElapsedTime(&c->last_ms, c->ev0, c->ev1);
+    if (hs[BS_ERR] == 1) return fail(LNS_EINVAL, "x must be 0/1");
+    return LNS_OK;
+}
+
+lns_status lns_bqp_tabu_run(lns_bqp *c, int32_t k, int64_t iters, int64_t tenure, const uint8_t *x0,
+                            uint8_t *x_out, int64_t *trace_rank, int64_t *trace_fit, int64_t *res, void *stream)
+{
+    uint64_t M;
+    lns_status s = bqp_check_k(c, k, M);
+    if (s != LNS_OK) return s;
+    if (!x0 || !res) return fail(LNS_EINVAL, "null argument");
+    if (iters < 0 || iters >= ((int64_t)1 << 31)) return fail(LNS_EINVAL, "iters outside [0, 2^31)");
+    const int64_t L = tenure < 0 ? (int64_t)(M / 6) : tenure;
+    if ((uint64_t)L >= M) return fail(LNS_ERANGE, "tenure >= C(n,k)");
+    if (iters + L >= ((int64_t)1 << 32) - 1) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    DeviceGuard dg(c->device);
+    const bool trace = trace_rank || trace_fit;
+    if ((s = grow(c->d_until, c->until_cap, M)) != LNS_OK) return s;
+    if (trace && c->tr_cap < (size_t)std::max<int64_t>(iters, 1)) {
+        pool_free(c->d_tr); pool_free(c->d_tf);
+        c->d_tr = c->d_tf = nullptr; c->tr_cap = 0;
+        const size_t cap = (size_t)std::max<int64_t>(iters, 1);
+        if (pool_alloc(&c->d_tr, 8 * cap) != cudaSuccess || pool_alloc(&c->d_tf, 8 * cap) != cudaSuccess)
+            return fail(LNS_ENOMEM, "cudaMalloc failed");
+        c->tr_cap = cap;
+    }
+    if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
+    CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * M, c->st));
+    if ((s = bqp_start(c, x0)) != LNS_OK) return s;
+    CK(cudaEventRecord(c->ev0, c->st));
+    // Every launch reads the iteration number from the device state, so a block of G iterations
+    // is captured once into a CUDA graph and replayed (no host round trip per iteration).
+    const int64_t G = std::min<int64_t>(iters, 64);
+    int64_t done = 0;
+    if (G > 0 && iters / G >= 2) {
+        cudaGraph_t graph = nullptr;
+        cudaGraphExec_t exec = nullptr;
+        CK(cudaStreamBeginCapture(c->st, cudaStreamCaptureModeThreadLocal));
+        for (int64_t q = 0; q < G; q++) {
+            lns_status e1 = bqp_launch_eval(c, k, M, c->d_until, nullptr);
+            lns_status e2 = e1 == LNS_OK ? bqp_launch_apply(c, k, M, L, trace) : e1;
+            if (e2 != LNS_OK) { cudaStreamEndCapture(c->st, &graph); if (graph) cudaGraphDestroy(graph); return e2; }
+        }
+        CK(cudaStreamEndCapture(c->st, &graph));
+        cudaError_t e = cudaGraphInstantiate(&exec, graph, 0);
+        cudaGraphDestroy(graph);
+        if (e != cudaSuccess) return fail(LNS_ECUDA, std::string("cudaGraphInstantiate: ") + cudaGetErrorString(e));
+        for (; done + G <= iters; done += G) {
+            e = cudaGraphLaunch(exec, c->st);
+            if (e != cudaSuccess) { cudaGraphExecDestroy(exec); return fail(LNS_ECUDA, cudaGetErrorString(e)); }
+        }
+        cudaGraphExecDestroy(exec);
+    }
+    for (; done < iters; done++) {
+        if ((s = bqp_launch_eval(c, k, M, c->d_until, nullptr)) != LNS_OK) return s;
+        if ((s = bqp_launch_apply(c, k, M, L, trace)) != LNS_OK) return s;
+    }
+    CK(cudaEventRecord(c->ev1, c->st));
+    int64_t hs[BS_N];
+    CK(cudaMemcpyAsync(hs, c->d_st, sizeof(hs), cudaMemcpyDeviceToHost, c->st));
+    if (x_out) CK(cudaMemcpyAsync(x_out, c->d_x, (size_t)c->n, cudaMemcpyDefault, c->st));
+    CK(cudaStreamSynchronize(c->st));
+    const int64_t nt = hs[BS_T];
+    if (trace_rank && nt > 0) CK(cudaMemcpy(trace_rank, c->d_tr, 8 * (size_t)nt, cudaMemcpyDefault));
+    if (trace_fit && nt > 0) CK(cudaMemcpy(trace_fit, c->d_tf, 8 * (size_t)nt, cudaMemcpyDefault));
+    cudaEventElapsedTime(&c->last_ms, c->ev0, c->ev1);
+    res[0] = nt; res[1] = hs[BS_F]; res[2] = hs[BS_BEST]; res[3] = hs[BS_BESTIT];
+    if (hs[BS_ERR] == 1) return fail(LNS_EINVAL, "x0 must be 0/1");
+    if (hs[BS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "every neighbour is tabu");
+    return LNS_OK;
+}
+
+double lns_bqp_last_kernel_ms(const lns_bqp *c) { return c ? (double)c->last_ms : -1.0; }
+
+}  // extern "C"

@@ -3822,3 +3822,5 @@ lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count,
 }
 
 }  // extern "C"
+
+#include "bqp.cuh"  // second binary fitness (UBQP), DESIGN.md §5.13
