@@ -14,6 +14,9 @@ namespace {
 constexpr int BQ_NT = 256;      // eval CTA
 constexpr int BQ_AT = 1024;     // init / apply CTA
 constexpr int BQ_N_MAX = 4096;
+// Keys span the whole u64 range (the biased fitness fills the high word), so "none" is all ones:
+// a real key has r < 2^32 - 1 in its low word.
+constexpr unsigned long long BQ_NONE = ~0ull;
 enum { BS_F = 0, BS_T, BS_BEST, BS_BESTIT, BS_ERR, BS_N };  // state (int64); ERR: 1 bad x, 2 no move
 
 __device__ __forceinline__ uint64_t bq_comb(uint64_t x, int e)
@@ -99,7 +102,7 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
         s_d[i] = d;
         s_h[i] = 2 * d * g[i] + Q[(size_t)i * n + i];
     }
-    if (threadIdx.x == 0) s_key = (unsigned long long)KEY_NONE;
+    if (threadIdx.x == 0) s_key = BQ_NONE;
     __syncthreads();
     const int32_t f0 = (int32_t)st[BS_F];
     const uint32_t t = (uint32_t)(st[BS_T] + 1);
@@ -107,7 +110,7 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     const uint64_t per = (M + T - 1) / T;
     const uint64_t lo = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) * per;
     const uint64_t hi = min(M, lo + per);
-    unsigned long long best = (unsigned long long)KEY_NONE;
+    unsigned long long best = BQ_NONE;
     if (lo < hi) {
         int idx[K];
         bq_unrank<K>(lo, n, M, idx);
@@ -131,9 +134,9 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
         }
     }
     best = warp_min_k(best);
-    if ((threadIdx.x & 31) == 0 && best != (unsigned long long)KEY_NONE) atomicMin(&s_key, best);
+    if ((threadIdx.x & 31) == 0 && best != BQ_NONE) atomicMin(&s_key, best);
     __syncthreads();
-    if (threadIdx.x == 0 && s_key != (unsigned long long)KEY_NONE) atomicMin(key, s_key);
+    if (threadIdx.x == 0 && s_key != BQ_NONE) atomicMin(key, s_key);
 }
 
 // Apply the winning move of iteration t = st[T] + 1: x ^= F, g += sum_{i in F} d_i Q_i., until[r] =
@@ -146,7 +149,7 @@ __global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__
 {
     if (st[BS_ERR]) return;
     const unsigned long long kv = *key;
-    if (kv == (unsigned long long)KEY_NONE) {
+    if (kv == BQ_NONE) {
         if (threadIdx.x == 0) st[BS_ERR] = 2;
         return;
     }
@@ -171,7 +174,7 @@ __global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__
         if (trace_r) { trace_r[t - 1] = r; trace_f[t - 1] = f; }
         st[BS_F] = f; st[BS_T] = t;
         if (f < st[BS_BEST]) { st[BS_BEST] = f; st[BS_BESTIT] = t; }
-        *key = (unsigned long long)KEY_NONE;
+        *key = BQ_NONE;
     }
 }
 
@@ -246,7 +249,7 @@ lns_status bqp_start(lns_bqp *c, const uint8_t *x)
     CK(cudaMemcpyAsync(c->d_x, x, (size_t)c->n, cudaMemcpyDefault, c->st));
     k_bqp_init<<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, c->d_x, c->d_g, c->d_st);
     CK(cudaGetLastError());
-    const unsigned long long none = (unsigned long long)KEY_NONE;
+    const unsigned long long none = BQ_NONE;
     CK(cudaMemcpyAsync(c->d_key, &none, sizeof(none), cudaMemcpyHostToDevice, c->st));
     return LNS_OK;
 }

@@ -101,6 +101,34 @@ def test_tabu_trajectory_bit_exact(L, k, n, iters, tenure):
     assert np.array_equal(tr, otr) and np.array_equal(tf, otf) and np.array_equal(xo, oxo)
 
 
+@pytest.mark.parametrize("k", [1, 2, 3])
+def test_positive_and_mixed_sign_fitnesses(L, k):
+    """Q >= 0 from x = 0: every neighbour has f > 0 (the key's biased high word above 2^31), then
+    trajectories that cross from positive to negative fitness: keys order correctly across the
+    sign boundary."""
+    n = 24
+    Q = np.abs(bi.random_q(n, 0.5, 21 + k)) + np.eye(n, dtype=np.int32)
+    x0 = np.zeros(n, np.uint8)
+    ctx = L.lns_bqp_create(Q, 0)
+    try:
+        got = L.lns_bqp_eval_all(ctx, k, x0).astype(np.int64)
+        assert got.min() > 0 and np.array_equal(got, bqp.eval_all(Q, x0, k))
+        tr, tf, xo, res = L.lns_bqp_tabu_run(ctx, k, 70, -1, x0)
+        otr, otf, oxo, ores = bqp.tabu_run(Q, x0, k, 70, -1)
+        assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+    finally:
+        L.lns_bqp_destroy(ctx)
+    Q2 = bi.random_q(n, 0.5, 31 + k) + 60 * np.eye(n, dtype=np.int32)  # mixed signs around 0
+    ctx = L.lns_bqp_create(Q2, 0)
+    try:
+        for x in _states(n, 3):
+            tr, tf, xo, res = L.lns_bqp_tabu_run(ctx, k, 80, -1, x)
+            otr, otf, oxo, ores = bqp.tabu_run(Q2, x, k, 80, -1)
+            assert res == ores and np.array_equal(tr, otr) and np.array_equal(tf, otf)
+    finally:
+        L.lns_bqp_destroy(ctx)
+
+
 def test_tabu_reaches_planted_optimum(L):
     """Planted Ising (closed-form optimum -n^2 + (sum z)^2, DESIGN.md §5.13): k = 2 from a random x;
     same trajectory as the oracle, and the optimum is reached."""
