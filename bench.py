@@ -20,6 +20,8 @@ over ranks), inputs resident in HBM. ``e2e`` = the same job through the C ABI wi
 (instance upload, start vectors, final vectors and results back inside the timed region).
 ``single_search`` = one search at a time (latency view: all SMs on one search, 2,000 iterations).
 ``c5_single_search`` = BASELINE configs[4] (1024 x 1024, 3-Hamming), one search, 5 iterations.
+``ubqp_single_search`` = the second binary fitness (UBQP): k = 3, n = 500, one
+search, 50 iterations (context; not part of the headline).
 ``roofline`` = the search kernel's integer throughput against the issue-rate peak.
 ``cpu_baseline`` = the CPU oracle on this host on a bounded sample. ``--impl reference`` times
 that oracle alone as the reference arm (this paper has no code).
@@ -213,6 +215,7 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-single", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
+    ap.add_argument("--no-ubqp", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)
     args = ap.parse_args()
     rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
@@ -364,6 +367,29 @@ def main():
               "ms_per_iteration": b5 / C5_ITERS, "iters": C5_ITERS,
               "note": "C5 single search from the config seed (packed plan for m > 255, DESIGN.md §5.11); device time of the launch"}
 
+    # ---- UBQP: k = 3, n = 500 OR-Library-style Q, one search (N = 1 only; context)
+    ubqp = None
+    if world == 1 and not args.no_ubqp:
+        from ppp_inputs import bqp as bi
+
+        nq, kq, itq = 500, 3, 50
+        Qb = bi.random_q(nq, 0.1, 1)
+        xq = bi.start_x(nq, 2)
+        cq = L.lns_bqp_create(Qb, 0)
+        L.lns_bqp_tabu_run(cq, kq, 64, -1, xq, trace=False)
+        msq = []
+        for _ in range(2):
+            flush.fill_(0)
+            torch.cuda.synchronize()
+            L.lns_bqp_tabu_run(cq, kq, itq, -1, xq, trace=False)
+            msq.append(L.lns_bqp_last_kernel_ms(cq))
+        L.lns_bqp_destroy(cq)
+        bq = min(msq)
+        Mq = L.lns_neighborhood_size(nq, kq)
+        ubqp = {"neighbors_per_s": itq * Mq / (bq / 1e3), "us_per_iteration": 1e3 * bq / itq, "iters": itq,
+                "note": "UBQP f = x^T Q x, n = 500, density 0.1, 3-Hamming (2.07e7 neighbours/iteration), one "
+                        "search; device time (eval + apply launches replayed from a CUDA graph)"}
+
     # ---- roofline: the search kernel (one launch per step)
     pk, src = peaks()
     mhz = float(pk.get("sm_max_mhz", 1965.0))
@@ -429,6 +455,7 @@ def main():
                     "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
             "single_search": single,
             "c5_single_search": c5,
+            "ubqp_single_search": ubqp,
             # our kernels per timed step: k_init_slots + the persistent k_search
             "gpu_launches": args.steps * 2,
             "clocks": clocks,
