@@ -55,6 +55,32 @@ __device__ __forceinline__ void bq_succ(int n, int *idx)
         if (j > i) idx[j] = idx[j - 1] + 1;
 }
 
+// Advance a sorted flip set by s ranks in lexicographic order (last index fastest): move the last
+// index; each time it runs past n - 1 the prefix takes its own successor (a (K-1)-subset of
+// [0, n - 2]) and the overshoot restarts after the new prefix. Exact for any s >= 0 that stays
+// inside [0, M).
+template <int K>
+__device__ __forceinline__ bool bq_advance(int n, int *idx, int s)
+{
+    int c = idx[K - 1] + s;
+    bool moved = false;
+    if (K > 1) {
+        while (c >= n) {
+            const int over = c - n;
+            int pre[K > 1 ? K - 1 : 1];
+#pragma unroll
+            for (int q = 0; q < K - 1; q++) pre[q] = idx[q];
+            bq_succ<(K > 1 ? K - 1 : 1)>(n - 1, pre);
+#pragma unroll
+            for (int q = 0; q < K - 1; q++) idx[q] = pre[q];
+            c = idx[K - 2] + 1 + over;
+            moved = true;
+        }
+    }
+    idx[K - 1] = c;
+    return moved;
+}
+
 __device__ __forceinline__ unsigned long long bq_key(int32_t f, uint32_t r)
 {
     return ((unsigned long long)((uint32_t)f ^ 0x80000000u) << 32) | r;  // order-preserving
@@ -106,31 +132,48 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     __syncthreads();
     const int32_t f0 = (int32_t)st[BS_F];
     const uint32_t t = (uint32_t)(st[BS_T] + 1);
+    // Warp-interleaved ranks: warp w owns [32 w per, 32 (w + 1) per) and lane l takes ranks
+    // base + l + 32 j, so consecutive lanes hold consecutive ranks: until[] and fit_out are
+    // coalesced, and (last index fastest) the Q row reads Q[a n + c], Q[b n + c] and the h[c], d[c]
+    // table reads hit consecutive addresses across the warp.
     const uint64_t T = (uint64_t)gridDim.x * blockDim.x;
     const uint64_t per = (M + T - 1) / T;
-    const uint64_t lo = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) * per;
-    const uint64_t hi = min(M, lo + per);
+    const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t lo = gw * 32 * per + (threadIdx.x & 31);
+    const uint64_t hi = min(M, (gw + 1) * 32 * per);
     unsigned long long best = BQ_NONE;
     if (lo < hi) {
         int idx[K];
         bq_unrank<K>(lo, n, M, idx);
-        for (uint64_t r = lo; r < hi; r++) {
-            // modular (u32) sums: every partial term fits int32 and so does f0 + delta
-            // (|f| <= sum |Q_ij| < 2^29), so the wrapped total is exact
-            uint32_t delta = (uint32_t)s_h[idx[0]];
-            if (K >= 2) {
-                const int d01 = s_d[idx[0]] * s_d[idx[1]];
-                delta += (uint32_t)s_h[idx[1]] + (uint32_t)(2 * d01 * Q[(size_t)idx[0] * n + idx[1]]);
-            }
+        // The prefix F \ {c} (all but the last index) changes only when the run wraps: its part of
+        // the delta (pre), its signs and its Q rows are kept in registers.
+        // Modular (u32) sums: every term fits int32 and so does f0 + delta (|f| <= sum |Q_ij| < 2^29),
+        // so the wrapped total is exact.
+        uint32_t pre = 0;
+        int dp0 = 0, dp1 = 0;
+        const int32_t *q0 = Q, *q1 = Q;
+        auto load_prefix = [&]() {
+            if (K >= 2) { dp0 = s_d[idx[0]]; q0 = Q + (size_t)idx[0] * n; pre = (uint32_t)s_h[idx[0]]; }
             if (K == 3) {
-                const int d02 = s_d[idx[0]] * s_d[idx[2]], d12 = s_d[idx[1]] * s_d[idx[2]];
-                delta += (uint32_t)s_h[idx[2]] + (uint32_t)(2 * d02 * Q[(size_t)idx[0] * n + idx[2]]) +
-                         (uint32_t)(2 * d12 * Q[(size_t)idx[1] * n + idx[2]]);
+                dp1 = s_d[idx[1]]; q1 = Q + (size_t)idx[1] * n;
+                pre += (uint32_t)s_h[idx[1]] + (uint32_t)(2 * dp0 * dp1 * q0[idx[1]]);
+            }
+        };
+        load_prefix();
+        for (uint32_t r = (uint32_t)lo;;) {
+            const int c = idx[K - 1];
+            uint32_t delta = pre + (uint32_t)s_h[c];
+            if (K >= 2) {
+                const int dc2 = 2 * s_d[c];
+                delta += (uint32_t)(dc2 * dp0 * q0[c]);
+                if (K == 3) delta += (uint32_t)(dc2 * dp1 * q1[c]);
             }
             const int32_t fr = (int32_t)((uint32_t)f0 + delta);
             if (fit_out) fit_out[r] = fr;
-            if (!until || until[r] < t) best = min(best, bq_key(fr, (uint32_t)r));
-            if (r + 1 < hi) bq_succ<K>(n, idx);
+            if (!until || until[r] < t) best = min(best, bq_key(fr, r));
+            if ((uint64_t)r + 32 >= hi) break;
+            r += 32;
+            if (bq_advance<K>(n, idx, 32)) load_prefix();
         }
     }
     best = warp_min_k(best);
