@@ -2,7 +2,8 @@
  * Plain-C use of the C ABI (include/lns.h), no Python or torch: build a planted PPP instance
  * (Definition 1) with its own splitmix64 stream, evaluate the 3-Hamming
  * neighbourhood once (lns_eval_neighborhood), run a tabu search (lns_tabu_run)
- * and a batch of restarts (lns_tabu_run_batch), all from host buffers.
+ * and a batch of restarts (lns_tabu_run_batch), all from host buffers; then the same search on the
+ * second binary fitness, UBQP f(x) = x^T Q x (lns_bqp_*).
  *
  *   cc -O2 -I include examples/tabu_c.c -L paper_conf_ipps_luongmt10_b200 -llns \
  *      -Wl,-rpath,$PWD/paper_conf_ipps_luongmt10_b200 -o build/tabu_c && build/tabu_c [m n k iters]
@@ -79,6 +80,32 @@ int main(int argc, char **argv)
     printf("8 restarts x %lld iterations: best f of restart 0 = %lld, %.3f ms\n", (long long)iters,
            (long long)rb[0].best_f, lns_last_kernel_ms(ctx));
     lns_destroy(ctx);
+
+    /* UBQP: symmetric Q with entries in [-100, 100] at density ~1/4, x0 = 0, 2-Hamming */
+    const int32_t nq = n < 200 ? n : 200;
+    int32_t *Q = calloc((size_t)nq * nq, sizeof(int32_t));
+    uint8_t *x0 = calloc((size_t)nq, 1), *xo = malloc((size_t)nq);
+    uint64_t sq = 2024;
+    for (int32_t i = 0; i < nq; i++)
+        for (int32_t j = i; j < nq; j++) {
+            const uint64_t z = next(&sq);
+            if ((z & 3) == 0) Q[(size_t)i * nq + j] = Q[(size_t)j * nq + i] = (int32_t)((z >> 8) % 201) - 100;
+        }
+    const int64_t Mq = lns_neighborhood_size(nq, 2);
+    int32_t *fq = malloc(sizeof(int32_t) * (size_t)Mq);
+    int64_t *trq = malloc(sizeof(int64_t) * 50), *tfq = malloc(sizeof(int64_t) * 50), rq[4];
+    lns_bqp *bq = NULL;
+    CHECK(lns_bqp_create(Q, nq, 0, &bq));
+    CHECK(lns_bqp_eval_all(bq, 2, x0, fq, NULL));
+    int64_t fmin = fq[0], rmin = 0;
+    for (int64_t r2 = 1; r2 < Mq; r2++)
+        if (fq[r2] < fmin) { fmin = fq[r2]; rmin = r2; }
+    CHECK(lns_bqp_tabu_run(bq, 2, 50, -1, x0, xo, trq, tfq, rq, NULL));
+    printf("UBQP n=%d, 2-Hamming: best neighbour of x0 f = %lld (rank %lld); 50 iterations: best f %lld, %.3f ms\n",
+           nq, (long long)fmin, (long long)rmin, (long long)rq[2], lns_bqp_last_kernel_ms(bq));
+    ok &= rq[0] == 50 && trq[0] == rmin && tfq[0] == fmin && rq[2] <= rq[1] && rq[2] <= fmin;
+    lns_bqp_destroy(bq);
+    free(Q); free(x0); free(xo); free(fq); free(trq); free(tfq);
     free(A); free(V); free(Vout); free(S); free(Y); free(tr); free(tf);
     printf(ok ? "ok\n" : "INCONSISTENT\n");
     return ok ? 0 : 2;

@@ -865,7 +865,8 @@ def test_eval_neighborhood_k_above_3_best_with_tabu(L, orc, m, n, k):
 
 
 def test_c_example_runs_on_the_gpu(L, tmp_path):
-    """examples/tabu_c.c -- the C ABI from plain C, host buffers only: eval, tabu run, batch."""
+    """examples/tabu_c.c -- the C ABI from plain C, host buffers only: eval, tabu run, batch, and the
+    UBQP calls (eval_all, tabu_run: the first move is the best neighbour of x0)."""
     import subprocess
 
     from test_abi import _build_c_example
