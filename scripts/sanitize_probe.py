@@ -34,4 +34,15 @@ big = pi.planted_instance(260, 40, 5)  # m > 255: segment-loop path, padded plac
 with L.Instance(big.A, big.S) as I:
     L.lns_config(I.ctx, 1)
     I.tabu_run(3, 4, -1, seed=2, stop_on_zero=False)
+from ppp_inputs import bqp as bi  # the UBQP kernels: eval, apply, init, graph replay
+
+bq = L.lns_bqp_create(bi.random_q(70, 0.3, 1), 0)
+try:
+    xq = bi.start_x(70, 2)
+    for k in (1, 2, 3):
+        L.lns_bqp_eval_all(bq, k, xq)
+    L.lns_bqp_tabu_run(bq, 3, 130, -1, xq)  # two graph blocks of 64 + 2 direct iterations
+    L.lns_bqp_tabu_run(bq, 2, 10, 3, xq)
+finally:
+    L.lns_bqp_destroy(bq)
 print("sanitize probe done")

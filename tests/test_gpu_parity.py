@@ -683,7 +683,7 @@ def test_pool_recycles_context_buffers(L, orc):
 @pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck"])
 def test_compute_sanitizer_clean(L, tool):
     """every kernel family (persistent search with one and several CTAs,
-    batched restarts, stepped search, eval_all, the m > 255 path) runs clean under
+    batched restarts, stepped search, eval_all, the m > 255 path, the UBQP kernels) runs clean under
     compute-sanitizer on small instances."""
     import os
     import shutil
