@@ -22,9 +22,22 @@ over ranks), inputs resident in HBM. ``e2e`` = the same job through the C ABI wi
 ``c5_single_search`` = BASELINE configs[4] (1024 x 1024, 3-Hamming), one search, 5 iterations.
 ``ubqp_single_search`` = the second binary fitness (UBQP): k = 3, n = 500, one
 search, 50 iterations (context; not part of the headline).
-``roofline`` = the search kernel's integer throughput against the issue-rate peak.
-``cpu_baseline`` = the CPU oracle on this host on a bounded sample. ``--impl reference`` times
-that oracle alone as the reference arm (this paper has no code).
+``c5_restarts`` = BASELINE configs[4]'s restart job per GPU: 8 restarts of C5 per GPU (64 on 8
+GPUs), a few iterations each, through lns_tabu_run_batch (sharded by the library over the NCCL
+communicator when N > 1).
+``partitioned`` = ONE search whose neighbourhood is partitioned over the N GPUs:
+C4 (2,000 iterations) and C5 (5 iterations) with one NCCL u64-MIN all-reduce per iteration
+(lns_attach_comm on torch's communicator), and the device-initiated exchange (peer_tabu_run, C4).
+At N = 1 it is the single-GPU persistent search.
+``roofline`` = the search kernel's issued integer instructions against the MEASURED issue peak
+(profiles/int_peaks.json), with the binding pipe (POPC on XU) against its measured peak; the
+per-neighbour instruction counts come from the committed ncu capture, which must have been taken
+from the current sources (hash check; a stale capture aborts the bench).
+``cpu_baseline`` = the CPU oracle on this host on a bounded sample, all cores and single-threaded.
+``--impl reference`` times that oracle alone as the reference arm (this paper has no code).
+
+``--gpus N`` with N > 1 and no torchrun environment re-launches this script under
+``torch.distributed.run`` with N ranks (127.0.0.1); with fewer than N visible GPUs it fails.
 """
 from __future__ import annotations
 
@@ -52,7 +65,13 @@ RUNS = 50        # independent searches per step
 ITERS = 400      # iterations per search per step
 SINGLE_ITERS = 2000
 C5_ITERS = 5     # C5 iterations timed beside the headline (9.5 ms each)
+C5_RESTARTS_PER_GPU = 8  # BASELINE configs[4]: 64 restarts sharded across 8 x B200
+C5_RESTART_ITERS = 3
+PART_C4_ITERS = 2000
+PART_C5_ITERS = 5
 L2_FLUSH_BYTES = 512 << 20  # > 126 MB L2
+PROFILE = os.path.join(ROOT, "profiles", "ncu_k_search_bench.json")  # ncu --set full of one bench step
+INT_PEAKS = os.path.join(ROOT, "profiles", "int_peaks.json")  # scripts/int_peaks.cu on the B200
 
 
 def env_int(name, default):
@@ -140,27 +159,53 @@ def start_vectors(n: int, step: int, runs) -> np.ndarray:
 
 
 # --------------------------------------------------------------------------------- oracle arm
-def oracle_sample(budget_s: float, nthreads: int = 0):
-    """The CPU oracle (as it stands) on the same job: whole runs (400 iterations each) of step 0,
-    as many as fit ~budget_s. Returns (neighbors/s, iters/s, iterations, cores, seconds)."""
+def oracle_sample(budget_s: float, nthreads: int = 0, per_run: int = ITERS):
+    """The CPU oracle (as it stands) on the same job: the first `per_run` iterations of runs 0, 1,
+    ... of step 0, as many runs as fit ~budget_s. Returns (neighbors/s, iters/s, iterations,
+    runs, cores, seconds)."""
     import oracle
 
     c = pi.CONFIGS[CFG]
     inst = pi.config_instance(CFG)
     M = comb(inst.n, c["k"])
     ten = pi.default_tenure(inst.n, c["k"])
-    # whole runs of the job (run 0, 1, ... of step 0) until ~budget_s of CPU work
     iters, runs, t = 0, 0, time.perf_counter()
     while True:
         V0 = start_vectors(inst.n, 0, [runs])[0]
-        oracle.tabu_run(inst.A, inst.S, c["k"], V0, ITERS, ten, stop_on_zero=False, nthreads=nthreads)
-        iters += ITERS
+        oracle.tabu_run(inst.A, inst.S, c["k"], V0, per_run, ten, stop_on_zero=False, nthreads=nthreads)
+        iters += per_run
         runs += 1
         if time.perf_counter() - t >= budget_s or runs >= RUNS:
             break
     dt = time.perf_counter() - t
     cores = nthreads or oracle.max_threads()
-    return iters * M / dt, iters / dt, iters, cores, dt
+    return iters * M / dt, iters / dt, iters, runs, cores, dt
+
+
+def cpu_model() -> str:
+    try:
+        with open("/proc/cpuinfo") as fh:
+            for line in fh:
+                if line.startswith("model name"):
+                    return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+def relaunch_under_torchrun(args) -> int:
+    """--gpus N (N > 1) without a torchrun environment: start N ranks on this node ourselves."""
+    import torch
+
+    have = torch.cuda.device_count()
+    if have < args.gpus:
+        print(json.dumps({"error": f"bench.py --gpus {args.gpus} needs {args.gpus} visible GPUs, found {have}"}),
+              flush=True)
+        return 2
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+           "--master-addr=127.0.0.1", f"--master-port={29400 + os.getpid() % 1000}", os.path.abspath(__file__),
+           *sys.argv[1:]]
+    return subprocess.call(cmd)
 
 
 def run_reference(args, rank, world):
@@ -204,6 +249,90 @@ def run_reference(args, rank, world):
 
 
 # --------------------------------------------------------------------------------- GPU arm
+def timed(stream, fn):
+    """Device time (ms) of fn() on `stream` by CUDA events, synchronised on both sides."""
+    import torch
+
+    torch.cuda.synchronize()
+    a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    a.record(stream)
+    out = fn()
+    b.record(stream)
+    torch.cuda.synchronize()
+    return a.elapsed_time(b), out
+
+
+def max_over_ranks(vals, world, dev):
+    """Element-wise max of a list of floats over ranks (device timing: the slowest rank)."""
+    if world == 1:
+        return list(vals)
+    import torch
+    import torch.distributed as dist
+
+    t = torch.tensor(vals, dtype=torch.float64, device=dev)
+    dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    return [float(x) for x in t]
+
+
+def sum_over_ranks(vals, world, dev):
+    if world == 1:
+        return list(vals)
+    import torch
+    import torch.distributed as dist
+
+    t = torch.tensor(vals, dtype=torch.int64, device=dev)
+    dist.all_reduce(t, op=dist.ReduceOp.SUM)
+    return [int(x) for x in t]
+
+
+def roofline_of(nbr_per_s_kernel, sms):
+    """The search kernel against the MEASURED integer peaks. The per-neighbour
+    instruction counts come from the committed ncu capture of the same kernel and job; a capture
+    taken from other sources than the current ones is refused (it would be silently stale)."""
+    from paper_conf_ipps_luongmt10_b200 import _build
+
+    pk, src = peaks()
+    mhz = float(pk.get("sm_max_mhz", 1965.0))
+    if not os.path.exists(PROFILE):
+        raise SystemExit(f"bench.py: {PROFILE} missing (capture it with scripts/capture_bench_kernel.sh)")
+    with open(PROFILE) as fh:
+        prof = json.load(fh)
+    want = _build.source_hash()
+    if prof.get("source_sha") != want:
+        raise SystemExit(f"bench.py: the committed ncu capture {os.path.relpath(PROFILE, ROOT)} was taken from "
+                         f"sources {prof.get('source_sha')}, the current sources are {want}: re-capture it "
+                         "(scripts/capture_bench_kernel.sh) instead of reporting stale per-neighbour counts")
+    per = prof["per_neighbor"]
+    ipn, ppn = per["issued_instructions"], per["popc"]
+    if os.path.exists(INT_PEAKS):
+        with open(INT_PEAKS) as fh:
+            ip = json.load(fh)
+        issue_lanes = ip["peaks"]["mix_lop3_imad"]["lanes_per_clk_per_sm"]
+        popc_lanes = ip["peaks"]["popc"]["lanes_per_clk_per_sm"]
+        peak_src = (f"measured on B200 (profiles/int_peaks.json: LOP3/IMAD alternating {issue_lanes:.1f}, "
+                    f"POPC {popc_lanes:.1f} lanes/clk/SM) x {sms} SMs x {mhz:.0f} MHz ({src} sm_max_mhz)")
+    else:
+        issue_lanes, popc_lanes = 128.0, 16.0
+        peak_src = f"fallback 128 / 16 lanes/clk/SM (no profiles/int_peaks.json) x {sms} SMs x {mhz:.0f} MHz"
+    peak = sms * issue_lanes * mhz * 1e6 / 1e12
+    achieved = nbr_per_s_kernel * ipn / 1e12
+    xu_ceiling = sms * popc_lanes * mhz * 1e6 / ppn
+    m, k = pi.CONFIGS[CFG]["m"], pi.CONFIGS[CFG]["k"]
+    ops = m * (k + 4)
+    return {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tops/s", "frac": achieved / peak,
+            "traffic": prof.get("dram_bytes_per_launch"),
+            "kernel": "k_search<3> (persistent, batched searches)",
+            "achieved_is": "issued thread-instructions/s = live neighbours/s (CUDA events) x issued instructions "
+                           "per neighbour (ncu source page of the committed capture, same sources)",
+            "instructions_per_neighbor": ipn, "peak_source": peak_src, "capture_source_sha": want,
+            "binding_pipe": {"pipe": "xu (POPC)", "popc_per_neighbor": ppn,
+                             "peak_lanes_per_clk_per_sm": popc_lanes,
+                             "ceiling_neighbors_per_s": xu_ceiling, "frac": nbr_per_s_kernel / xu_ceiling},
+            "stalls_per_issue": prof.get("stalls_per_issue"),
+            "model": {"ops_per_neighbor": ops, "frac": nbr_per_s_kernel * ops / 1e12 / peak,
+                      "note": "SURVEY.md §8(d) m(k+4) model; the bit-sliced kernel needs fewer ops, so > 1 is possible"}}
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -216,19 +345,26 @@ def main():
     ap.add_argument("--no-single", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--no-ubqp", action="store_true")
+    ap.add_argument("--no-partitioned", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)
     args = ap.parse_args()
+    in_torchrun = "WORLD_SIZE" in os.environ
     rank, world, local = env_int("RANK", 0), env_int("WORLD_SIZE", 1), env_int("LOCAL_RANK", 0)
-    if args.impl == "reference":
+    if args.impl == "reference":  # the CPU oracle: rank 0 alone works, other ranks exit 0
         run_reference(args, rank, world)
         return
+    if args.gpus > 1 and not in_torchrun:
+        sys.exit(relaunch_under_torchrun(args))
+    if world != args.gpus:
+        print(json.dumps({"error": f"bench.py --gpus {args.gpus} launched with WORLD_SIZE={world}"}), flush=True)
+        sys.exit(2)
     args.warmup = max(args.warmup, 3)
 
     import torch
     import torch.distributed as dist
 
     import paper_conf_ipps_luongmt10_b200 as L
-    from paper_conf_ipps_luongmt10_b200.parallel import restart_shard
+    from paper_conf_ipps_luongmt10_b200 import parallel as par
 
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
@@ -240,7 +376,7 @@ def main():
     M = comb(inst.n, k)
     ten = pi.default_tenure(inst.n, k)
     iters = args.iters
-    mine = restart_shard(args.runs, rank, world)  # runs of this rank: r = rank, rank + world, ...
+    mine = par.restart_shard(args.runs, rank, world)  # runs of this rank: r = rank, rank + world, ...
     R = len(mine)
     ctx = L.lns_create(inst.A, inst.S, local)
     stream = torch.cuda.current_stream(dev)
@@ -249,11 +385,16 @@ def main():
     Vo = torch.empty((max(R, 1), inst.n), dtype=torch.int8, device=dev)
     flush = torch.empty(L2_FLUSH_BYTES // 4, dtype=torch.int32, device=dev)
 
+    def barrier():
+        if world > 1:
+            dist.barrier()
+
     def step(s):
         if R == 0:
             return []
         return L.lns_tabu_run_batch(ctx, k, R, iters, ten, 0, V0s[s], 0, Vo, stream)
 
+    # ---- headline: the C4 job, inputs resident in HBM
     for s in range(args.warmup):
         step(s)
     torch.cuda.synchronize()
@@ -263,8 +404,7 @@ def main():
     with ClockSampler(local) as clk:
         for i in range(args.steps):
             flush.fill_(i)  # evict L2 between timed steps
-            if world > 1:
-                dist.barrier()
+            barrier()
             torch.cuda.synchronize()
             ev0[i].record(stream)
             res = step(args.warmup + i)
@@ -274,15 +414,9 @@ def main():
             iters_done += sum(r["iters_done"] for r in res)
     clocks = clk.summary()
     step_ms = [a.elapsed_time(b) for a, b in zip(ev0, ev1)]
-    total_ms, kern_ms = sum(step_ms), sum(kernel_ms)
     my_iters = iters_done
-    if world > 1:
-        t = torch.tensor([total_ms, kern_ms], dtype=torch.float64, device=dev)
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        total_ms, kern_ms = float(t[0]), float(t[1])
-        n_it = torch.tensor([iters_done], dtype=torch.int64, device=dev)
-        dist.all_reduce(n_it, op=dist.ReduceOp.SUM)
-        iters_done = int(n_it[0])
+    total_ms, kern_ms = max_over_ranks([sum(step_ms), sum(kernel_ms)], world, dev)
+    (iters_done,) = sum_over_ranks([iters_done], world, dev)
     value = iters_done * M / (total_ms / 1e3)
 
     # ---- end to end through the C ABI with host buffers (pinned), same job
@@ -299,26 +433,20 @@ def main():
     e2e_ms, e2e_iters, e2e_steps = 0.0, 0, []
     for i in range(args.steps):
         flush.fill_(i)
-        if world > 1:
-            dist.barrier()
-        torch.cuda.synchronize()
-        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-        e0.record(stream)
-        c2 = L.lns_create(A_h, S_h, local)
-        r2 = L.lns_tabu_run_batch(c2, k, R, iters, ten, 0, V0_h[args.warmup + i], 0, Vo_h, stream) if R else []
-        L.lns_destroy(c2)
-        e1.record(stream)
-        torch.cuda.synchronize()
-        e2e_steps.append(e0.elapsed_time(e1))
-        e2e_ms += e2e_steps[-1]
+        barrier()
+
+        def e2e_step():
+            c2 = L.lns_create(A_h, S_h, local)
+            r2 = L.lns_tabu_run_batch(c2, k, R, iters, ten, 0, V0_h[args.warmup + i], 0, Vo_h, stream) if R else []
+            L.lns_destroy(c2)
+            return r2
+
+        ms, r2 = timed(stream, e2e_step)
+        e2e_steps.append(ms)
+        e2e_ms += ms
         e2e_iters += sum(r["iters_done"] for r in r2)
-    if world > 1:
-        t = torch.tensor([e2e_ms], dtype=torch.float64, device=dev)
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        e2e_ms = float(t[0])
-        n_it = torch.tensor([e2e_iters], dtype=torch.int64, device=dev)
-        dist.all_reduce(n_it, op=dist.ReduceOp.SUM)
-        e2e_iters = int(n_it[0])
+    (e2e_ms,) = max_over_ranks([e2e_ms], world, dev)
+    (e2e_iters,) = sum_over_ranks([e2e_iters], world, dev)
     e2e_value = e2e_iters * M / (e2e_ms / 1e3)
     if rank == 0:
         print(f"[bench] e2e ms per step: {[round(x, 2) for x in e2e_steps]}", file=sys.stderr)
@@ -336,13 +464,7 @@ def main():
         ms = []
         for _ in range(3):
             flush.fill_(0)
-            torch.cuda.synchronize()
-            a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-            a.record(stream)
-            L.lns_tabu_run(ctx, k, SINGLE_ITERS, ten, 0, v0, 0, v1, tr, tf, stream)
-            b.record(stream)
-            torch.cuda.synchronize()
-            ms.append(a.elapsed_time(b))
+            ms.append(timed(stream, lambda: L.lns_tabu_run(ctx, k, SINGLE_ITERS, ten, 0, v0, 0, v1, tr, tf, stream))[0])
         best = min(ms)
         single = {"neighbors_per_s": SINGLE_ITERS * M / (best / 1e3), "tabu_iters_per_s": SINGLE_ITERS / (best / 1e3),
                   "us_per_iteration": 1e3 * best / SINGLE_ITERS, "iters": SINGLE_ITERS,
@@ -350,10 +472,10 @@ def main():
 
     # ---- C5 (BASELINE configs[4], 1024 x 1024, 3-Hamming, 1.78e8 neighbours per iteration): one
     #      search on all SMs, a few iterations (N = 1 only; context beside the headline)
+    inst5 = pi.config_instance("C5")
+    M5 = comb(inst5.n, 3)
     c5 = None
     if world == 1 and not args.no_c5:
-        inst5 = pi.config_instance("C5")
-        M5 = L.lns_neighborhood_size(inst5.n, 3)
         with L.Instance(inst5.A, inst5.S) as I5:
             L.lns_tabu_run(I5.ctx, 3, 1, -1, pi.config_seed("C5"), None, 0)
             ms5 = []
@@ -367,16 +489,78 @@ def main():
               "ms_per_iteration": b5 / C5_ITERS, "iters": C5_ITERS,
               "note": "C5 single search from the config seed (packed plan for m > 255, DESIGN.md §5.11); device time of the launch"}
 
+    # ---- C5 restarts (BASELINE configs[4]: "64 independent restarts sharded across 8 x B200"):
+    #      8 restarts per GPU through lns_tabu_run_batch; with N > 1 the library shards restart r
+    #      to rank r mod N over the attached NCCL communicator and gathers every result
+    c5r = None
+    if not args.no_c5:
+        R5 = C5_RESTARTS_PER_GPU * world
+        with L.Instance(inst5.A, inst5.S, local) as I5:
+            comm = par.nccl_comm_ptr(device=dev) if world > 1 else None
+            if comm:
+                L.lns_attach_comm(I5.ctx, comm, rank, world)
+            L.lns_tabu_run_batch(I5.ctx, 3, R5, 1, -1, 1005, None, 0)  # warm-up (buffers)
+            barrier()
+            ms, r5 = timed(stream, lambda: L.lns_tabu_run_batch(I5.ctx, 3, R5, C5_RESTART_ITERS, -1, 1005, None, 0))
+            kms = L.lns_last_kernel_ms(I5.ctx)
+            if comm:
+                L.lns_attach_comm(I5.ctx, None, 0, 1)
+        ms, kms = max_over_ranks([ms, kms], world, dev)
+        done5 = sum(r["iters_done"] for r in r5)  # every rank holds every restart's result
+        c5r = {"restarts": R5, "restarts_per_gpu": C5_RESTARTS_PER_GPU, "iters_per_restart": C5_RESTART_ITERS,
+               "neighbors_per_s": done5 * M5 / (ms / 1e3), "tabu_iters_per_s": done5 / (ms / 1e3),
+               "kernel_neighbors_per_s": done5 * M5 / (kms / 1e3) if kms > 0 else None,
+               "note": "lns_tabu_run_batch, restart r on rank r mod N, results gathered by the library (NCCL)"}
+
+    # ---- one search partitioned over the N GPUs
+    part = None
+    if not args.no_partitioned:
+        part = {}
+        comm = par.nccl_comm_ptr(device=dev) if world > 1 else None
+        for name, inst_p, kp, itp in (("C4", inst, 3, PART_C4_ITERS), ("C5", inst5, 3, PART_C5_ITERS)):
+            Mp = comb(inst_p.n, kp)
+            with L.Instance(inst_p.A, inst_p.S, local) as Ip:
+                if comm:
+                    L.lns_attach_comm(Ip.ctx, comm, rank, world)
+                trp = torch.empty(itp, dtype=torch.int64, device=dev)
+                v0 = torch.from_numpy(pi.start_vector(inst_p.n, pi.config_seed(name))).to(dev)
+                L.lns_tabu_run(Ip.ctx, kp, min(itp, 70), -1, 0, v0, 0, None, trp, None, stream)  # warm-up
+                barrier()
+                ms, _ = timed(stream, lambda: L.lns_tabu_run(Ip.ctx, kp, itp, -1, 0, v0, 0, None, trp, None, stream))
+                trace_sha = __import__("hashlib").sha256(trp.cpu().numpy().tobytes()).hexdigest()[:16]
+                if comm:
+                    L.lns_attach_comm(Ip.ctx, None, 0, 1)
+            (ms,) = max_over_ranks([ms], world, dev)
+            part[name] = {"iters": itp, "us_per_iteration": 1e3 * ms / itp, "tabu_iters_per_s": itp / (ms / 1e3),
+                          "neighbors_per_s": itp * Mp / (ms / 1e3), "trace_sha16": trace_sha,
+                          "exchange": "ncclAllReduce u64 MIN per iteration (lns_attach_comm, CUDA-graph stepped loop)"
+                          if world > 1 else "none (N = 1: the persistent single-GPU search)"}
+        if world > 1:  # the device-initiated exchange: persistent kernels meet in peer memory
+            with L.Instance(inst.A, inst.S, local) as Ip:
+                trp = torch.empty(PART_C4_ITERS, dtype=torch.int64, device=dev)
+                v0 = torch.from_numpy(pi.start_vector(inst.n, pi.config_seed("C4"))).to(dev)
+                par.peer_tabu_run(Ip.ctx, 3, 70, -1, 0, v0, 0, trace_rank=trp, stream=stream)
+                barrier()
+                ms, _ = timed(stream, lambda: par.peer_tabu_run(Ip.ctx, 3, PART_C4_ITERS, -1, 0, v0, 0,
+                                                                trace_rank=trp, stream=stream))
+                trace_sha = __import__("hashlib").sha256(trp.cpu().numpy().tobytes()).hexdigest()[:16]
+            (ms,) = max_over_ranks([ms], world, dev)
+            part["C4_peer"] = {"iters": PART_C4_ITERS, "us_per_iteration": 1e3 * ms / PART_C4_ITERS,
+                               "tabu_iters_per_s": PART_C4_ITERS / (ms / 1e3),
+                               "neighbors_per_s": PART_C4_ITERS * M / (ms / 1e3), "trace_sha16": trace_sha,
+                               "exchange": "device-initiated: red.min.sys / red.release.sys into every GPU's "
+                                           "exchange buffer (CUDA IPC), no host step"}
+
     # ---- UBQP: k = 3, n = 500 OR-Library-style Q, one search (N = 1 only; context)
     ubqp = None
     if world == 1 and not args.no_ubqp:
         from ppp_inputs import bqp as bi
 
-        nq, kq, itq = 500, 3, 50
+        nq, kq, itq = 500, 3, 256  # >= 128 iterations: the CUDA-graph path (64-iteration blocks)
         Qb = bi.random_q(nq, 0.1, 1)
         xq = bi.start_x(nq, 2)
         cq = L.lns_bqp_create(Qb, 0)
-        L.lns_bqp_tabu_run(cq, kq, 64, -1, xq, trace=False)
+        L.lns_bqp_tabu_run(cq, kq, 128, -1, xq, trace=False)
         msq = []
         for _ in range(2):
             flush.fill_(0)
@@ -388,55 +572,25 @@ def main():
         Mq = L.lns_neighborhood_size(nq, kq)
         ubqp = {"neighbors_per_s": itq * Mq / (bq / 1e3), "us_per_iteration": 1e3 * bq / itq, "iters": itq,
                 "note": "UBQP f = x^T Q x, n = 500, density 0.1, 3-Hamming (2.07e7 neighbours/iteration), one "
-                        "search; device time (eval + apply launches replayed from a CUDA graph)"}
+                        "search; device time of the replay (eval + apply launches, CUDA graphs of 64 iterations)"}
 
     # ---- roofline: the search kernel (one launch per step)
-    pk, src = peaks()
-    mhz = float(pk.get("sm_max_mhz", 1965.0))
     sms = torch.cuda.get_device_properties(dev).multi_processor_count
-    ops_per_nbr = inst.m * (k + 4)  # SURVEY.md §8(d) model: k sign reads + Y' add + penalty + 2 histogram moves per row
     kern_avg_s = kern_ms / 1e3 / args.steps
-    achieved = (my_iters / args.steps) * M * ops_per_nbr / kern_avg_s / 1e12 if kern_avg_s > 0 else 0.0
-    peak = sms * 128 * mhz * 1e6 / 1e12  # 128 integer lanes issued per SM per clock (4 SMSP x 1 warp-instr)
-    traffic, per_nbr = None, None
-    prof = os.path.join(ROOT, "profiles", "r01_ncu_k_search_bench.json")  # ncu --set full of one bench step
-    if os.path.exists(prof):
-        try:
-            with open(prof) as fh:
-                pj = json.load(fh)
-            traffic, per_nbr = pj.get("dram_bytes_per_launch"), pj.get("per_neighbor")
-        except (OSError, ValueError):
-            traffic = None
     nbr_per_s_kernel = (my_iters / args.steps) * M / kern_avg_s if kern_avg_s > 0 else 0.0
-    # "the 'fraction of integer-pipe peak' uses achieved issued int instructions /
-    # peak, and the model figure is reported beside it, not instead of it" -- the bit-sliced kernel
-    # issues fewer instructions than the m(k+4) model counts, so the model figure can exceed 1
-    model = {"ops_per_neighbor": ops_per_nbr, "achieved": achieved, "frac": achieved / peak,
-             "note": "SURVEY.md §8(d) model: m(k+4) integer ops per neighbour (k sign reads, Y' add, "
-                     "penalty, 2 histogram moves per row); a bit-sliced kernel needs fewer, so frac > 1 is possible"}
-    roofline = {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "Tops/s", "frac": achieved / peak,
-                "traffic": traffic, "kernel": "k_search<3> (persistent, batched searches)",
-                "peak_source": f"{sms} SMs x 128 int lanes/clk x {mhz:.0f} MHz ({src} sm_max_mhz)",
-                "achieved_is": "model ops (no ncu capture found)", "model": model}
-    if per_nbr:
-        # what the kernel actually issues (ncu source page of the committed capture, same kernel and job)
-        ipn, ppn = per_nbr["issued_instructions"], per_nbr["popc"]
-        issued = nbr_per_s_kernel * ipn / 1e12
-        roofline.update({"achieved": issued, "frac": issued / peak,
-                         "achieved_is": "issued thread-instructions/s = live neighbours/s x issued instructions "
-                                        "per neighbour (ncu source page of the committed capture)",
-                         "instructions_per_neighbor": ipn})
-        # the pipe that binds the piece loop: POPC on XU at 1/8 of the issue rate (16 lanes/clk/SM)
-        xu_ceiling = sms * 16 * mhz * 1e6 / ppn
-        roofline["binding_pipe"] = {"pipe": "xu (POPC, 16 lanes/clk/SM)", "popc_per_neighbor": ppn,
-                                    "ceiling_neighbors_per_s": xu_ceiling, "frac": nbr_per_s_kernel / xu_ceiling}
+    roofline = roofline_of(nbr_per_s_kernel, sms)
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
-        v, ips, it, cores, dt = oracle_sample(args.cpu_budget)
-        cpu = {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle",
-               "sample": f"{it // ITERS} runs x {ITERS} tabu iterations of step 0 of the {CFG} job (same instance, tenure, start vectors), "
-                         f"{dt:.1f} s, from-scratch fitness per neighbour", "tabu_iters_per_s": ips}
+        v, ips, it, runs, cores, dt = oracle_sample(args.cpu_budget)
+        v1, ips1, it1, runs1, _, dt1 = oracle_sample(args.cpu_budget, nthreads=1, per_run=10)
+        cpu = {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle", "cpu_model": cpu_model(),
+               "sample": f"{runs} runs x {ITERS} tabu iterations of step 0 of the {CFG} job (same instance, tenure, "
+                         f"start vectors), {dt:.1f} s on {cores} OpenMP threads, from-scratch fitness per neighbour",
+               "tabu_iters_per_s": ips,
+               "single_thread": {"value": v1, "unit": UNIT, "cores": 1, "tabu_iters_per_s": ips1,
+                                 "sample": f"first 10 iterations of runs 0..{runs1 - 1} of step 0, {dt1:.1f} s, "
+                                           "one thread (the paper's sequential CPU baseline style, PAPER.md:245-248)"}}
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
@@ -454,7 +608,9 @@ def main():
             "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                     "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
             "single_search": single,
+            "partitioned": part,
             "c5_single_search": c5,
+            "c5_restarts": c5r,
             "ubqp_single_search": ubqp,
             # our kernels per timed step: k_init_slots + the persistent k_search
             "gpu_launches": args.steps * 2,

@@ -52,6 +52,7 @@ typedef int32_t lns_status;
 #define LNS_EPEER (-7)          /* device-side peer exchange: a partition did not arrive in time */
 
 #define LNS_IPC_HANDLE_BYTES 64 /* size of a cudaIpcMemHandle_t (lns_exchange_ipc_handle) */
+#define LNS_UNIQUE_ID_BYTES 128 /* size of an ncclUniqueId (lns_get_unique_id) */
 
 #define LNS_STOP_ON_ZERO 1      /* stop the search when f = 0 */
 #define LNS_FORCE_STEPPED 2     /* run one launch sequence per iteration instead of the persistent kernel */
@@ -134,11 +135,16 @@ lns_status lns_tabu_run(lns_ctx *ctx, int32_t k, int64_t iters, int64_t tenure, 
                         const int8_t *V0, int32_t flags, int8_t *V_out, int64_t *trace_rank,
                         int64_t *trace_fit, lns_result *res, void *stream);
 
-/* lns_tabu_run_batch -- R independent searches (restarts) of lns_tabu_run on this device.
+/* lns_tabu_run_batch -- R independent searches (restarts) of lns_tabu_run (the paper runs every
+ *   configuration 50 times).
  *   Restart r starts from V0 + r*n when V0 != NULL, else from the splitmix64 vector of
  *   seed_r = first splitmix64 output of a stream seeded with seed + r (reading R12).
- *   V_out: (host|device) R x n int8, nullable.  res: host, R entries.  Ignores partitions and
- *   communicators (restarts are sharded across GPUs by the caller).  Synchronous.
+ *   V_out: (host|device) R x n int8, nullable.  res: host, R entries.  Partitions set with
+ *   lns_set_partition are ignored (each restart runs whole on one device). With a communicator
+ *   attached (lns_attach_comm / lns_comm_init_rank, world G > 1) every rank must call this with
+ *   identical arguments: restart r runs on rank r mod G, and every rank receives all R results
+ *   and final vectors (gathered by NCCL sums of zero-padded arrays; no per-iteration
+ *   collective).  Synchronous.
  *   Errors: as lns_tabu_run. */
 lns_status lns_tabu_run_batch(lns_ctx *ctx, int32_t k, int32_t R, int64_t iters, int64_t tenure,
                               uint64_t seed, const int8_t *V0, int32_t flags, int8_t *V_out,
@@ -157,10 +163,29 @@ lns_status lns_unrank(int32_t n, int32_t k, const int64_t *ranks, int64_t count,
  *   B(nparts) = C(n,k). Errors: EINVAL. */
 lns_status lns_set_partition(lns_ctx *ctx, int32_t part, int32_t nparts);
 
-/* lns_attach_comm -- borrow an NCCL communicator (ncclComm_t of the libnccl already loaded in
- *   the process, e.g. torch's) for multi-GPU lns_tabu_run; sets the partition to (rank, world).
- *   The communicator is not freed by the library. comm = NULL detaches. Errors: ENCCL. */
+/* lns_attach_comm -- borrow an NCCL communicator (ncclComm_t) for multi-GPU lns_tabu_run /
+ *   lns_tabu_run_batch; sets the partition to (rank, world). The communicator
+ *   must come from the libnccl ALREADY LOADED in the process (e.g. torch's, via
+ *   ProcessGroupNCCL._comm_ptr()): ncclAllReduce is looked up in that copy only (dlopen
+ *   RTLD_NOLOAD of libnccl.so.2, else the global symbol scope), never in a freshly loaded one.
+ *   The communicator is borrowed (not freed). comm = NULL detaches (and destroys a communicator
+ *   made by lns_comm_init_rank).
+ *   Errors: EINVAL (rank/world), ENCCL (no libnccl loaded in the process). */
 lns_status lns_attach_comm(lns_ctx *ctx, void *nccl_comm, int32_t rank, int32_t world);
+
+/* NCCL bootstrap without torch (one process per GPU, plain C callers):
+ *   lns_get_unique_id  -- on ONE rank: write a fresh ncclUniqueId (LNS_UNIQUE_ID_BYTES bytes,
+ *                         host buffer) to id_out; the caller distributes it to every rank
+ *                         (MPI, a file, a socket...).
+ *   lns_comm_init_rank -- on EVERY rank (collective over `world` processes): create an NCCL
+ *                         communicator from that id on the context's device (ncclCommInitRank),
+ *                         owned by the context, and attach it as lns_attach_comm would (partition
+ *                         (rank, world)). Destroyed by lns_destroy or lns_attach_comm(NULL).
+ *   Both use the libnccl already loaded in the process, else load libnccl.so.2 (the same copy
+ *   then serves every call on that communicator).
+ *   Errors: EINVAL (null id, rank/world), ENCCL (libnccl not found, NCCL call failed). */
+lns_status lns_get_unique_id(uint8_t *id_out);
+lns_status lns_comm_init_rank(lns_ctx *ctx, const uint8_t *id, int32_t rank, int32_t world);
 
 /* Device-initiated multi-GPU exchange (the partition of P:448-454 with
  * the per-iteration argmin moved inside the persistent kernel, no host collective):

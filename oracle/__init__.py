@@ -48,7 +48,6 @@ def _load():
         sig = {
             "oracle_splitmix64_next": (u64, [ctypes.POINTER(u64)]),
             "oracle_start_vector": (None, [i32, u64, _i8p]),
-            "oracle_matvec": (None, [_i8p, i32, i32, _i8p, _i32p]),
             "oracle_fitness": (i64, [_i8p, i32, i32, _i32p, _i8p]),
             "oracle_fitness_packed": (i64, [_i8p, i32, i32, _i32p, _i8p]),
             "oracle_neighborhood_size": (i64, [i32, i32]),
@@ -93,15 +92,6 @@ def start_vector(n: int, seed: int) -> np.ndarray:
     V = np.empty(n, dtype=np.int8)
     _load().oracle_start_vector(n, seed, _p(V, _i8p))
     return V
-
-
-def matvec(A, V) -> np.ndarray:
-    A = np.ascontiguousarray(A, dtype=np.int8)
-    V = np.ascontiguousarray(V, dtype=np.int8)
-    m, n = A.shape
-    Y = np.empty(m, dtype=np.int32)
-    _load().oracle_matvec(_p(A, _i8p), m, n, _p(V, _i8p), _p(Y, _i32p))
-    return Y
 
 
 def fitness(A, S, V, packed: bool = False) -> int:

@@ -101,16 +101,6 @@ int64_t oracle_fitness(const int8_t *A, int32_t m, int32_t n, const int32_t *S, 
     return f;
 }
 
-/* A V' for every row, by the scalar definition. */
-void oracle_matvec(const int8_t *A, int32_t m, int32_t n, const int8_t *V, int32_t *Y)
-{
-    for (int32_t j = 0; j < m; j++) {
-        int32_t acc = 0;
-        for (int32_t i = 0; i < n; i++) acc += (int32_t)A[(size_t)j * n + i] * V[i];
-        Y[j] = acc;
-    }
-}
-
 /* ---------------------------------------------------------------------------------------
  * Packed representation for speed: a +-1 vector is stored as sign bits (bit = 1 <=> -1), 64 per
  * word. Textbook identity: for x, v in {+-1}^n, <x, v> = n - 2 * popcount(bits(x) xor bits(v)).

@@ -34,6 +34,7 @@ LNS_TABU_SOLUTIONS = 16
 LNS_PLAIN_LAUNCH = 8
 KEY_NONE = (1 << 63) - 1
 LNS_IPC_HANDLE_BYTES = 64
+LNS_UNIQUE_ID_BYTES = 128
 
 RESULT_FIELDS = ("iters_done", "final_f", "best_f", "best_iter", "first_zero_iter", "solved")
 
@@ -65,6 +66,8 @@ _SIGS = {
     "lns_unrank": (_i32, [_i32, _i32, _vp, _i64, _vp, _vp]),
     "lns_set_partition": (_i32, [_vp, _i32, _i32]),
     "lns_attach_comm": (_i32, [_vp, _vp, _i32, _i32]),
+    "lns_get_unique_id": (_i32, [_vp]),
+    "lns_comm_init_rank": (_i32, [_vp, _vp, _i32, _i32]),
     "lns_exchange_buffer": (_i32, [_vp, ctypes.POINTER(_vp)]),
     "lns_exchange_ipc_handle": (_i32, [_vp, _vp]),
     "lns_attach_peers": (_i32, [_vp, _i32, _i32, ctypes.POINTER(_vp), _i64]),
@@ -219,6 +222,21 @@ def lns_set_partition(ctx: int, part: int, nparts: int) -> None:
 
 def lns_attach_comm(ctx: int, comm_ptr: Optional[int], rank: int, world: int) -> None:
     _check(load().lns_attach_comm(ctx, comm_ptr, rank, world), "lns_attach_comm")
+
+
+def lns_get_unique_id() -> bytes:
+    """A fresh ncclUniqueId (LNS_UNIQUE_ID_BYTES) for lns_comm_init_rank (call on one rank)."""
+    buf = ctypes.create_string_buffer(LNS_UNIQUE_ID_BYTES)
+    _check(load().lns_get_unique_id(buf), "lns_get_unique_id")
+    return buf.raw
+
+
+def lns_comm_init_rank(ctx: int, uid: bytes, rank: int, world: int) -> None:
+    """Create (collectively over `world` processes) an NCCL communicator owned by ctx and attach it."""
+    if len(uid) != LNS_UNIQUE_ID_BYTES:
+        raise ValueError("uid must be LNS_UNIQUE_ID_BYTES long")
+    buf = ctypes.create_string_buffer(bytes(uid), LNS_UNIQUE_ID_BYTES)
+    _check(load().lns_comm_init_rank(ctx, buf, rank, world), "lns_comm_init_rank")
 
 
 def lns_exchange_buffer(ctx: int) -> int:

@@ -19,6 +19,20 @@ NVCC_FLAGS = [
 ]
 
 
+def source_hash() -> str:
+    """sha256 (16 hex) of everything that determines the kernels' SASS: the CUDA sources, the header
+    and the nvcc flags. A committed ncu capture records it; bench.py refuses a capture whose hash
+    differs from the current sources (its per-neighbour instruction counts would be stale)."""
+    import hashlib
+
+    h = hashlib.sha256()
+    for p in SRC + DEPS + HDR:
+        with open(p, "rb") as fh:
+            h.update(fh.read())
+    h.update(" ".join(NVCC_FLAGS).encode())
+    return h.hexdigest()[:16]
+
+
 def nvcc() -> str:
     for cand in (os.environ.get("NVCC"), "/usr/local/cuda/bin/nvcc", "nvcc"):
         if cand and (os.path.sep not in cand or os.path.exists(cand)):

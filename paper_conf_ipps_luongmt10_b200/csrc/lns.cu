@@ -86,7 +86,7 @@ struct DevInst {
 
 // fstate layout (int64): current f, iterations done, best f, best iter, first zero iter, done, error
 enum { FS_F = 0, FS_T, FS_BEST, FS_BESTIT, FS_ZERO, FS_DONE, FS_ERR, FS_N };
-// FS_ERR: 1 = bad V0, 2 = no admissible move, 3 = peer exchange timed out
+// FS_ERR: 1 = bad V0, 2 = no admissible move, 3 = peer exchange timed out, 4 = grid exchange timed out
 #define MAX_PEERS 16
 #define LNS_MAXPH 4
 
@@ -130,6 +130,7 @@ struct SearchArgs {
     int32_t npeers, part;
     int64_t nb_total;       // CTAs over all partitions (the arrival count per exchange)
     int64_t timeout_ns;     // a partition missing for this long ends the run (FS_ERR = 3)
+    int64_t grid_timeout_ns;  // a CTA of this grid missing at an exchange for this long ends the run (FS_ERR = 4)
     int32_t plain_launch;   // LNS_PLAIN_LAUNCH: cudaLaunchKernel instead of the cooperative launch
 };
 
@@ -311,6 +312,26 @@ __device__ __forceinline__ unsigned long long warp_min_k(unsigned long long v) {
         v = w < v ? w : v;
     }
     return v;
+}
+
+// Wait (one thread) until the monotonic counter *ctr reaches target (acquire, gpu scope). A
+// persistent grid is co-resident by construction (cooperative launch), so this always ends; a
+// plain launch (LNS_PLAIN_LAUNCH) on a busy device has no such guarantee, so the wait gives up
+// after timeout_ns of %globaltimer and returns false (the run then fails with LNS_EPEER instead
+// of hanging).
+__device__ __forceinline__ bool spin_until_ge(const unsigned long long *ctr, unsigned long long target,
+                                              long long timeout_ns)
+{
+    unsigned long long seen, t_start, t_now;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+    if (seen >= target) return true;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_start));
+    for (;;) {
+        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
+        if (seen >= target) return true;
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_now));
+        if ((long long)(t_now - t_start) > timeout_ns) return false;
+    }
 }
 
 // Value range of Y: every thread passes its partial (min, max); a __syncthreads, then warp 0 sets
@@ -1374,7 +1395,7 @@ __device__ const uint32_t *load_state(const SearchArgs &A, unsigned char *sm, co
 template <int K>
 __device__ void sol_tabu(const SearchArgs &A, const unsigned char *sm, const Smem &L, const uint32_t *vbs,
                          int gg, uint32_t *until, int64_t t, int bid, int nb, unsigned long long *bar,
-                         unsigned long long tb)
+                         unsigned long long tb, int *xto)
 {
     const int NW = A.I.NWn, n = A.I.n;
     const int64_t Lt = A.L;
@@ -1406,11 +1427,7 @@ __device__ void sol_tabu(const SearchArgs &A, const unsigned char *sm, const Sme
         if (threadIdx.x == 0) {
             __threadfence();
             asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(bar) : "memory");
-            const unsigned long long target = (unsigned long long)nb * tb;
-            unsigned long long seen;
-            do {
-                asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(bar) : "memory");
-            } while (seen < target);
+            if (!spin_until_ge(bar, (unsigned long long)nb * tb, A.grid_timeout_ns)) *xto = 2;
             __threadfence();
         }
     }
@@ -1547,7 +1564,10 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
             else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr, mv);
             // (the solution-list barrier is passed once per iteration, before the exchange: pass tg + 1)
-            if (A.sol_list) sol_tabu<K>(A, sm, L, vbs, gg, until, t, bid, nb, gslots + 24, tg + 1);
+            if (A.sol_list) {
+                sol_tabu<K>(A, sm, L, vbs, gg, until, t, bid, nb, gslots + 24, tg + 1, &s_xto);
+                if (s_xto) { failed = true; break; }
+            }
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
                                                   nullptr, tri, A.aspiration, (int)best_f)
@@ -1651,11 +1671,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                     // the release orders the MIN above before the arrival; the acquire below orders
                     // the slot read after every CTA's arrival (and hence its MIN)
                     asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
-                    const unsigned long long target = (unsigned long long)nb * tg;
-                    unsigned long long seen;
-                    do {
-                        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
-                    } while (seen < target);
+                    if (!spin_until_ge(ctr, (unsigned long long)nb * tg, A.grid_timeout_ns)) s_xto = 2;
                     unsigned long long gk;
                     asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
                     ps.gkey = gk;
@@ -1665,6 +1681,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                 }
                 __syncthreads();
                 key = ps.gkey;
+                if (s_xto) { failed = true; break; }
             }
             PH(5);
             if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
@@ -1691,7 +1708,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                     int64_t *o = A.res + (size_t)rs * FS_N;
                     o[FS_F] = f; o[FS_T] = t - 1; o[FS_BEST] = best_f; o[FS_BESTIT] = best_it;
                     o[FS_ZERO] = zero_it; o[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
-                    o[FS_ERR] = failed ? 2 : 0;
+                    o[FS_ERR] = failed ? (s_xto == 2 ? 4 : 2) : 0;
                 }
             }
         } else {
@@ -1703,7 +1720,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                 if (threadIdx.x == 0) {
                     A.fs[FS_F] = f; A.fs[FS_T] = t - 1; A.fs[FS_BEST] = best_f; A.fs[FS_BESTIT] = best_it;
                     A.fs[FS_ZERO] = zero_it; A.fs[FS_DONE] = (A.stop_on_zero && f == 0) ? 1 : 0;
-                    if (failed) A.fs[FS_ERR] = s_xto ? 3 : 2;
+                    if (failed) A.fs[FS_ERR] = s_xto == 2 ? 4 : s_xto ? 3 : 2;
                 }
             }
         }
@@ -1895,6 +1912,7 @@ struct GenArgs {
     // batched restarts (R > 0): G groups of nbg CTAs; until[] of M entries and 64 exchange slots
     // per group; restart r from V0s + r n, results into res + r FS_N and vouts + r NWn
     int32_t R, G, nbg;
+    int64_t grid_timeout_ns;  // give-up time of the in-kernel group exchange (then: no admissible move)
     const int8_t *V0s;
     int64_t *res;
     uint32_t *vouts;
@@ -2255,13 +2273,9 @@ __global__ void __launch_bounds__(NTG, KGEN_OCC) k_gen(GenArgs A)
                     if (key != (unsigned long long)KEY_NONE)
                         asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(slot), "l"(key) : "memory");
                     asm volatile("red.release.gpu.global.add.u64 [%0], 1;" ::"l"(ctr) : "memory");
-                    const unsigned long long target = (unsigned long long)nbg * tg;
-                    unsigned long long seen;
-                    do {
-                        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(seen) : "l"(ctr) : "memory");
-                    } while (seen < target);
                     unsigned long long gk;
-                    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
+                    if (!spin_until_ge(ctr, (unsigned long long)nbg * tg, A.grid_timeout_ns)) gk = KEY_NONE;
+                    else asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(gk) : "l"(slot) : "memory");
                     gs.gkey = gk;
                     if (bid == 0)
                         asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(slots + 16 * ((tg + 2) % 3)),
@@ -2350,11 +2364,14 @@ struct lns_ctx {
     int part = 0, nparts = 1;
     void *comm = nullptr;
     nccl_allreduce_fn nccl_allreduce = nullptr;
+    void *comm_owned = nullptr;       // created by lns_comm_init_rank (destroyed with the context)
+    void *nccl_lib = nullptr;         // dl handle the communicator's NCCL calls come from
     int blocks_override = 0;
     int no_pad = 0;  // LNS_NO_PAD=1 at create: plain (unpadded) row placement, for A/B measurement
     int no_pkw = 0;  // LNS_NO_PKW=1 at create: m > 255 always takes the segment plan (A/B measurement)
     int force_pkw = 0;  // LNS_FORCE_PKW=1 at create: m > 255 tries the packed plan for any slice size
     int no_graph = 0;   // LNS_NO_GRAPH=1 at create: the stepped loop launches directly (A/B measurement)
+    int64_t grid_timeout_ms = 60000;  // LNS_GRID_TIMEOUT_MS at create: give-up time of an in-kernel grid exchange
     cudaStream_t cap_stream = nullptr;  // private stream for capturing the stepped loop's graph
     // device-initiated exchange (lns_attach_peers)
     unsigned long long *d_xbuf = nullptr;            // own 64-word exchange buffer (its own allocation)
@@ -2381,6 +2398,7 @@ struct lns_ctx {
     uint32_t *d_X = nullptr; size_t X_cap = 0;                // global X fallback (per CTA)
     uint32_t *d_ring = nullptr; size_t ring_cap = 0;          // LNS_TABU_SOLUTIONS: visited solutions
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
+    cudaEvent_t ev2 = nullptr, ev3 = nullptr;  // stepped loop: graph build excluded from last_ms
     double last_ms = 0.0;
     // stepped search
     bool step_active = false;
@@ -2654,6 +2672,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
     A.peers = nullptr; A.npeers = 0; A.part = 0; A.nb_total = 0; A.timeout_ns = 0;
+    A.grid_timeout_ns = c->grid_timeout_ms * 1000000LL;
     A.plain_launch = (flags & LNS_PLAIN_LAUNCH) ? 1 : 0;
     return A;
 }
@@ -2692,6 +2711,7 @@ lns_status search_finish(lns_ctx *c, int8_t *V_out, int64_t *trace_rank, int64_t
     if (fs[FS_ERR] == 1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
     if (fs[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
     if (fs[FS_ERR] == 3) return fail(LNS_EPEER, "a partition did not reach the exchange in time");
+    if (fs[FS_ERR] == 4) return fail(LNS_EPEER, "a CTA of the grid did not reach the exchange in time (not co-resident?)");
     const int64_t done = fs[FS_T];
     if (trace_rank && done > 0) CK(cudaMemcpyAsync(trace_rank, c->d_tr, done * 8, cudaMemcpyDefault, st));
     if (trace_fit && done > 0) CK(cudaMemcpyAsync(trace_fit, c->d_tf, done * 8, cudaMemcpyDefault, st));
@@ -2922,6 +2942,7 @@ GenArgs gen_args(lns_ctx *c, int k, uint32_t M, int64_t iters, int64_t L, int fl
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until; A.slots = c->d_slots;
     A.trace_r = c->d_tr; A.trace_f = c->d_tf; A.fit_out = nullptr; A.best_out = nullptr;
     A.R = 0; A.G = 1; A.nbg = 1; A.V0s = nullptr; A.res = nullptr; A.vouts = nullptr;
+    A.grid_timeout_ns = c->grid_timeout_ms * 1000000LL;
     return A;
 }
 
@@ -2990,7 +3011,9 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     const int n = c->n, SMs = c->numSMs;
     std::vector<int8_t> hv((size_t)R * n);
     if (V0) {
-        CK(cudaMemcpy(hv.data(), V0, hv.size(), cudaMemcpyDefault));
+        // ordered after the caller's work on `stream` (a device V0 may still be being written there)
+        CK(cudaMemcpyAsync(hv.data(), V0, hv.size(), cudaMemcpyDefault, st));
+        CK(cudaStreamSynchronize(st));
         for (int8_t v : hv)
             if (v != 1 && v != -1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
     } else {
@@ -3032,6 +3055,7 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     if (cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
     for (int r = 0; r < R; r++) {
         const int64_t *o = hres.data() + (size_t)r * FS_N;
+        if (o[FS_ERR] == 4) return fail(LNS_EPEER, "a CTA of the grid did not reach the exchange in time");
         if (o[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
         res[r].iters_done = o[FS_T]; res[r].final_f = o[FS_F]; res[r].best_f = o[FS_BEST];
         res[r].best_iter = o[FS_BESTIT]; res[r].first_zero_iter = o[FS_ZERO];
@@ -3042,7 +3066,8 @@ lns_status gen_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
         for (int r = 0; r < R; r++)
             for (int i = 0; i < n; i++)
                 ho[(size_t)r * n + i] = ((hvo[(size_t)r * c->NWn + i / 32] >> (i % 32)) & 1) ? -1 : 1;
-        CK(cudaMemcpy(V_out, ho.data(), ho.size(), cudaMemcpyDefault));
+        CK(cudaMemcpyAsync(V_out, ho.data(), ho.size(), cudaMemcpyDefault, st));
+        CK(cudaStreamSynchronize(st));
     }
     return LNS_OK;
 }
@@ -3119,6 +3144,36 @@ lns_status gen_eval_all(lns_ctx *c, int32_t k, const int8_t *V, int32_t *fitness
     float ms = 0; cudaEventElapsedTime(&ms, c->ev0, c->ev1); c->last_ms = ms;
     if (fs[FS_ERR]) return fail(LNS_EINVAL, "V must be +-1");
     return LNS_OK;
+}
+
+// NCCL entry points (resolved at run time: the library does not link NCCL)
+struct NcclUid { uint8_t b[LNS_UNIQUE_ID_BYTES]; };  // ncclUniqueId, passed by value to ncclCommInitRank
+typedef int (*nccl_get_uid_fn)(NcclUid *);
+typedef int (*nccl_init_rank_fn)(void **, int, NcclUid, int);
+typedef int (*nccl_destroy_fn)(void *);
+
+// The libnccl to use: the copy already loaded in the process (by soname, or its symbols in the
+// global scope); with allow_load, else a fresh dlopen (only for communicators this library
+// creates itself, so every call on them goes to that same copy).
+void *nccl_handle(bool allow_load)
+{
+    void *h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD);
+    if (h) return h;
+    if (dlsym(RTLD_DEFAULT, "ncclAllReduce")) return RTLD_DEFAULT;
+    if (!allow_load) return nullptr;
+    h = dlopen("libnccl.so.2", RTLD_NOW);
+    if (!h) h = dlopen("libnccl.so", RTLD_NOW);
+    return h;
+}
+
+void drop_owned_comm(lns_ctx *c)
+{
+    if (c->comm_owned && c->nccl_lib) {
+        nccl_destroy_fn d = (nccl_destroy_fn)dlsym(c->nccl_lib, "ncclCommDestroy");
+        if (d) d(c->comm_owned);
+    }
+    if (c->comm_owned && c->comm == c->comm_owned) { c->comm = nullptr; c->part = 0; c->nparts = 1; }
+    c->comm_owned = nullptr;
 }
 
 lns_status resolve_tenure(int64_t M, int64_t tenure, int64_t &L)
@@ -3219,6 +3274,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     { const char *e = getenv("LNS_NO_PKW"); c->no_pkw = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_FORCE_PKW"); c->force_pkw = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_NO_GRAPH"); c->no_graph = (e && e[0] == '1') ? 1 : 0; }
+    { const char *e = getenv("LNS_GRID_TIMEOUT_MS"); if (e && atoll(e) > 0) c->grid_timeout_ms = atoll(e); }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
     auto cleanup = [&](lns_status s) { lns_destroy(c); return s; };
@@ -3235,7 +3291,8 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     if (cudaMemcpy(c->d_Arow, arow.data(), arow.size() * 4, cudaMemcpyHostToDevice) != cudaSuccess ||
         cudaMemcpy(c->d_H, H.data(), (n + 1) * 4, cudaMemcpyHostToDevice) != cudaSuccess ||
         cudaMemset(c->d_counter, 0, sizeof(unsigned)) != cudaSuccess ||
-        cudaEventCreate(&c->ev0) != cudaSuccess || cudaEventCreate(&c->ev1) != cudaSuccess)
+        cudaEventCreate(&c->ev0) != cudaSuccess || cudaEventCreate(&c->ev1) != cudaSuccess ||
+        cudaEventCreate(&c->ev2) != cudaSuccess || cudaEventCreate(&c->ev3) != cudaSuccess)
         return cleanup(fail(LNS_ECUDA, "upload"));
     *out = c;
     return LNS_OK;
@@ -3252,9 +3309,12 @@ void lns_destroy(lns_ctx *c)
                     (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X, (void *)c->d_ring})
         pool_free(p);
     for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
+    drop_owned_comm(c);
     cudaFree(c->d_xbuf); cudaFree(c->d_peers);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
+    if (c->ev2) cudaEventDestroy(c->ev2);
+    if (c->ev3) cudaEventDestroy(c->ev3);
     if (c->cap_stream) cudaStreamDestroy(c->cap_stream);
     delete c;
 }
@@ -3278,14 +3338,52 @@ lns_status lns_set_partition(lns_ctx *c, int32_t part, int32_t nparts)
 lns_status lns_attach_comm(lns_ctx *c, void *comm, int32_t rank, int32_t world)
 {
     if (!c) return fail(LNS_EINVAL, "null context");
-    if (!comm) { c->comm = nullptr; c->part = 0; c->nparts = 1; return LNS_OK; }
+    if (!comm) { drop_owned_comm(c); c->comm = nullptr; c->part = 0; c->nparts = 1; return LNS_OK; }
     if (world < 1 || rank < 0 || rank >= world) return fail(LNS_EINVAL, "bad rank/world");
-    void *h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD);
-    if (!h) h = dlopen("libnccl.so.2", RTLD_NOW);
-    void *sym = h ? dlsym(h, "ncclAllReduce") : dlsym(RTLD_DEFAULT, "ncclAllReduce");
-    if (!sym) return fail(LNS_ENCCL, "ncclAllReduce not found (load torch's libnccl first)");
+    // a BORROWED communicator belongs to the NCCL already in the process (e.g. torch's): its
+    // ncclAllReduce is looked up there and never in a freshly loaded copy, which could be another
+    // build than the one that created the communicator
+    void *h = nccl_handle(false);
+    void *sym = h ? dlsym(h, "ncclAllReduce") : nullptr;
+    if (!sym) return fail(LNS_ENCCL, "ncclAllReduce not found: no libnccl loaded in this process (load torch's, or use lns_comm_init_rank)");
+    drop_owned_comm(c);
     c->nccl_allreduce = (nccl_allreduce_fn)sym;
+    c->nccl_lib = h;
     c->comm = comm;
+    c->part = rank; c->nparts = world; c->npeers = 0;
+    return LNS_OK;
+}
+
+lns_status lns_get_unique_id(uint8_t *id_out)
+{
+    if (!id_out) return fail(LNS_EINVAL, "null argument");
+    void *h = nccl_handle(true);
+    nccl_get_uid_fn fn = h ? (nccl_get_uid_fn)dlsym(h, "ncclGetUniqueId") : nullptr;
+    if (!fn) return fail(LNS_ENCCL, "libnccl.so.2 not found");
+    NcclUid uid;
+    if (fn(&uid) != 0) return fail(LNS_ENCCL, "ncclGetUniqueId failed");
+    memcpy(id_out, uid.b, LNS_UNIQUE_ID_BYTES);
+    return LNS_OK;
+}
+
+lns_status lns_comm_init_rank(lns_ctx *c, const uint8_t *id, int32_t rank, int32_t world)
+{
+    if (!c || !id) return fail(LNS_EINVAL, "null argument");
+    if (world < 1 || rank < 0 || rank >= world) return fail(LNS_EINVAL, "bad rank/world");
+    void *h = nccl_handle(true);
+    nccl_init_rank_fn init = h ? (nccl_init_rank_fn)dlsym(h, "ncclCommInitRank") : nullptr;
+    void *ar = h ? dlsym(h, "ncclAllReduce") : nullptr;
+    if (!init || !ar || !dlsym(h, "ncclCommDestroy")) return fail(LNS_ENCCL, "libnccl.so.2 not found");
+    DeviceGuard dg(c->device);
+    NcclUid uid;
+    memcpy(uid.b, id, LNS_UNIQUE_ID_BYTES);
+    void *comm = nullptr;
+    if (init(&comm, world, uid, rank) != 0 || !comm) return fail(LNS_ENCCL, "ncclCommInitRank failed");
+    drop_owned_comm(c);
+    c->comm_owned = comm;
+    c->comm = comm;
+    c->nccl_allreduce = (nccl_allreduce_fn)ar;
+    c->nccl_lib = h;
     c->part = rank; c->nparts = world; c->npeers = 0;
     return LNS_OK;
 }
@@ -3513,6 +3611,7 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     if (sols && (s = grow(c->d_ring, c->ring_cap, (size_t)L * c->NWn)) != LNS_OK) return s;
     if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
     SearchArgs A = make_args(c, g, iters, L, flags);
+    bool stepped_timing = false;
     if (c->npeers > 0) {
         // device-initiated exchange: one persistent kernel per partition, meeting in the peers'
         // exchange buffers every iteration; every partition uses the same CTA count
@@ -3543,6 +3642,8 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         // and the graph is replayed on `st`; the remainder runs directly. LNS_NO_GRAPH=1 at create
         // keeps every launch direct.
         constexpr int64_t CH = 64;
+        // timed as [ev0, ev2] (the direct first iteration) + [ev3, ev1] (the rest): the host-side
+        // capture and instantiation in between leave the GPU idle and are not search time
         cudaGraphExec_t ge = nullptr;
         CK(cudaEventRecord(c->ev0, st));
         int64_t t = 0;
@@ -3550,6 +3651,7 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
             if ((s = one(st)) != LNS_OK) return s;
             t = 1;
         }
+        CK(cudaEventRecord(c->ev2, st));
         if (!c->no_graph && iters - t >= CH) {
             if (!c->cap_stream) CK(cudaStreamCreateWithFlags(&c->cap_stream, cudaStreamNonBlocking));
             cudaGraph_t gr = nullptr;
@@ -3563,6 +3665,8 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
             cudaGraphDestroy(gr);
             CK(ie);
         }
+        CK(cudaEventRecord(c->ev3, st));
+        stepped_timing = true;
         while (t < iters) {
             const int64_t t_prev = t;
             if (ge && iters - t >= CH) {
@@ -3584,8 +3688,14 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
         CK(cudaEventRecord(c->ev1, st));
     }
     s = search_finish(c, V_out, trace_rank, trace_fit, res, st);
-    float ms = 0;
-    if (iters > 0 && cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
+    float ms = 0, ms2 = 0;
+    if (iters > 0 && stepped_timing) {
+        if (cudaEventElapsedTime(&ms, c->ev0, c->ev2) == cudaSuccess &&
+            cudaEventElapsedTime(&ms2, c->ev3, c->ev1) == cudaSuccess)
+            c->last_ms = (double)ms + (double)ms2;
+    } else if (iters > 0 && cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) {
+        c->last_ms = ms;
+    }
     cudaGetLastError();
     return s;
 }
@@ -3611,7 +3721,9 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     const int n = c->n;
     std::vector<int8_t> hv((size_t)R * n);
     if (V0) {
-        CK(cudaMemcpy(hv.data(), V0, hv.size(), cudaMemcpyDefault));
+        // ordered after the caller's work on `stream` (a device V0 may still be being written there)
+        CK(cudaMemcpyAsync(hv.data(), V0, hv.size(), cudaMemcpyDefault, st));
+        CK(cudaStreamSynchronize(st));
         for (int8_t v : hv)
             if (v != 1 && v != -1) return fail(LNS_EINVAL, "V0 entries must be +1 or -1");
     } else {
@@ -3620,6 +3732,25 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
             vector_from_seed(n, splitmix64_next(sr), hv.data() + (size_t)r * n);
         }
     }
+    // With a communicator attached (lns_attach_comm / lns_comm_init_rank) the restarts are sharded:
+    // restart r runs on rank r mod world (the 50-run protocol of PAPER.md:250-253
+    // spread over GPUs), and the results are gathered on every rank by one NCCL sum of the
+    // zero-padded result arrays (each restart has exactly one owner). No per-iteration collective.
+    const int R_all = R;
+    const bool shard = c->comm && c->nparts > 1;
+    std::vector<int> mine;
+    for (int r = 0; r < R_all; r++)
+        if (!shard || r % c->nparts == c->part) mine.push_back(r);
+    if (shard) {
+        std::vector<int8_t> hl(mine.size() * (size_t)n);
+        for (size_t q = 0; q < mine.size(); q++)
+            memcpy(hl.data() + q * n, hv.data() + (size_t)mine[q] * n, n);
+        hv.swap(hl);
+        R = (int)mine.size();
+    }
+    std::vector<int64_t> hres((size_t)R * FS_N);
+    std::vector<uint32_t> hvo((size_t)R * c->NWn);
+    if (R > 0) {
     // Schedule: up to two phases, k1 rounds of G1 concurrent searches on
     // SMs / G1 CTAs each, then the R2 = R - k1 G1 remaining searches at once on SMs / R2 CTAs each,
     // minimising the makespan under the iteration-time model
@@ -3697,15 +3828,38 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     default: s = launch_batch<3>(c, A, g, grid, ngroups, nb_min, c->d_gslots, st); break;
     }
     if (s != LNS_OK) return s;
-    std::vector<int64_t> hres((size_t)R * FS_N);
-    std::vector<uint32_t> hvo((size_t)R * c->NWn);
     CK(cudaMemcpyAsync(hres.data(), c->d_res, hres.size() * 8, cudaMemcpyDeviceToHost, st));
     CK(cudaMemcpyAsync(hvo.data(), c->d_vouts, hvo.size() * 4, cudaMemcpyDeviceToHost, st));
     CK(cudaStreamSynchronize(st));
     float ms = 0;
     if (cudaEventElapsedTime(&ms, c->ev0, c->ev1) == cudaSuccess) c->last_ms = ms;
+    } else {
+        c->last_ms = 0.0;
+    }
+    if (shard) {  // gather: zero-padded full arrays, one owner per restart, NCCL sum
+        std::vector<int64_t> fres((size_t)R_all * FS_N, 0);
+        std::vector<uint32_t> fvo((size_t)R_all * c->NWn, 0u);
+        for (size_t q = 0; q < mine.size(); q++) {
+            memcpy(fres.data() + (size_t)mine[q] * FS_N, hres.data() + q * FS_N, 8 * FS_N);
+            memcpy(fvo.data() + (size_t)mine[q] * c->NWn, hvo.data() + q * c->NWn, 4 * (size_t)c->NWn);
+        }
+        if ((s = grow(c->d_res, c->res_cap, fres.size())) != LNS_OK) return s;
+        if ((s = grow(c->d_vouts, c->vouts_cap, fvo.size())) != LNS_OK) return s;
+        CK(cudaMemcpyAsync(c->d_res, fres.data(), fres.size() * 8, cudaMemcpyHostToDevice, st));
+        CK(cudaMemcpyAsync(c->d_vouts, fvo.data(), fvo.size() * 4, cudaMemcpyHostToDevice, st));
+        if (c->nccl_allreduce(c->d_res, c->d_res, fres.size(), /*ncclInt64*/ 4, /*ncclSum*/ 0, c->comm, st) != 0 ||
+            c->nccl_allreduce(c->d_vouts, c->d_vouts, fvo.size(), /*ncclUint32*/ 3, /*ncclSum*/ 0, c->comm, st) != 0)
+            return fail(LNS_ENCCL, "ncclAllReduce (restart gather) failed");
+        CK(cudaMemcpyAsync(fres.data(), c->d_res, fres.size() * 8, cudaMemcpyDeviceToHost, st));
+        CK(cudaMemcpyAsync(fvo.data(), c->d_vouts, fvo.size() * 4, cudaMemcpyDeviceToHost, st));
+        CK(cudaStreamSynchronize(st));
+        hres.swap(fres);
+        hvo.swap(fvo);
+        R = R_all;
+    }
     for (int r = 0; r < R; r++) {
         const int64_t *o = hres.data() + (size_t)r * FS_N;
+        if (o[FS_ERR] == 4) return fail(LNS_EPEER, "a CTA of the grid did not reach the exchange in time");
         if (o[FS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "no admissible move");
         res[r].iters_done = o[FS_T]; res[r].final_f = o[FS_F]; res[r].best_f = o[FS_BEST];
         res[r].best_iter = o[FS_BESTIT]; res[r].first_zero_iter = o[FS_ZERO];
@@ -3716,7 +3870,8 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
         for (int r = 0; r < R; r++)
             for (int i = 0; i < n; i++)
                 ho[(size_t)r * n + i] = ((hvo[(size_t)r * c->NWn + i / 32] >> (i % 32)) & 1) ? -1 : 1;
-        CK(cudaMemcpy(V_out, ho.data(), ho.size(), cudaMemcpyDefault));
+        CK(cudaMemcpyAsync(V_out, ho.data(), ho.size(), cudaMemcpyDefault, st));
+        CK(cudaStreamSynchronize(st));
     }
     return LNS_OK;
 }

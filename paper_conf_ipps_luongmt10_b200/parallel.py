@@ -121,6 +121,22 @@ class LnsStepper:
         return tr[:it], tf[:it], Vo, res
 
 
+def nccl_comm_ptr(group=None, device: Optional[torch.device] = None) -> int:
+    """The ncclComm_t of a torch NCCL process group (for lns_attach_comm): torch's own libnccl
+    created it, and lns_attach_comm looks ncclAllReduce up in that same loaded copy."""
+    device = device or torch.device("cuda", torch.cuda.current_device())
+    pg = group or dist.group.WORLD
+    backend = pg._get_backend(device)
+    # make sure the communicator exists (torch creates it lazily unless device_id was given)
+    t = torch.zeros(1, device=device)
+    dist.all_reduce(t, group=pg)
+    torch.cuda.synchronize(device)
+    ptr = int(backend._comm_ptr())
+    if not ptr:
+        raise RuntimeError("no NCCL communicator behind this process group")
+    return ptr
+
+
 def restart_shard(R: int, rank: int, world: int) -> list[int]:
     """Restarts owned by `rank`: r = rank, rank + world, ... (restart r on GPU r mod world)."""
     return list(range(rank, R, world))

@@ -41,6 +41,7 @@ def main():
     ap.add_argument("--capture", required=True)
     ap.add_argument("--source", help="`--page source --csv` export of the same capture (per-SASS counts)")
     ap.add_argument("--units", type=float, default=0.0, help="neighbour evaluations in the profiled launch")
+    ap.add_argument("--source-sha", default=None, help="_build.source_hash() of the profiled build")
     a = ap.parse_args()
     with open(a.raw) as fh:
         rows = list(csv.reader(fh))
@@ -48,14 +49,15 @@ def main():
     data = rows[2]  # the first (profiled) launch
     metrics = {}
     for name, unit, val in zip(hdr, units, data):
-        if name in KEEP or ("pipe_" in name and name.endswith(".avg.pct_of_peak_sustained_active")):
+        if name in KEEP or ("pipe_" in name and name.endswith(".avg.pct_of_peak_sustained_active")) or \
+                (name.startswith("smsp__average_warp_latency_issue_stalled_") and name.endswith(".ratio")):
             metrics[name] = [val, unit]
 
     def nbytes(key):
         v, u = metrics.get(key, ["0", "byte"])
         return float(v.replace(",", "")) * SCALE.get(u, 1)
 
-    out = {"kernel": a.kernel, "capture": a.capture,
+    out = {"kernel": a.kernel, "capture": a.capture, "source_sha": a.source_sha,
            "dram_bytes_per_launch": nbytes("dram__bytes_read.sum") + nbytes("dram__bytes_write.sum"),
            "metrics": metrics}
     if a.source and a.units:
@@ -63,6 +65,7 @@ def main():
         h = src[1]
         isrc, ie = h.index("Source"), h.index("Instructions Executed")
         tot = popc = 0
+        mix = {}
         for r in src[2:]:
             if len(r) <= ie:
                 continue
@@ -70,11 +73,18 @@ def main():
             tot += e
             op = r[isrc].split()
             op = op[1] if op and op[0].startswith("@") and len(op) > 1 else (op[0] if op else "")
+            op = op.split(".")[0]
+            mix[op] = mix.get(op, 0) + e
             if op == "POPC":
                 popc += e
         # warp-level counts x 32 lanes / neighbours = per-neighbour (per-lane) instruction counts
         out["per_neighbor"] = {"units": a.units, "issued_instructions": 32 * tot / a.units,
-                               "popc": 32 * popc / a.units}
+                               "popc": 32 * popc / a.units,
+                               "mix": {k: round(32 * v / a.units, 2) for k, v in
+                                       sorted(mix.items(), key=lambda kv: -kv[1])[:16]}}
+    stalls = {k.replace("smsp__average_warp_latency_issue_stalled_", "").replace(".ratio", ""): float(v[0].replace(",", ""))
+              for k, v in metrics.items() if k.startswith("smsp__average_warp_latency_issue_stalled_")}
+    out["stalls_per_issue"] = dict(sorted(stalls.items(), key=lambda kv: -kv[1]))
     with open(a.out, "w") as fh:
         json.dump(out, fh, indent=1)
     print(json.dumps(out, indent=1)[:3000])
