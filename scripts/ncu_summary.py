@@ -50,7 +50,7 @@ def main():
     metrics = {}
     for name, unit, val in zip(hdr, units, data):
         if name in KEEP or ("pipe_" in name and name.endswith(".avg.pct_of_peak_sustained_active")) or \
-                (name.startswith("smsp__average_warp_latency_issue_stalled_") and name.endswith(".ratio")):
+                (name.startswith("smsp__average_warps_issue_stalled_") and name.endswith("_per_issue_active.ratio")):
             metrics[name] = [val, unit]
 
     def nbytes(key):
@@ -82,8 +82,9 @@ def main():
                                "popc": 32 * popc / a.units,
                                "mix": {k: round(32 * v / a.units, 2) for k, v in
                                        sorted(mix.items(), key=lambda kv: -kv[1])[:16]}}
-    stalls = {k.replace("smsp__average_warp_latency_issue_stalled_", "").replace(".ratio", ""): float(v[0].replace(",", ""))
-              for k, v in metrics.items() if k.startswith("smsp__average_warp_latency_issue_stalled_")}
+    stalls = {k.replace("smsp__average_warps_issue_stalled_", "").replace("_per_issue_active.ratio", ""):
+              float(v[0].replace(",", "")) for k, v in metrics.items()
+              if k.startswith("smsp__average_warps_issue_stalled_") and k.endswith("_per_issue_active.ratio")}
     out["stalls_per_issue"] = dict(sorted(stalls.items(), key=lambda kv: -kv[1]))
     with open(a.out, "w") as fh:
         json.dump(out, fh, indent=1)
