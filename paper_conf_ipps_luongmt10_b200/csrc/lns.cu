@@ -121,6 +121,14 @@ struct SearchArgs {
     int32_t *Y;             // state: m
     int64_t *fs;            // FS_N
     uint32_t *until;        // M entries: rank r is tabu at iteration t iff until[r] >= t
+    // compact tabu state (bits_mode), used instead of a global until[] when the
+    // CTA's slice does not fit in shared memory and neither variant (aspiration, solution list) is
+    // on: bit r of tbits = rank r is in the FIFO of the last L accepted ranks; tring[(s-1) % L] = the
+    // rank accepted at iteration s (only when the run can outlast the tenure: ring_on)
+    uint32_t *tbits;        // per group: bit_words words
+    uint32_t *tring;        // per group: L words (ring_on)
+    int32_t bits_mode, ring_on;
+    uint32_t bit_words;     // words per group bitmap (ceil(M/32))
     int64_t *slots;         // 3 x MAX_SLOTS parity-tagged keys (persistent) / accumulator (stepped)
     unsigned *counter;      // stepped: last-CTA counter
     int64_t *trace_r, *trace_f;
@@ -1167,8 +1175,14 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                                          const PlanScalars &ps, const uint32_t *Xarg, uint32_t M, uint32_t blo, uint32_t bhi,
                                          const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
                                          const uint2 *tri = nullptr, int aspire = 0,
-                                         int best_f = 0)
+                                         int best_f = 0, const uint32_t *tbits = nullptr)
 {
+    // rank r tabu at iteration t: the until[] array (smem slice or global), or the bitmap
+    auto is_tabu = [&](uint32_t r) -> bool {
+        if (until) return until[r - ubase] >= t;
+        // plain (L1-coherent) load: the CTA's own thread 0 updates these words between iterations
+        return tbits && ((tbits[r >> 5] >> (r & 31)) & 1u);
+    };
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     // X from the shared window when it lives there, so the compiler emits LDS (not generic loads)
     const uint32_t *X = XG ? Xarg : (const uint32_t *)(sm + L.X);
@@ -1204,8 +1218,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             int fA, fB;
             if (ps.rneg > 0) eval_pk<K, 2, true, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
             else eval_pk<K, 2, false, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
-            const bool tA = until && until[rA - ubase] >= t;
-            const bool tB = until && until[rb - ubase] >= t;
+            const bool tA = is_tabu(rA);
+            const bool tB = is_tabu(rb);
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
             const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
             const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
@@ -1236,8 +1250,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             int fA, fB;
             if (ps.rneg > 0) eval_pk<K, 2, true, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
             else eval_pk<K, 2, false, XG>(ps, cabs, X, pk, pstart, bins, I.n, a0, b0, c0, a1, b1, c1, fA, fB);
-            const bool tA = until && until[rA - ubase] >= t;
-            const bool tB = until && until[rb - ubase] >= t;
+            const bool tA = is_tabu(rA);
+            const bool tB = is_tabu(rb);
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
             const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
             const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
@@ -1249,8 +1263,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     for (uint32_t r0 = blo + 32u * warp; r0 < bhi; r0 += NT) {
         const uint32_t r = r0 + lane;
         if (r < bhi) {
-            const bool is_tabu = until && until[r - ubase] >= t;
-            if (!is_tabu || WRITE_ALL || aspire) {
+            const bool tab = is_tabu(r);
+            if (!tab || WRITE_ALL || aspire) {
                 int a, b, c;
                 if (tri) {  // flip sets of this CTA's fixed slice, precomputed at launch
                     const uint2 q = tri[r - blo];
@@ -1269,7 +1283,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                 if (WRITE_ALL) fit_out[r] = f;
                 const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
                 // admissible: not tabu, or (aspiration) better than the best fitness so far
-                if ((!is_tabu || (aspire && f < best_f)) && key < best) best = key;
+                if ((!tab || (aspire && f < best_f)) && key < best) best = key;
             }
         }
     }
@@ -1518,13 +1532,16 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     unsigned long long *gslots = (unsigned long long *)A.slots + 64 * (size_t)gg;
     uint32_t blo, bhi;
     cta_slice(A.lo, A.hi, bid, nb, blo, bhi);
-    // the CTA's until[] slice: shared-memory copy when it fits, else the group's global array
-    uint32_t *until = A.until + (batch ? (size_t)gg * A.M : 0);
+    // the CTA's until[] slice: shared-memory copy when it fits, else the group's global array, or
+    // (bits_mode) the group's bitmap + ring of accepted ranks
+    uint32_t *until = A.bits_mode ? nullptr : A.until + (batch ? (size_t)gg * A.M : 0);
+    uint32_t *tb = A.bits_mode ? A.tbits + (size_t)gg * A.bit_words : nullptr;
+    uint32_t *tring = (A.bits_mode && A.ring_on) ? A.tring + (size_t)gg * (size_t)A.L : nullptr;
     uint32_t ubase = 0;
     if (A.until_smem) {
         uint32_t *us = (uint32_t *)(sm + L.a_end);
-        if (!batch)
-            for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) us[r - blo] = A.until[r];
+        if (!batch)  // a new search: nothing is tabu
+            for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) us[r - blo] = 0u;
         until = us;
         ubase = blo;
     }
@@ -1547,7 +1564,10 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         int64_t f, best_f, best_it, zero_it, t0;
         if (batch) {
             init_restart<K>(A, Ar, A.V0s + (size_t)rs * A.I.n, sm, L, ps);
-            for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) until[r - ubase] = 0u;
+            if (tb)  // this CTA's words of the bitmap (slices are 32-aligned: no word is shared)
+                for (uint32_t w = (blo >> 5) + threadIdx.x; w < ((bhi + 31) >> 5); w += NT) tb[w] = 0u;
+            else
+                for (uint32_t r = blo + threadIdx.x; r < bhi; r += NT) until[r - ubase] = 0u;
             __syncthreads();
             f = 30 * (int64_t)ps.fpen + ps.fhd;
             best_f = f; best_it = 0; zero_it = (f == 0) ? 0 : -1; t0 = 0;
@@ -1570,11 +1590,15 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             }
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                  nullptr, tri, A.aspiration, (int)best_f)
+                                                  nullptr, tri, A.aspiration, (int)best_f, tb)
                      : eval_range<K, false, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                   nullptr, tri, A.aspiration, (int)best_f);
+                                                   nullptr, tri, A.aspiration, (int)best_f, tb);
             mine = warp_min_k(mine);
             if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
+            // the rank leaving the FIFO after this iteration (accepted at t - L), read before this
+            // CTA's arrival at exchange t; the leader overwrites its ring slot only after exchange t
+            uint32_t evict = 0xffffffffu;
+            if (tring && threadIdx.x == 0 && t > A.L) evict = __ldcg(tring + (size_t)((t - 1) % A.L));
             __syncthreads();
             PH(4);
             unsigned long long key = ps.key;
@@ -1687,7 +1711,17 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
             const uint32_t r = (uint32_t)(key & 0xffffffffu);
             f = (int64_t)(key >> 32);
-            if (!A.sol_list && threadIdx.x == 0 && r >= blo && r < bhi) until[r - ubase] = (uint32_t)(t + A.L);
+            if (tb) {
+                // bits_mode: r_{t-L} leaves the tabu list, r_t enters it (owner CTA's thread 0: the
+                // only writer of its slice's words; its threads read them after the next barrier)
+                if (threadIdx.x == 0) {
+                    if (evict >= blo && evict < bhi) tb[evict >> 5] &= ~(1u << (evict & 31));
+                    if (A.L > 0 && r >= blo && r < bhi) tb[r >> 5] |= 1u << (r & 31);
+                    if (tring && bid == 0) __stcg(tring + (size_t)((t - 1) % A.L), r);
+                }
+            } else if (!A.sol_list && threadIdx.x == 0 && r >= blo && r < bhi) {
+                until[r - ubase] = (uint32_t)(t + A.L);
+            }
             if (leader) {
                 if (A.trace_r) A.trace_r[t - 1] = r;
                 if (A.trace_f) A.trace_f[t - 1] = f;
@@ -1712,8 +1746,6 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
                 }
             }
         } else {
-            if (A.until_smem)
-                for (uint32_t q = blo + threadIdx.x; q < bhi; q += NT) A.until[q] = until[q - ubase];
             if (bid == 0) {
                 for (int j = threadIdx.x; j < A.I.m; j += NT) A.Y[j] = Ys[j];
                 for (int w = threadIdx.x; w < A.I.NWn; w += NT) A.vb[w] = vbs[w];
@@ -2389,6 +2421,9 @@ struct lns_ctx {
     int32_t *d_Yin = nullptr;
     uint32_t *d_bits = nullptr; size_t bits_cap = 0;
     uint32_t *d_until = nullptr; size_t until_cap = 0;
+    uint32_t *d_tbits = nullptr; size_t tbits_cap = 0;        // bits_mode tabu bitmaps (per group)
+    uint32_t *d_tring = nullptr; size_t tring_cap = 0;        // bits_mode rings of accepted ranks
+    int no_bits = 0;    // LNS_NO_BITS=1 at create: global until[] instead of bitmap + ring (A/B)
     int64_t *d_tr = nullptr, *d_tf = nullptr; size_t trace_cap = 0, trace_cap_f = 0;
     int32_t *d_fit = nullptr; size_t fit_cap = 0;
     int8_t *d_V0s = nullptr; size_t v0s_cap = 0;       // batched restarts
@@ -2671,6 +2706,8 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.nph = 0;
     A.vb = c->d_vb; A.Y = c->d_Y; A.fs = c->d_fs; A.until = c->d_until;
     A.slots = c->d_slots; A.counter = c->d_counter; A.trace_r = c->d_tr; A.trace_f = c->d_tf;
+    A.tbits = c->d_tbits; A.tring = c->d_tring; A.bits_mode = 0; A.ring_on = 0;
+    A.bit_words = (uint32_t)(((uint64_t)g.M + 31) / 32);
     A.peers = nullptr; A.npeers = 0; A.part = 0; A.nb_total = 0; A.timeout_ns = 0;
     A.grid_timeout_ns = c->grid_timeout_ms * 1000000LL;
     A.plain_launch = (flags & LNS_PLAIN_LAUNCH) ? 1 : 0;
@@ -2678,7 +2715,8 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
 }
 
 // Prepare a search: V0 -> state, until[] cleared, trace buffers sized.
-lns_status search_setup(lns_ctx *c, const Geometry &g, int64_t iters, uint64_t seed, const int8_t *V0, cudaStream_t st)
+lns_status search_setup(lns_ctx *c, const Geometry &g, int64_t iters, uint64_t seed, const int8_t *V0, cudaStream_t st,
+                        bool need_until = true)
 {
     lns_status s;
     std::vector<int8_t> hv;
@@ -2688,8 +2726,10 @@ lns_status search_setup(lns_ctx *c, const Geometry &g, int64_t iters, uint64_t s
         vector_from_seed(c->n, seed, hv.data());
         CK(cudaMemcpyAsync(c->d_V, hv.data(), c->n, cudaMemcpyHostToDevice, st));
     }
-    if ((s = grow(c->d_until, c->until_cap, g.M)) != LNS_OK) return s;
-    CK(cudaMemsetAsync(c->d_until, 0, (size_t)g.M * 4, st));
+    if (need_until) {  // the global until[] (stepped path, variants); persistent searches keep their own state
+        if ((s = grow(c->d_until, c->until_cap, g.M)) != LNS_OK) return s;
+        CK(cudaMemsetAsync(c->d_until, 0, (size_t)g.M * 4, st));
+    }
     const size_t tc = (size_t)std::max<int64_t>(iters, 1);
     if ((s = grow(c->d_tr, c->trace_cap, tc)) != LNS_OK) return s;
     if ((s = grow(c->d_tf, c->trace_cap_f, tc)) != LNS_OK) return s;
@@ -2783,6 +2823,30 @@ inline int pad_for(const Geometry &g, uint32_t span, int nb)
     return (g.pad && span / (uint32_t)std::max(nb, 1) >= 4u * NT) ? 1 : 0;
 }
 
+// bits_mode: when the until[] slice of a CTA does not fit in shared memory and the
+// default tabu list is used (no aspiration, no solution list), keep one bit per rank plus a ring of
+// the last L accepted ranks instead of a u32 per rank: ceil(M/32) words per group (C5: 22 MB instead
+// of 713 MB), and the ring only when a search can outlast its tenure (L < iterations). groups
+// bitmaps and rings are allocated; zero_now clears the bitmaps on `st` (a single search: batched
+// restarts clear their words in the kernel).
+lns_status setup_bits(lns_ctx *c, SearchArgs &A, int groups, bool zero_now, cudaStream_t st)
+{
+    A.bits_mode = 0; A.ring_on = 0;
+    if (c->no_bits || A.until_smem || A.sol_list || A.aspiration) return LNS_OK;
+    lns_status s;
+    const size_t per = A.bit_words;
+    if ((s = grow(c->d_tbits, c->tbits_cap, per * (size_t)groups)) != LNS_OK) return s;
+    A.tbits = c->d_tbits;
+    if (zero_now) CK(cudaMemsetAsync(c->d_tbits, 0, per * groups * 4, st));
+    if (A.L > 0 && A.L < A.iters) {
+        if ((s = grow(c->d_tring, c->tring_cap, (size_t)A.L * groups)) != LNS_OK) return s;
+        A.tring = c->d_tring;
+        A.ring_on = 1;
+    }
+    A.bits_mode = 1;
+    return LNS_OK;
+}
+
 template <int K>
 lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st, int nb_force = 0)
 {
@@ -2798,6 +2862,9 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     A.I.pad = pad_for(g, A.hi - A.lo, nb);
     A.I.pkw = pkw_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
+    lns_status sb = setup_bits(c, A, 1, true, st);
+    if (sb != LNS_OK) return sb;
+    if (!A.until_smem && !A.bits_mode && !c->d_until) return fail(LNS_EINVAL, "internal: no tabu state allocated");
     // exchange slots (3 keys on separate lines) = KEY_NONE, arrival counter = 0
     k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
     void *args[] = {&A};
@@ -2818,7 +2885,9 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int grid, i
     A.I.pad = pad_for(g, A.hi - A.lo, nb_min);
     A.I.pkw = pkw_for(g, A.hi - A.lo, nb_min);
     const size_t smem = cache_geometry(A, g, nb_min, budget);
-    if (!A.until_smem) {  // one global until[] per group of every phase
+    lns_status sb = setup_bits(c, A, ngroups, false, st);  // each restart clears its words in the kernel
+    if (sb != LNS_OK) return sb;
+    if (!A.until_smem && !A.bits_mode) {  // one global until[] per group of every phase
         lns_status s = grow(c->d_until, c->until_cap, (size_t)ngroups * g.M);
         if (s != LNS_OK) return s;
         A.until = c->d_until;
@@ -3274,6 +3343,7 @@ lns_status lns_create(const int8_t *A, int32_t m, int32_t n, const int32_t *S, i
     { const char *e = getenv("LNS_NO_PKW"); c->no_pkw = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_FORCE_PKW"); c->force_pkw = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_NO_GRAPH"); c->no_graph = (e && e[0] == '1') ? 1 : 0; }
+    { const char *e = getenv("LNS_NO_BITS"); c->no_bits = (e && e[0] == '1') ? 1 : 0; }
     { const char *e = getenv("LNS_GRID_TIMEOUT_MS"); if (e && atoll(e) > 0) c->grid_timeout_ms = atoll(e); }
     for (int b = 0; b <= n; b++)
         if (H[b] > 0) c->maxS = b;
@@ -3306,7 +3376,8 @@ void lns_destroy(lns_ctx *c)
     for (void *p : {(void *)c->d_Arow, (void *)c->d_H, (void *)c->d_vb, (void *)c->d_Y, (void *)c->d_fs,
                     (void *)c->d_slots, (void *)c->d_counter, (void *)c->d_V, (void *)c->d_Yin, (void *)c->d_bits,
                     (void *)c->d_until, (void *)c->d_tr, (void *)c->d_tf, (void *)c->d_fit, (void *)c->d_V0s,
-                    (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X, (void *)c->d_ring})
+                    (void *)c->d_res, (void *)c->d_vouts, (void *)c->d_gslots, (void *)c->d_X, (void *)c->d_ring,
+                    (void *)c->d_tbits, (void *)c->d_tring})
         pool_free(p);
     for (void *p : c->ipc_opened) cudaIpcCloseMemHandle(p);
     drop_owned_comm(c);
@@ -3609,7 +3680,9 @@ lns_status lns_tabu_run(lns_ctx *c, int32_t k, int64_t iters, int64_t tenure, ui
     DeviceGuard dg(c->device);
     cudaStream_t st = (cudaStream_t)stream;
     if (sols && (s = grow(c->d_ring, c->ring_cap, (size_t)L * c->NWn)) != LNS_OK) return s;
-    if ((s = search_setup(c, g, iters, seed, V0, st)) != LNS_OK) return s;
+    const bool persistent = c->npeers > 0 || !(c->comm != nullptr || c->nparts > 1 || (flags & LNS_FORCE_STEPPED));
+    const bool need_until = !persistent || sols || (flags & LNS_ASPIRATION) || c->no_bits;
+    if ((s = search_setup(c, g, iters, seed, V0, st, need_until)) != LNS_OK) return s;
     SearchArgs A = make_args(c, g, iters, L, flags);
     bool stepped_timing = false;
     if (c->npeers > 0) {
@@ -3763,8 +3836,11 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     const double fixed = 2.0 + 7.5e-4 * (double)c->m * (double)c->n;
     auto T = [&](int nbq) { return fixed + work / nbq; };
     const int budget = c->smemOptin - 1024;
-    // a global until[] per group (unless the slice fits in shared memory), capped at 8 GiB in total
-    const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / (4LL * g.M));
+    // a global tabu state per group (unless the slice fits in shared memory), capped at 8 GiB in
+    // total: a bitmap (+ ring) in bits_mode, else a u32 until[] per rank
+    const bool bits = !c->no_bits && !sols && !(flags & LNS_ASPIRATION);
+    const int64_t per_group = bits ? 4 * (((int64_t)g.M + 31) / 32) + (L > 0 && L < iters ? 4 * L : 0) : 4LL * g.M;
+    const int64_t cap_groups = std::max<int64_t>(1, (8LL << 30) / std::max<int64_t>(per_group, 1));
     // LNS_TABU_SOLUTIONS: a global until[] and a visited ring per group, 8 GiB in total at most
     const int64_t cap_sol = std::max<int64_t>(1, (8LL << 30) / (4LL * ((int64_t)g.M + L * c->NWn)));
     auto fits = [&](int groups, int nb_min) {
@@ -3808,7 +3884,6 @@ lns_status lns_tabu_run_batch(lns_ctx *c, int32_t k, int32_t R, int64_t iters, i
     if ((s = grow(c->d_vouts, c->vouts_cap, (size_t)R * c->NWn)) != LNS_OK) return s;
     if ((s = grow(c->d_gslots, c->gslots_cap, (size_t)ngroups * 64)) != LNS_OK) return s;
     if (sols && (s = grow(c->d_ring, c->ring_cap, (size_t)ngroups * L * c->NWn)) != LNS_OK) return s;
-    if ((s = grow(c->d_until, c->until_cap, std::max<size_t>(g.M, 1))) != LNS_OK) return s;
     CK(cudaMemcpyAsync(c->d_V0s, hv.data(), hv.size(), cudaMemcpyHostToDevice, st));
     const int savep = c->part, saven = c->nparts;
     c->part = 0; c->nparts = 1;

@@ -32,9 +32,9 @@ for s in range(INST):
 lines = ["# UBQP quality vs k (round 1)", "",
          f"`scripts/quality_bqp.py`: {INST} instances `random_q({N}, {DENS}, 1000 + s)`, {STARTS} starts each "
          f"(`start_x(n, 50 s + q)`), {ITERS} iterations for every k, tenure floor(C(n,k)/6). One B200; device "
-         "time per run. Best fitness per run (lower is better); `best-known` = the least over all 15 runs "
+         "time per run. Best fitness per run (lower is better); `best found in this experiment` = the least over all 15 runs "
          "of the instance.", "",
-         "| instance | best-known | k=1 mean / min | k=2 mean / min | k=3 mean / min | ms per run k=1 / 2 / 3 |",
+         "| instance | best found in this experiment | k=1 mean / min | k=2 mean / min | k=3 mean / min | ms per run k=1 / 2 / 3 |",
          "|---|---|---|---|---|---|"]
 hits = {1: 0, 2: 0, 3: 0}
 for s in range(INST):
@@ -44,7 +44,7 @@ for s in range(INST):
         hits[k] += sum(b == bk for b in best_of[(s, k)])
     lines.append(f"| {s} | {bk} | " + " | ".join(f"{r[k][2]:.1f} / {r[k][3]}" for k in (1, 2, 3)) +
                  " | " + " / ".join(f"{r[k][4]:.1f}" for k in (1, 2, 3)) + " |")
-lines += ["", "Runs reaching the best-known value (of " + str(INST * STARTS) + "): " +
+lines += ["", "Runs reaching the best value found in this experiment (of " + str(INST * STARTS) + "): " +
           ", ".join(f"k={k}: {hits[k]}" for k in (1, 2, 3)), ""]
 os.makedirs("results", exist_ok=True)
 open("results/quality_bqp_r01.md", "w").write("\n".join(lines))
