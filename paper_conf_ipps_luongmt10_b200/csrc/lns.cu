@@ -610,10 +610,29 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
         rowAt[p] = j;
     }
-    __syncthreads();  // rows placed: step D (X, warps 1..) overlaps the rest of C (warp 0)
+    __syncthreads();  // rows placed: step D (X, warps 2..) overlaps the rest of C (warps 0, 1)
     PH(2);
-    if (warp != 0) {
-        plan_transpose_warps(I, Ar, sm, L, ps, X, 1, NWARP - 1);
+    if (warp >= 2) {
+        plan_transpose_warps(I, Ar, sm, L, ps, X, 2, NWARP - 2);
+    } else if (warp == 1) {
+        // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form); bin constants; H of the walked
+        // bins (sums by warp reductions, no shared atomics)
+        unsigned dneg = 0;
+        for (int v = lane; v < uneg; v += 32)
+            dneg += (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v)));
+        const int z0 = ps.pkz[0], z1 = ps.pkz[1];
+        int hw = 0;
+        for (int beta = lane; beta < NB; beta += 32) {
+            const int b = vmin + 2 * (beta - K);
+            const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
+            bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
+            // walked bins: [first point, last point + 2K] of the walk of beta's parity
+            const int zp = ((beta - uneg) & 1) ? z1 : z0;
+            if (Hb && beta >= uneg && zp >= 0 && beta <= zp + 2 * K) hw += Hb;
+        }
+        dneg = __reduce_add_sync(FULL, dneg);
+        hw = __reduce_add_sync(FULL, hw);
+        if (lane == 0) { ps.cneg = (int)dneg; ps.hwalk = hw; }
     } else {
         for (int v = uneg + lane; v < utop; v += 32) {
             const int st = seg[v], Lv = cnt[uf + v], en = st + Lv;
@@ -648,20 +667,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
                 atomicMin((unsigned *)&pstart[w], pk0 + 16u * p);
             }
         }
-        for (int v = lane; v < uneg; v += 32)  // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form)
-            if (cnt[uf + v] > 0)
-                atomicAdd((unsigned *)&ps.cneg, (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v))));
-        const int z0 = ps.pkz[0], z1 = ps.pkz[1];
-        for (int beta = lane; beta < NB; beta += 32) {
-            const int b = vmin + 2 * (beta - K);
-            const int Hb = (b >= 0 && b <= n) ? Hs[b] : 0;
-            bins[beta] = make_int2(Hb, b < 0 ? 60 * (-b) - 1 : 0);
-            // walked bins: [first point, last point + 2K] of the walk of beta's parity
-            const int zp = ((beta - uneg) & 1) ? z1 : z0;
-            if (Hb && beta >= uneg && zp >= 0 && beta <= zp + 2 * K) atomicAdd(&ps.hwalk, Hb);
-        }
-        __syncwarp();  // the last readers of cnt[] and the writers of pkw0 are in this warp
-        for (int u = lane; u < Uc; u += 32) cnt[u] = 0;  // zero for the next plan
+        __syncwarp();  // the writers of pkw0 are in this warp
         if (lane < 2) {  // the walks' ready-to-use addresses and constants (read by pk_walk)
             const int q = tid, wd = ps.pkw0[q];
             const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
@@ -671,7 +677,8 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
             ps.pkwt[q] = make_uint4(ps.pkwin[q], ps.pkhtr[q], (uint32_t)ps.pktrl[q], (uint32_t)ps.pkz[q]);
         }
     }
-    __syncthreads();  // X (warps 1..), records, bins, pkwk / pkwt are published
+    __syncthreads();  // X (warps 2..), records, bins, pkwk / pkwt are published
+    for (int u = tid; u < Uc; u += NT) cnt[u] = 0;  // zero for the next plan (its first barrier orders it)
     PH(3);
 }
 
@@ -1042,12 +1049,15 @@ __device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int
     }
 }
 
+#ifndef PK_TWO_PLANES
+#define PK_TWO_PLANES 1  // c3 = |lo & hi & mask| by one three-input LOP3 (no lh register per neighbour)
+#endif
 template <int K>
 __device__ __forceinline__ void pk_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &w, int &f)
 {
     w += 255u * (uint32_t)__popc(lo & r.x);
     if (K >= 2) w += 65535u * (uint32_t)__popc(hi & r.x);
-    if (K == 3) w += 16711425u * (uint32_t)__popc(lh & r.x);
+    if (K == 3) w += 16711425u * (uint32_t)__popc((PK_TWO_PLANES ? lo & hi : lh) & r.x);
     // hb: byte 1 = h (byte 0 of w) for a final piece (selector 0x4404), 0 otherwise (0x4444)
     uint32_t hb, fu = (uint32_t)f;
     asm("prmt.b32 %0, %1, %2, %3;" : "=r"(hb) : "r"(w), "r"(0u), "r"(r.w));
@@ -1099,7 +1109,7 @@ __device__ __forceinline__ void pk_planes(const uint32_t *__restrict__ xg, uint3
     } else {
         lo = xa ^ xb ^ xc;
         hi = (xa & xb) | (xc & (xa ^ xb));
-        lh = lo & hi;
+        lh = PK_TWO_PLANES ? 0u : lo & hi;
     }
 }
 

@@ -1,0 +1,10 @@
+# round-2 call H: two planes + plan step C split + warp-0 counting + 16-byte exchange poll, vs head2p
+timeout 1200 python -m pytest tests -m gpu -x -q > gpurun_out/pytest_gpu_h.log 2>&1; echo pytest=$?
+tail -3 gpurun_out/pytest_gpu_h.log
+for v in head2p cur; do
+  lib=build/variants/liblns_$v.so; [ $v = cur ] && lib=paper_conf_ipps_luongmt10_b200/liblns.so
+  echo "== $v"
+  LNS_LIB=$lib timeout 300 python scripts/probe_batch.py C4:50:400 C4:50:400 C3:50:400 C2:148:2000 2>&1 | tail -4
+  LNS_LIB=$lib timeout 300 python scripts/probe_single.py 2>&1 | tail -4
+done
+echo "== phases cur"; timeout 300 python scripts/phases.py C4:148:1000 C3:148:1000 2>&1 | tail -20
