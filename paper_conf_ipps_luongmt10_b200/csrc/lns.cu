@@ -55,7 +55,7 @@ thread_local std::string g_err;
 
 // Optional per-phase cycle accounting (compile with -DLNS_PHASE_TIMING; tools/profiling only).
 #ifdef LNS_PHASE_TIMING
-constexpr int NPH = 8;
+constexpr int NPH = 12;
 __shared__ long long s_ph[NPH];
 __shared__ long long s_last;
 __device__ unsigned long long g_ph[NPH];
@@ -140,6 +140,7 @@ struct SearchArgs {
     int64_t timeout_ns;     // a partition missing for this long ends the run (FS_ERR = 3)
     int64_t grid_timeout_ns;  // a CTA of this grid missing at an exchange for this long ends the run (FS_ERR = 4)
     int32_t plain_launch;   // LNS_PLAIN_LAUNCH: cudaLaunchKernel instead of the cooperative launch
+    int32_t enc_keys;       // keys carry the flip set (enc_flip) instead of the rank: no unranking after the exchange
 };
 
 // The CTA's X (sorted sign bits): shared memory, or its own slot of the global fallback buffer.
@@ -214,10 +215,8 @@ struct PlanScalars {
     int rtop;  // rows below the top cut (points < utop), unpadded
     int vlo, Uc;  // conservative lattice of the NEXT plan: every Y lies in vlo + 2 [0, Uc)
     // packed path, parity walks (build_plan_pk): records of walk 0 are [0, pkb1),
-    // of walk 1 [pkb1, P); first row word, initial byte window, last point, trailing H bytes and
-    // "a trailing bin is negative" of each walk
-    int pkb1, pkw0[2], pkz[2], pktrl[2];
-    uint32_t pkwin[2], pkhtr[2];
+    // of walk 1 [pkb1, P); first row word of each walk
+    int pkb1, pkw0[2];
     unsigned long long key, gkey;
     int red[2 * NWARP + 2];
 };
@@ -297,6 +296,36 @@ __device__ __forceinline__ void succ_flip(int n, int &a, int &b, int &c)
     }
 }
 
+// The low word of a selection key: the rank r, or (enc_keys) the flip set itself packed so that
+// its order is the lexicographic order of (a, b, c), i.e. the rank order (reading R6): a << 20 |
+// b << 10 | c for k = 3 (n <= 1024), a << 16 | b for k = 2 (n <= 65536). The u64 MIN of
+// (f << 32 | low) then picks the same neighbour, and the winner's flip set needs no unranking.
+template <int K>
+__device__ __forceinline__ uint32_t enc_flip(int a, int b, int c)
+{
+    if (K == 3) return ((uint32_t)a << 20) | ((uint32_t)b << 10) | (uint32_t)c;
+    if (K == 2) return ((uint32_t)a << 16) | (uint32_t)b;
+    return (uint32_t)a;
+}
+
+template <int K>
+__device__ __forceinline__ void dec_flip(uint32_t e, int &a, int &b, int &c)
+{
+    if (K == 3) { a = (int)(e >> 20); b = (int)((e >> 10) & 1023u); c = (int)(e & 1023u); }
+    else if (K == 2) { a = (int)(e >> 16); b = (int)(e & 0xffffu); c = -1; }
+    else { a = (int)e; b = -1; c = -1; }
+}
+
+// lex_rank(a < b < c) = M - 1 - [C(n-1-a, 3) + C(n-1-b, 2) + (n-1-c)] from the shared tables
+template <int K>
+__device__ __forceinline__ uint32_t rank_tab(int n, uint32_t M, const uint32_t *T2, const uint32_t *T3, int a, int b,
+                                             int c)
+{
+    if (K == 3) return M - 1u - (T3[n - 1 - a] + T2[n - 1 - b] + (uint32_t)(n - 1 - c));
+    if (K == 2) return M - 1u - (T2[n - 1 - a] + (uint32_t)(n - 1 - b));
+    return (uint32_t)a;
+}
+
 __device__ __forceinline__ void fill_tables(uint32_t *T2, uint32_t *T3, int n)
 {
     for (int i = threadIdx.x; i < n; i += blockDim.x) {
@@ -314,12 +343,13 @@ __device__ __forceinline__ int warp_max_i(int v) {
     for (int o = 16; o; o >>= 1) v = max(v, __shfl_xor_sync(FULL, v, o));
     return v;
 }
+// u64 warp minimum with two 32-bit warp reductions (REDUX): the least high word, then the least
+// low word among the lanes holding it -- the same as the 64-bit minimum of (hi << 32 | lo)
 __device__ __forceinline__ unsigned long long warp_min_k(unsigned long long v) {
-    for (int o = 16; o; o >>= 1) {
-        unsigned long long w = __shfl_xor_sync(FULL, v, o);
-        v = w < v ? w : v;
-    }
-    return v;
+    const uint32_t hi = (uint32_t)(v >> 32), lo = (uint32_t)v;
+    const uint32_t mh = __reduce_min_sync(FULL, hi);
+    const uint32_t ml = __reduce_min_sync(FULL, hi == mh ? lo : 0xffffffffu);
+    return ((unsigned long long)mh << 32) | ml;
 }
 
 // Wait (one thread) until the monotonic counter *ctr reaches target (acquire, gpu scope). A
@@ -456,7 +486,7 @@ __device__ __forceinline__ void flip_bits(uint32_t *vbs, int K, const Move &mv)
 // completes bin u inserts it as the window's new top byte. w_b = 60|b| - 1 for b < 0, else 0.
 // pstart[w] = first record in row word w (INT_MAX if none).
 // ------------------------------------------------------------------------------------------
-template <int K, bool XG = false>
+template <int K, bool XG = false, bool OVL = true>
 __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
                               uint32_t *Xarg, const Move &mv, bool a_done = false)
 {
@@ -501,7 +531,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
         uneg = min(max(uneg, 0), U);
         int utop = ((I.maxS + 2 * K - vmin) >> 1) + 1;  // least u with vmin + 2u > maxS + 2K
         utop = min(max(utop, uneg), U);
-        const int n0 = (utop - uneg + 1) >> 1, n1 = (utop - uneg) >> 1;  // points of walk 0 / 1
+        const int n0 = (utop - uneg + 1) >> 1;  // points of walk 0 (walk 1: the rest of [uneg, utop))
         // the placement is sequential (padding depends on the position within the row word), so
         // one thread walks the points: deep (contiguous), walk 0, walk 1 (padded), top (contiguous)
         int pos = 0, runp = 0, rneg = 0, rtop = 0, pkb1 = 0;
@@ -532,6 +562,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
                 pos += __shfl_sync(FULL, inc, 31);
                 runp += __shfl_sync(FULL, incp, 31);
             }
+            PH(7);
             // broadcast to lane 0 (the cuts at q = U take the totals)
             const unsigned b1 = __ballot_sync(FULL, sel & 1), b2 = __ballot_sync(FULL, sel & 2), b4 = __ballot_sync(FULL, sel & 4);
             rneg = b1 ? __shfl_sync(FULL, rneg, __ffs(b1) - 1) : pos;
@@ -574,22 +605,7 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
                 pos += Lv;
             }
         }
-        if (lane < 2) {  // walk p = lane: first / last point, initial window, trailing bins
-            const int np = lane ? n1 : n0, a = uneg + lane, z = a + 2 * (np - 1);
-            uint32_t win = 0, htr = 0;
-            int trl = 0;
-            if (np > 0) {
-                for (int i = 0; i < 4; i++)
-                    if (a + 2 * i <= z) win |= (uint32_t)cnt[uf + a + 2 * i] << (8 * i);
-                for (int i = 1; i <= K; i++) {
-                    const int b = vmin + 2 * (z + 2 * i - K);
-                    if (b >= 0 && b <= n) htr |= (uint32_t)Hs[b] << (8 * (i - 1));
-                    if (b < 0) trl = 1;
-                }
-            }
-            ps.pkwin[lane] = win; ps.pkhtr[lane] = htr; ps.pktrl[lane] = trl; ps.pkz[lane] = np > 0 ? z : -1;
-            ps.pkw0[lane] = 0;
-        }
+        if (lane < 2) ps.pkw0[lane] = 0;  // (the walks' window constants: step C, warp 1)
         if (lane == 0) {
             ps.P = runp; ps.pkb1 = pkb1; ps.Wp = (pos + 31) >> 5;
             ps.vmin = vmin; ps.U = U; ps.NB = U + 2 * K; ps.ufirst = uf;
@@ -606,21 +622,55 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
     //    pstart[w] = shared address of the first record in row word w
     const int vmin = ps.vmin, NB = ps.NB, uf = ps.ufirst, uneg = ps.uneg, utop = ps.utop;
     const uint32_t pk0 = (uint32_t)__cvta_generic_to_shared(pk);
-    for (int j = tid; j < m; j += NT) {
-        const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
-        rowAt[p] = j;
+    // OVL (one search, latency-bound): warps 2.. place the rows, meet at a named barrier and
+    // transpose X (step D) while warp 0 builds the records and warp 1 the bin constants (neither
+    // needs the placement). Batched searches place the rows first with every thread.
+    if (!OVL) {
+        for (int j = tid; j < m; j += NT) {
+            const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
+            rowAt[p] = j;
+        }
+        __syncthreads();
     }
-    __syncthreads();  // rows placed: step D (X, warps 2..) overlaps the rest of C (warps 0, 1)
     PH(2);
     if (warp >= 2) {
+        if (OVL) {
+            for (int j = tid - 64; j < m; j += NT - 64) {
+                const int p = atomicAdd(&cur[(Ys[j] - vlo) >> 1], 1);
+                rowAt[p] = j;
+            }
+            asm volatile("bar.sync 1, %0;" ::"r"(NT - 64) : "memory");
+        }
         plan_transpose_warps(I, Ar, sm, L, ps, X, 2, NWARP - 2);
     } else if (warp == 1) {
         // deep rows: 60 |b| per row at t = 0, minus 240 t (abs form); bin constants; H of the walked
         // bins (sums by warp reductions, no shared atomics)
+        // walk q = lane (q = 0, 1): last point z, initial window (rows of the first four points),
+        // trailing bins (the K bins past z: H bytes, one of them negative?) -> pkwt[q]
+        int zq = -1;
+        if (lane < 2) {
+            const int n0 = (utop - uneg + 1) >> 1, n1 = (utop - uneg) >> 1;
+            const int np = lane ? n1 : n0, a = uneg + lane, z = a + 2 * (np - 1);
+            uint32_t win = 0, htr = 0;
+            int trl = 0;
+            if (np > 0) {
+#pragma unroll
+                for (int i = 0; i < 4; i++)
+                    if (a + 2 * i <= z) win |= (uint32_t)cnt[uf + a + 2 * i] << (8 * i);
+#pragma unroll
+                for (int i = 1; i <= K; i++) {
+                    const int b = vmin + 2 * (z + 2 * i - K);
+                    if (b >= 0 && b <= n) htr |= (uint32_t)Hs[b] << (8 * (i - 1));
+                    if (b < 0) trl = 1;
+                }
+            }
+            zq = np > 0 ? z : -1;
+            ps.pkwt[lane] = make_uint4(win, htr, (uint32_t)trl, (uint32_t)zq);
+        }
         unsigned dneg = 0;
         for (int v = lane; v < uneg; v += 32)
             dneg += (unsigned)cnt[uf + v] * (unsigned)(60 * (2 * K - (vmin + 2 * v)));
-        const int z0 = ps.pkz[0], z1 = ps.pkz[1];
+        const int z0 = __shfl_sync(FULL, zq, 0), z1 = __shfl_sync(FULL, zq, 1);
         int hw = 0;
         for (int beta = lane; beta < NB; beta += 32) {
             const int b = vmin + 2 * (beta - K);
@@ -668,13 +718,13 @@ __device__ void build_plan_pk(const DevInst &I, const uint32_t *Ar, unsigned cha
             }
         }
         __syncwarp();  // the writers of pkw0 are in this warp
+        PH(9);
         if (lane < 2) {  // the walks' ready-to-use addresses and constants (read by pk_walk)
             const int q = tid, wd = ps.pkw0[q];
             const int pb = q ? ps.pkb1 : 0, pe = q ? ps.P : ps.pkb1;
             const uint32_t xb = XG ? (uint32_t)(wd * n) : (uint32_t)__cvta_generic_to_shared(X + wd * n);
             ps.pkwk[q] = make_uint4(xb, pk0 + 16u * pb, pk0 + 16u * pe,
                                     (uint32_t)__cvta_generic_to_shared(pstart + wd + 1));
-            ps.pkwt[q] = make_uint4(ps.pkwin[q], ps.pkhtr[q], (uint32_t)ps.pktrl[q], (uint32_t)ps.pkz[q]);
         }
     }
     __syncthreads();  // X (warps 2..), records, bins, pkwk / pkwt are published
@@ -834,11 +884,11 @@ __device__ void build_plan_seg(const DevInst &I, const uint32_t *Ar, unsigned ch
 // every byte the walk window can hold -- a walked bin's own rows plus the rows K points below it in
 // its walk -- is <= 255, and so is H_b of every walked bin; else the segment plan. Decided per
 // iteration by warp 0 after the shared counting sort.
-template <int K, bool XG = false>
+template <int K, bool XG = false, bool OVL = true>
 __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
                            uint32_t *Xarg, const Move &mv = Move{0, 0, 0, 0})
 {
-    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv); return; }
+    if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG, OVL>(I, Ar, sm, L, ps, Xarg, mv); return; }
     if (!I.pkw) { build_plan_seg<K, XG>(I, Ar, sm, L, ps, Xarg, mv, false); return; }
     const int tid = threadIdx.x, lane = tid & 31;
     int *cnt = (int *)(sm + L.cnt);
@@ -875,7 +925,7 @@ __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *
         if (lane == 0) ps.pkok = anybad ? 0 : 1;
     }
     __syncthreads();
-    if (ps.pkok) build_plan_pk<K, XG>(I, Ar, sm, L, ps, Xarg, mv, true);
+    if (ps.pkok) build_plan_pk<K, XG, OVL>(I, Ar, sm, L, ps, Xarg, mv, true);
     else build_plan_seg<K, XG>(I, Ar, sm, L, ps, Xarg, mv, true);
 }
 
@@ -1055,9 +1105,11 @@ __device__ __forceinline__ void load_planes(const uint32_t *__restrict__ xr, int
 template <int K>
 __device__ __forceinline__ void pk_step(const uint4 &r, uint32_t lo, uint32_t hi, uint32_t lh, uint32_t &w, int &f)
 {
-    w += 255u * (uint32_t)__popc(lo & r.x);
-    if (K >= 2) w += 65535u * (uint32_t)__popc(hi & r.x);
+    // (c3 first: with this order ptxas's register assignment of the record loop avoids the dispatch
+    // stalls the c1, c2, c3 order showed in the batched kernel)
     if (K == 3) w += 16711425u * (uint32_t)__popc((PK_TWO_PLANES ? lo & hi : lh) & r.x);
+    if (K >= 2) w += 65535u * (uint32_t)__popc(hi & r.x);
+    w += 255u * (uint32_t)__popc(lo & r.x);
     // hb: byte 1 = h (byte 0 of w) for a final piece (selector 0x4404), 0 otherwise (0x4444)
     uint32_t hb, fu = (uint32_t)f;
     asm("prmt.b32 %0, %1, %2, %3;" : "=r"(hb) : "r"(w), "r"(0u), "r"(r.w));
@@ -1185,7 +1237,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                                          const PlanScalars &ps, const uint32_t *Xarg, uint32_t M, uint32_t blo, uint32_t bhi,
                                          const uint32_t *until, uint32_t ubase, uint32_t t, int32_t *fit_out,
                                          const uint2 *tri = nullptr, int aspire = 0,
-                                         int best_f = 0, const uint32_t *tbits = nullptr)
+                                         int best_f = 0, const uint32_t *tbits = nullptr, bool enc = false)
 {
     // rank r tabu at iteration t: the until[] array (smem slice or global), or the bitmap
     auto is_tabu = [&](uint32_t r) -> bool {
@@ -1231,6 +1283,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const bool tA = is_tabu(rA);
             const bool tB = is_tabu(rb);
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
+            // (rank keys only: launch_search sets enc_keys only when no CTA takes this path)
             const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
             const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
             if ((!tA || (aspire && fA < best_f)) && kA < best) best = kA;
@@ -1263,8 +1316,8 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
             const bool tA = is_tabu(rA);
             const bool tB = is_tabu(rb);
             if (WRITE_ALL) { fit_out[rA] = fA; if (vB) fit_out[rB] = fB; }
-            const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | rA;
-            const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | rb;
+            const unsigned long long kA = ((unsigned long long)(uint32_t)fA << 32) | (enc ? enc_flip<K>(a0, b0, c0) : rA);
+            const unsigned long long kB = ((unsigned long long)(uint32_t)fB << 32) | (enc ? enc_flip<K>(a1, b1, c1) : rb);
             if ((!tA || (aspire && fA < best_f)) && kA < best) best = kA;
             if ((!tB || (aspire && fB < best_f)) && kB < best) best = kB;
         }
@@ -1291,7 +1344,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
                                     : eval_fit<K, false>(X, pieces, bins, I.n, er, 2 * I.m, a, b, c);
                 }
                 if (WRITE_ALL) fit_out[r] = f;
-                const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | r;
+                const unsigned long long key = ((unsigned long long)(uint32_t)f << 32) | (enc ? enc_flip<K>(a, b, c) : r);
                 // admissible: not tabu, or (aspiration) better than the best fitness so far
                 if ((!tab || (aspire && f < best_f)) && key < best) best = key;
             }
@@ -1511,9 +1564,11 @@ __global__ void __launch_bounds__(NT) k_init(DevInst I, const int8_t *V0, uint32
     }
 }
 
-// The persistent tabu search: all iterations in one cooperative launch. With A.R > 0 the grid is
-// split into A.groups groups; each group runs its restarts one after another (batched restarts).
-template <int K>
+// The persistent tabu search: all iterations in one cooperative launch. BATCH (A.R > 0): the grid
+// is split into groups; each group runs its restarts one after another (batched restarts). The two
+// modes are separate instantiations, so code that only one of them runs (the peer exchange and the
+// flip-set keys of a single search) does not weigh on the other's register allocation.
+template <int K, bool BATCH>
 __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
 {
     extern __shared__ __align__(16) unsigned char sm[];
@@ -1521,7 +1576,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
     const Smem L = smem_layout(A.I.m, A.I.n, A.I.XW, A.I.NWn, K, A.a_in_smem, A.Xg != nullptr, A.I.pkw);
     int *Ys = (int *)(sm + L.Y);
     uint32_t *vbs = (uint32_t *)(sm + L.vb);
-    const bool batch = A.R > 0;
+    constexpr bool batch = BATCH;
     const int lane = threadIdx.x & 31;
     const uint32_t *Ar = batch ? load_common<K>(A, sm, L) : load_state<K>(A, sm, L, ps);
     __shared__ unsigned long long *s_peers[MAX_PEERS];
@@ -1591,8 +1646,8 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
         Move mv{0, 0, 0, 0};  // accepted, not yet applied
         for (; t <= t0 + A.iters; t++) {
             if (A.stop_on_zero && f == 0) break;
-            if (A.Xg) build_plan<K, true>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
-            else build_plan<K, false>(A.I, Ar, sm, L, ps, nullptr, mv);
+            if (A.Xg) build_plan<K, true, !BATCH>(A.I, Ar, sm, L, ps, X_OF(A, sm, L), mv);
+            else build_plan<K, false, !BATCH>(A.I, Ar, sm, L, ps, nullptr, mv);
             // (the solution-list barrier is passed once per iteration, before the exchange: pass tg + 1)
             if (A.sol_list) {
                 sol_tabu<K>(A, sm, L, vbs, gg, until, t, bid, nb, gslots + 24, tg + 1, &s_xto);
@@ -1600,9 +1655,9 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             }
             unsigned long long mine =
                 A.Xg ? eval_range<K, false, true>(A.I, sm, L, ps, X_OF(A, sm, L), A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                  nullptr, tri, A.aspiration, (int)best_f, tb)
+                                                  nullptr, tri, A.aspiration, (int)best_f, tb, !BATCH && A.enc_keys)
                      : eval_range<K, false, false>(A.I, sm, L, ps, nullptr, A.M, blo, bhi, until, ubase, (uint32_t)t,
-                                                   nullptr, tri, A.aspiration, (int)best_f, tb);
+                                                   nullptr, tri, A.aspiration, (int)best_f, tb, !BATCH && A.enc_keys);
             mine = warp_min_k(mine);
             if (lane == 0 && mine != (unsigned long long)KEY_NONE) atomicMin(&ps.key, mine);
             // the rank leaving the FIFO after this iteration (accepted at t - L), read before this
@@ -1613,7 +1668,7 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             PH(4);
             unsigned long long key = ps.key;
             tg++;
-            if (A.npeers > 0) {
+            if (!BATCH && A.npeers > 0) {
                 // cross-GPU exchange (lns_attach_peers), two levels:
                 //  1. inside the partition as below (.gpu scope): MIN into the local slot tg%3, one
                 //     arrival on the local counter;
@@ -1719,7 +1774,15 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             }
             PH(5);
             if (key == (unsigned long long)KEY_NONE) { failed = true; break; }
-            const uint32_t r = (uint32_t)(key & 0xffffffffu);
+            // the accepted move: its flip set (the next plan applies it) and its rank
+            uint32_t r;
+            if (!BATCH && A.enc_keys) {
+                dec_flip<K>((uint32_t)(key & 0xffffffffu), mv.a, mv.b, mv.c);
+                r = rank_tab<K>(A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), mv.a, mv.b, mv.c);
+            } else {
+                r = (uint32_t)(key & 0xffffffffu);
+                unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), mv.a, mv.b, mv.c);
+            }
             f = (int64_t)(key >> 32);
             if (tb) {
                 // bits_mode: r_{t-L} leaves the tabu list, r_t enters it (owner CTA's thread 0: the
@@ -1740,7 +1803,6 @@ __global__ void __launch_bounds__(NT, 1) k_search(SearchArgs A)
             if (f == 0 && zero_it < 0) zero_it = t;
             // the move is applied by the next plan's step A (or below, after the last iteration)
             mv.on = 1;
-            unrank_tab<K>(r, A.I.n, A.M, (const uint32_t *)(sm + L.T2), (const uint32_t *)(sm + L.T3), mv.a, mv.b, mv.c);
             PH(6);
         }
         if (mv.on) apply_move<K>(A.I, Ar, Ys, vbs, mv.a, mv.b, mv.c);
@@ -2721,6 +2783,7 @@ SearchArgs make_args(lns_ctx *c, const Geometry &g, int64_t iters, int64_t L, in
     A.peers = nullptr; A.npeers = 0; A.part = 0; A.nb_total = 0; A.timeout_ns = 0;
     A.grid_timeout_ns = c->grid_timeout_ms * 1000000LL;
     A.plain_launch = (flags & LNS_PLAIN_LAUNCH) ? 1 : 0;
+    A.enc_keys = 0;
     return A;
 }
 
@@ -2860,15 +2923,21 @@ lns_status setup_bits(lns_ctx *c, SearchArgs &A, int groups, bool zero_now, cuda
 template <int K>
 lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream_t st, int nb_force = 0)
 {
+    const void *kern = (const void *)k_search<K, false>;
     // persistent geometry: first the CTA count at the eval footprint, then cache the until[]
     // slice in shared memory if it fits next to it
     const int budget = c->smemOptin - 1024;  // static shared memory of the kernels stays < 1 KiB
-    CK(allow_smem((const void *)k_search<K>, budget));
+    CK(allow_smem(kern, budget));
     int occ = 0;
-    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K>, NT, g.smem_eval));
+    CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k_search<K, false>, NT, g.smem_eval));
     if (occ < 1) return fail(LNS_ERANGE, "persistent kernel does not fit on an SM");
     const int nb = nb_force > 0 ? nb_force : search_blocks(c, A.hi - A.lo, 1);
     if (A.npeers > 0) A.nb_total = (int64_t)nb * A.npeers;
+    // one search over all its CTAs (latency-bound): keys carry the flip set, so the winner needs no
+    // unranking after the exchange (every partition of a peer run takes the same choice: same n, k)
+    // (not when a CTA's slice takes eval_range's contiguous-run path: its keys carry ranks)
+    A.enc_keys = ((K == 3 && A.I.n <= 1024) || (K == 2 && A.I.n <= 65536)) &&
+                 (A.hi - A.lo) / (uint32_t)nb + 64u < 4u * NT ? 1 : 0;
     A.I.pad = pad_for(g, A.hi - A.lo, nb);
     A.I.pkw = pkw_for(g, A.hi - A.lo, nb);
     const size_t smem = cache_geometry(A, g, nb, budget);
@@ -2879,8 +2948,8 @@ lns_status launch_search(lns_ctx *c, SearchArgs A, const Geometry &g, cudaStream
     k_init_slots<<<1, 64, 0, st>>>(c->d_slots, 1);
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
-    if (A.plain_launch) CK(cudaLaunchKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
-    else CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(nb), dim3(NT), args, smem, st));
+    if (A.plain_launch) CK(cudaLaunchKernel(kern, dim3(nb), dim3(NT), args, smem, st));
+    else CK(cudaLaunchCooperativeKernel(kern, dim3(nb), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     return LNS_OK;
 }
@@ -2891,7 +2960,7 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int grid, i
                         int64_t *gslots, cudaStream_t st)
 {
     const int budget = c->smemOptin - 1024;
-    CK(allow_smem((const void *)k_search<K>, budget));
+    CK(allow_smem((const void *)k_search<K, true>, budget));
     A.I.pad = pad_for(g, A.hi - A.lo, nb_min);
     A.I.pkw = pkw_for(g, A.hi - A.lo, nb_min);
     const size_t smem = cache_geometry(A, g, nb_min, budget);
@@ -2907,7 +2976,7 @@ lns_status launch_batch(lns_ctx *c, SearchArgs A, const Geometry &g, int grid, i
     A.groups = 0;
     void *args[] = {&A};
     CK(cudaEventRecord(c->ev0, st));
-    CK(cudaLaunchCooperativeKernel((void *)k_search<K>, dim3(grid), dim3(NT), args, smem, st));
+    CK(cudaLaunchCooperativeKernel((void *)k_search<K, true>, dim3(grid), dim3(NT), args, smem, st));
     CK(cudaEventRecord(c->ev1, st));
     return LNS_OK;
 }

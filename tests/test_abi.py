@@ -106,3 +106,31 @@ def test_c_example_builds_against_the_header_and_fails_loudly_without_gpu(tmp_pa
         return
     out = subprocess.run([exe, "21", "21", "1", "10"], capture_output=True, text=True, timeout=120)
     assert out.returncode == 1 and "CUDA error" in out.stderr, out.stderr
+
+
+def test_bench_refuses_more_gpus_than_visible():
+    """bench.py --gpus N without torchrun re-launches itself with N ranks only if N GPUs are
+    visible; otherwise it prints an error line and exits 2 (it never reports n_gpus: 1 for N > 1).
+    On this GPU-less host: 0 visible GPUs."""
+    import json
+    import sys
+
+    import torch
+
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is visible")
+    out = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--gpus", "2", "--steps", "1"],
+                         capture_output=True, text=True, timeout=300)
+    assert out.returncode == 2, out.stdout + out.stderr
+    line = json.loads(out.stdout.strip().splitlines()[-1])
+    assert "error" in line and "--gpus 2" in line["error"]
+
+
+def test_bench_reference_arm_ignores_gpu_count_on_nonzero_ranks():
+    """--impl reference under torchrun: ranks other than 0 exit 0 without work (and print nothing)."""
+    import sys
+
+    env = {**os.environ, "RANK": "1", "WORLD_SIZE": "2", "LOCAL_RANK": "1"}
+    out = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--impl", "reference", "--gpus", "2"],
+                         capture_output=True, text=True, timeout=300, env=env)
+    assert out.returncode == 0 and out.stdout.strip() == "", out.stdout + out.stderr
