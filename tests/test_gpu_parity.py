@@ -723,12 +723,18 @@ def test_pool_recycles_context_buffers(L, orc):
 def test_compute_sanitizer_clean(L, tool):
     """every kernel family (persistent search with one and several CTAs,
     batched restarts, stepped search, eval_all, the m > 255 path, the UBQP kernels) runs clean under
-    compute-sanitizer on small instances."""
+    compute-sanitizer on small instances.
+
+    Opt-in (LNS_SANITIZE=1): the GPU pool this round runs on has closed compute-sanitizer (runs
+    under it left GPUs needing a reset), so the default suite does not start it. Round 1 ran all
+    three tools clean; the bounds-checked parity tests below stand in for it."""
     import os
     import shutil
     import subprocess
     import sys
 
+    if os.environ.get("LNS_SANITIZE") != "1":
+        pytest.skip("compute-sanitizer is opt-in (LNS_SANITIZE=1): closed on this GPU pool")
     exe = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
     if not os.path.exists(exe):
         pytest.skip("compute-sanitizer not found")
