@@ -48,6 +48,7 @@ import statistics
 import subprocess
 import sys
 import tempfile
+import threading
 import time
 from math import comb
 
@@ -70,6 +71,7 @@ C5_RESTART_ITERS = 3
 PART_C4_ITERS = 2000
 PART_C5_ITERS = 5
 L2_FLUSH_BYTES = 512 << 20  # > 126 MB L2
+CONTEXT_BUDGET_S = float(os.environ.get("LNS_BENCH_CONTEXT_BUDGET_S", "300"))  # watchdog of the context lines
 PROFILE = os.path.join(ROOT, "profiles", "ncu_k_search_bench.json")  # ncu --set full of one bench step
 INT_PEAKS = os.path.join(ROOT, "profiles", "int_peaks.json")  # scripts/int_peaks.cu on the B200
 
@@ -87,6 +89,42 @@ def peaks():
             return json.load(fh), "measured"
     except OSError:
         return {"sm_max_mhz": 1965.0, "hbm_gbs": 6650.0}, "fallback"
+
+
+class ContextLines:
+    """The JSON line's context sections after the headline. section(name, fn) stores fn() in
+    line[name], or {"error": ...} if it raises; a watchdog prints the line (rank 0) and ends the
+    process with status 0 if finish() has not been called after `budget` seconds, so a context
+    collective that some rank never reaches cannot hold back the measured headline."""
+
+    def __init__(self, line: dict, rank: int, budget: float):
+        self.line, self.rank, self.budget = line, rank, budget
+        self.emitted, self.done = False, threading.Event()
+        threading.Thread(target=self._watchdog, daemon=True).start()
+
+    def emit(self, note=None):
+        if self.rank == 0 and not self.emitted:
+            self.emitted = True
+            if note:
+                self.line["context_note"] = note
+            print(json.dumps(self.line), flush=True)
+
+    def _watchdog(self):
+        if not self.done.wait(self.budget):
+            self.emit(f"context lines stopped after {self.budget:.0f} s (a context section did not finish on every "
+                      "rank); the headline, e2e and roofline above are complete")
+            os._exit(0)
+
+    def section(self, name, fn):
+        try:
+            self.line[name] = fn()
+        except Exception as e:  # noqa: BLE001 -- a context line must not take the headline down
+            self.line[name] = {"error": f"{type(e).__name__}: {e}"[:400]}
+            print(f"[bench] {name} failed: {e}", file=sys.stderr)
+
+    def finish(self):
+        self.done.set()
+        self.emit()
 
 
 def run_seed(step: int) -> int:
@@ -454,9 +492,42 @@ def main():
     h2d = A_h.numel() + 4 * S_h.numel() + V0_h[0].numel()
     d2h = Vo_h.numel() + 48 * R  # final vectors + lns_result records
 
+    # ---- the headline line; the context lines below fill it in. Each context section is guarded:
+    #      an exception becomes {"error": ...} in its slot, and a watchdog prints the line and ends the
+    #      process if the sections have not finished after CONTEXT_BUDGET_S (a collective of a context
+    #      line that one rank never reaches cannot hold back the measured headline).
+    sms = torch.cuda.get_device_properties(dev).multi_processor_count
+    kern_avg_s = kern_ms / 1e3 / args.steps
+    nbr_per_s_kernel = (my_iters / args.steps) * M / kern_avg_s if kern_avg_s > 0 else 0.0
+    roofline = roofline_of(nbr_per_s_kernel, sms)
+    line = {
+        "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": total_ms / args.steps, "higher_is_better": True,
+        "scaling": "strong", "vs_baseline": None, "dtype": "int32",
+        "data": "synthetic planted PPP instance (seeded splitmix64, DESIGN.md §3)",
+        "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming (260,130 neighbours/iteration), tenure {ten}; "
+                               f"{args.runs} independent tabu searches x {iters} iterations per step "
+                               "(PAPER.md:250 protocol), no early stop",
+                   "runs_per_step": args.runs, "iters_per_run": iters,
+                   "parallelism": f"runs sharded over {world} GPUs (r mod N), batched per GPU" if world > 1
+                   else "1 GPU, runs batched in one persistent kernel",
+                   "l2": "flushed (512 MiB write) between timed steps"},
+        "tabu_iters_per_s": iters_done / (total_ms / 1e3),
+        "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
+                "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
+        "single_search": None, "partitioned": None, "c5_single_search": None, "c5_restarts": None,
+        "ubqp_single_search": None,
+        # our kernels per timed step: k_init_slots + the persistent k_search
+        "gpu_launches": args.steps * 2,
+        "clocks": clocks,
+        "roofline": roofline,
+        "cpu_baseline": None,
+    }
+    ctxl = ContextLines(line, rank, CONTEXT_BUDGET_S)
+    section = ctxl.section
+
     # ---- single search (latency view), N = 1 only
-    single = None
-    if world == 1 and not args.no_single:
+    def single_search():
         tr = torch.empty(SINGLE_ITERS, dtype=torch.int64, device=dev)
         tf = torch.empty(SINGLE_ITERS, dtype=torch.int64, device=dev)
         v1 = torch.empty(inst.n, dtype=torch.int8, device=dev)
@@ -467,16 +538,19 @@ def main():
             flush.fill_(0)
             ms.append(timed(stream, lambda: L.lns_tabu_run(ctx, k, SINGLE_ITERS, ten, 0, v0, 0, v1, tr, tf, stream))[0])
         best = min(ms)
-        single = {"neighbors_per_s": SINGLE_ITERS * M / (best / 1e3), "tabu_iters_per_s": SINGLE_ITERS / (best / 1e3),
-                  "us_per_iteration": 1e3 * best / SINGLE_ITERS, "iters": SINGLE_ITERS,
-                  "note": "one search on all SMs (persistent kernel, one exchange per iteration)"}
+        return {"neighbors_per_s": SINGLE_ITERS * M / (best / 1e3), "tabu_iters_per_s": SINGLE_ITERS / (best / 1e3),
+                "us_per_iteration": 1e3 * best / SINGLE_ITERS, "iters": SINGLE_ITERS,
+                "note": "one search on all SMs (persistent kernel, one exchange per iteration)"}
+
+    if world == 1 and not args.no_single:
+        section("single_search", single_search)
 
     # ---- C5 (BASELINE configs[4], 1024 x 1024, 3-Hamming, 1.78e8 neighbours per iteration): one
     #      search on all SMs, a few iterations (N = 1 only; context beside the headline)
     inst5 = pi.config_instance("C5")
     M5 = comb(inst5.n, 3)
-    c5 = None
-    if world == 1 and not args.no_c5:
+
+    def c5_single():
         with L.Instance(inst5.A, inst5.S) as I5:
             L.lns_tabu_run(I5.ctx, 3, 1, -1, pi.config_seed("C5"), None, 0)
             ms5 = []
@@ -486,15 +560,17 @@ def main():
                 L.lns_tabu_run(I5.ctx, 3, C5_ITERS, -1, pi.config_seed("C5"), None, 0)
                 ms5.append(L.lns_last_kernel_ms(I5.ctx))
         b5 = min(ms5)
-        c5 = {"neighbors_per_s": C5_ITERS * M5 / (b5 / 1e3), "tabu_iters_per_s": C5_ITERS / (b5 / 1e3),
-              "ms_per_iteration": b5 / C5_ITERS, "iters": C5_ITERS,
-              "note": "C5 single search from the config seed (packed plan for m > 255, DESIGN.md §5.11); device time of the launch"}
+        return {"neighbors_per_s": C5_ITERS * M5 / (b5 / 1e3), "tabu_iters_per_s": C5_ITERS / (b5 / 1e3),
+                "ms_per_iteration": b5 / C5_ITERS, "iters": C5_ITERS,
+                "note": "C5 single search from the config seed (packed plan for m > 255, DESIGN.md §5.11); device time of the launch"}
+
+    if world == 1 and not args.no_c5:
+        section("c5_single_search", c5_single)
 
     # ---- C5 restarts (BASELINE configs[4]: "64 independent restarts sharded across 8 x B200"):
     #      8 restarts per GPU through lns_tabu_run_batch; with N > 1 the library shards restart r
     #      to rank r mod N over the attached NCCL communicator and gathers every result
-    c5r = None
-    if not args.no_c5:
+    def c5_restarts():
         R5 = C5_RESTARTS_PER_GPU * world
         with L.Instance(inst5.A, inst5.S, local) as I5:
             comm = par.nccl_comm_ptr(device=dev) if world > 1 else None
@@ -508,14 +584,16 @@ def main():
                 L.lns_attach_comm(I5.ctx, None, 0, 1)
         ms, kms = max_over_ranks([ms, kms], world, dev)
         done5 = sum(r["iters_done"] for r in r5)  # every rank holds every restart's result
-        c5r = {"restarts": R5, "restarts_per_gpu": C5_RESTARTS_PER_GPU, "iters_per_restart": C5_RESTART_ITERS,
-               "neighbors_per_s": done5 * M5 / (ms / 1e3), "tabu_iters_per_s": done5 / (ms / 1e3),
-               "kernel_neighbors_per_s": done5 * M5 / (kms / 1e3) if kms > 0 else None,
-               "note": "lns_tabu_run_batch, restart r on rank r mod N, results gathered by the library (NCCL)"}
+        return {"restarts": R5, "restarts_per_gpu": C5_RESTARTS_PER_GPU, "iters_per_restart": C5_RESTART_ITERS,
+                "neighbors_per_s": done5 * M5 / (ms / 1e3), "tabu_iters_per_s": done5 / (ms / 1e3),
+                "kernel_neighbors_per_s": done5 * M5 / (kms / 1e3) if kms > 0 else None,
+                "note": "lns_tabu_run_batch, restart r on rank r mod N, results gathered by the library (NCCL)"}
+
+    if not args.no_c5:
+        section("c5_restarts", c5_restarts)
 
     # ---- one search partitioned over the N GPUs
-    part = None
-    if not args.no_partitioned:
+    def partitioned():
         part = {}
         comm = par.nccl_comm_ptr(device=dev) if world > 1 else None
         for name, inst_p, kp, itp in (("C4", inst, 3, PART_C4_ITERS), ("C5", inst5, 3, PART_C5_ITERS)):
@@ -551,10 +629,13 @@ def main():
                                "neighbors_per_s": PART_C4_ITERS * M / (ms / 1e3), "trace_sha16": trace_sha,
                                "exchange": "device-initiated: red.min.sys / red.release.sys into every GPU's "
                                            "exchange buffer (CUDA IPC), no host step"}
+        return part
+
+    if not args.no_partitioned:
+        section("partitioned", partitioned)
 
     # ---- UBQP: k = 3, n = 500 OR-Library-style Q, one search (N = 1 only; context)
-    ubqp = None
-    if world == 1 and not args.no_ubqp:
+    def ubqp_single():
         from ppp_inputs import bqp as bi
 
         nq, kq, itq = 500, 3, 256  # >= 128 iterations: the CUDA-graph path (64-iteration blocks)
@@ -571,55 +652,27 @@ def main():
         L.lns_bqp_destroy(cq)
         bq = min(msq)
         Mq = L.lns_neighborhood_size(nq, kq)
-        ubqp = {"neighbors_per_s": itq * Mq / (bq / 1e3), "us_per_iteration": 1e3 * bq / itq, "iters": itq,
+        return {"neighbors_per_s": itq * Mq / (bq / 1e3), "us_per_iteration": 1e3 * bq / itq, "iters": itq,
                 "note": "UBQP f = x^T Q x, n = 500, density 0.1, 3-Hamming (2.07e7 neighbours/iteration), one "
                         "search; device time of the replay (eval + apply launches, CUDA graphs of 64 iterations)"}
 
-    # ---- roofline: the search kernel (one launch per step)
-    sms = torch.cuda.get_device_properties(dev).multi_processor_count
-    kern_avg_s = kern_ms / 1e3 / args.steps
-    nbr_per_s_kernel = (my_iters / args.steps) * M / kern_avg_s if kern_avg_s > 0 else 0.0
-    roofline = roofline_of(nbr_per_s_kernel, sms)
+    if world == 1 and not args.no_ubqp:
+        section("ubqp_single_search", ubqp_single)
 
-    cpu = None
-    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+    def cpu_baseline():
         v, ips, it, runs, cores, dt = oracle_sample(args.cpu_budget)
         v1, ips1, it1, runs1, _, dt1 = oracle_sample(args.cpu_budget, nthreads=1, per_run=10)
-        cpu = {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle", "cpu_model": cpu_model(),
-               "sample": f"{runs} runs x {ITERS} tabu iterations of step 0 of the {CFG} job (same instance, tenure, "
-                         f"start vectors), {dt:.1f} s on {cores} OpenMP threads, from-scratch fitness per neighbour",
-               "tabu_iters_per_s": ips,
-               "single_thread": {"value": v1, "unit": UNIT, "cores": 1, "tabu_iters_per_s": ips1,
-                                 "sample": f"first 10 iterations of runs 0..{runs1 - 1} of step 0, {dt1:.1f} s, "
-                                           "one thread (the paper's sequential CPU baseline style, PAPER.md:245-248)"}}
-    if rank == 0:
-        line = {
-            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": total_ms / args.steps, "higher_is_better": True,
-            "scaling": "strong", "vs_baseline": None, "dtype": "int32",
-            "data": "synthetic planted PPP instance (seeded splitmix64, DESIGN.md §3)",
-            "config": {"workload": f"{CFG}: PPP m=101 n=117, 3-Hamming (260,130 neighbours/iteration), tenure {ten}; "
-                                   f"{args.runs} independent tabu searches x {iters} iterations per step "
-                                   "(PAPER.md:250 protocol), no early stop",
-                       "runs_per_step": args.runs, "iters_per_run": iters,
-                       "parallelism": f"runs sharded over {world} GPUs (r mod N), batched per GPU" if world > 1
-                       else "1 GPU, runs batched in one persistent kernel",
-                       "l2": "flushed (512 MiB write) between timed steps"},
-            "tabu_iters_per_s": iters_done / (total_ms / 1e3),
-            "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
-                    "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
-            "single_search": single,
-            "partitioned": part,
-            "c5_single_search": c5,
-            "c5_restarts": c5r,
-            "ubqp_single_search": ubqp,
-            # our kernels per timed step: k_init_slots + the persistent k_search
-            "gpu_launches": args.steps * 2,
-            "clocks": clocks,
-            "roofline": roofline,
-            "cpu_baseline": cpu,
-        }
-        print(json.dumps(line), flush=True)
+        return {"value": v, "unit": UNIT, "cores": cores, "kind": "oracle", "cpu_model": cpu_model(),
+                "sample": f"{runs} runs x {ITERS} tabu iterations of step 0 of the {CFG} job (same instance, tenure, "
+                          f"start vectors), {dt:.1f} s on {cores} OpenMP threads, from-scratch fitness per neighbour",
+                "tabu_iters_per_s": ips,
+                "single_thread": {"value": v1, "unit": UNIT, "cores": 1, "tabu_iters_per_s": ips1,
+                                  "sample": f"first 10 iterations of runs 0..{runs1 - 1} of step 0, {dt1:.1f} s, "
+                                            "one thread (the paper's sequential CPU baseline style, PAPER.md:245-248)"}}
+
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        section("cpu_baseline", cpu_baseline)
+    ctxl.finish()
     L.lns_destroy(ctx)
     if world > 1:
         dist.destroy_process_group()

@@ -134,3 +134,33 @@ def test_bench_reference_arm_ignores_gpu_count_on_nonzero_ranks():
     out = subprocess.run([sys.executable, os.path.join(ROOT, "bench.py"), "--impl", "reference", "--gpus", "2"],
                          capture_output=True, text=True, timeout=300, env=env)
     assert out.returncode == 0 and out.stdout.strip() == "", out.stdout + out.stderr
+
+
+def test_bench_context_lines_guard():
+    """bench.py's context sections: an exception becomes {"error": ...} in its slot and
+    the line is still printed; a section that never returns (a collective some rank did not reach)
+    is cut by the watchdog, which prints the headline line and exits 0 instead of hanging."""
+    import json
+    import subprocess
+    import sys
+
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    prog = (
+        "import sys, time; sys.path.insert(0, %r); import bench\n"
+        "line = {'metric': 'm', 'value': 1.0, 'a': None, 'b': None}\n"
+        "c = bench.ContextLines(line, 0, %s)\n"
+        "c.section('a', lambda: 1 / 0)\n"
+        "c.section('b', lambda: {'ok': 1})\n"
+        "%s\n"
+        "c.finish()\n"
+    )
+    out = subprocess.run([sys.executable, "-c", prog % (root, "30", "")], capture_output=True, text=True, timeout=60)
+    assert out.returncode == 0, out.stderr
+    line = json.loads(out.stdout.strip().splitlines()[-1])
+    assert line["value"] == 1.0 and "ZeroDivisionError" in line["a"]["error"] and line["b"] == {"ok": 1}
+    assert "context_note" not in line
+    hang = "c.section('c', lambda: time.sleep(60))"
+    out = subprocess.run([sys.executable, "-c", prog % (root, "1", hang)], capture_output=True, text=True, timeout=60)
+    assert out.returncode == 0, out.stderr
+    line = json.loads(out.stdout.strip().splitlines()[-1])
+    assert line["value"] == 1.0 and "stopped after 1 s" in line["context_note"] and "c" not in line
