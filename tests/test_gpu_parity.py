@@ -3,6 +3,7 @@
 All work is integer, so every comparison is exact (bit-exact fitness values, ranks and whole
 trajectories). Inputs are the seeded planted instances of ppp_inputs.
 """
+import os
 from math import comb
 
 import numpy as np
@@ -473,6 +474,32 @@ def test_batched_two_phase_schedule(L, orc, cfg, R, iters):
         V0 = pi.start_vector(inst.n, pi.restart_seed(seed, r))
         _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, c["k"], V0, iters, ten, stop_on_zero=False)
         assert batch[r] == ores, r
+        assert np.array_equal(Vo[r], oVo), r
+
+
+def test_bench_job_full_size_sampled_runs(L, orc):
+    """The bench's timed job exactly as bench.py launches it (C4, 50 searches x 400 iterations,
+    tenure floor(M/6), start vectors of bench step 3 from device memory, the two-phase schedule):
+    sampled runs of both phases -- final result and final vector -- equal the oracle run for the
+    full 400 iterations."""
+    import sys
+
+    import torch
+
+    sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+    import bench
+
+    inst = pi.config_instance(bench.CFG)
+    ten = pi.default_tenure(inst.n, 3)
+    step = 3  # the first timed step of a default run (warm-up 3)
+    V0 = bench.start_vectors(inst.n, step, range(bench.RUNS))
+    with L.Instance(inst.A, inst.S) as I:
+        Vo = torch.empty((bench.RUNS, inst.n), dtype=torch.int8, device="cuda")
+        res = L.lns_tabu_run_batch(I.ctx, 3, bench.RUNS, bench.ITERS, ten, 0, torch.from_numpy(V0).cuda(), 0, Vo)
+        Vo = Vo.cpu().numpy()
+    for r in (0, 1, 25, bench.RUNS - 1):
+        _, _, oVo, ores = orc.tabu_run(inst.A, inst.S, 3, V0[r], bench.ITERS, ten, stop_on_zero=False)
+        assert res[r] == ores, r
         assert np.array_equal(Vo[r], oVo), r
 
 
