@@ -516,7 +516,7 @@ def main():
         "e2e": {"value": e2e_value, "unit": UNIT, "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
                 "tabu_iters_per_s": e2e_iters / (e2e_ms / 1e3)},
         "single_search": None, "partitioned": None, "c5_single_search": None, "c5_restarts": None,
-        "ubqp_single_search": None,
+        "ubqp_single_search": None, "ubqp_restarts": None,
         # our kernels per timed step: k_init_slots + the persistent k_search
         "gpu_launches": args.steps * 2,
         "clocks": clocks,
@@ -658,6 +658,33 @@ def main():
 
     if world == 1 and not args.no_ubqp:
         section("ubqp_single_search", ubqp_single)
+
+    # ---- UBQP restarts side by side (lns_bqp_tabu_run_batch): the quality
+    #      protocol's shape, 50 starts of n = 200, k = 3 (N = 1 only; context)
+    def ubqp_restarts():
+        from ppp_inputs import bqp as bi
+
+        nq, kq, Rq, itq = 200, 3, 50, 256
+        Qb = bi.random_q(nq, 0.1, 1000)
+        X0 = np.stack([bi.start_x(nq, 100 + r) for r in range(Rq)])
+        cq = L.lns_bqp_create(Qb, 0)
+        L.lns_bqp_tabu_run_batch(cq, kq, X0, 128)
+        msq = []
+        for _ in range(2):
+            flush.fill_(0)
+            torch.cuda.synchronize()
+            L.lns_bqp_tabu_run_batch(cq, kq, X0, itq)
+            msq.append(L.lns_bqp_last_kernel_ms(cq))
+        L.lns_bqp_destroy(cq)
+        bq = min(msq)
+        Mq = L.lns_neighborhood_size(nq, kq)
+        return {"neighbors_per_s": Rq * itq * Mq / (bq / 1e3), "tabu_iters_per_s": Rq * itq / (bq / 1e3),
+                "restarts": Rq, "iters": itq,
+                "note": "UBQP n = 200, density 0.1, 3-Hamming, 50 restarts in one batched call (one grid row per "
+                        "restart); device time"}
+
+    if world == 1 and not args.no_ubqp:
+        section("ubqp_restarts", ubqp_restarts)
 
     def cpu_baseline():
         v, ips, it, runs, cores, dt = oracle_sample(args.cpu_budget)

@@ -298,6 +298,18 @@ lns_status lns_bqp_tabu_run(lns_bqp *ctx, int32_t k, int64_t iters, int64_t tenu
                             uint8_t *x_out, int64_t *trace_rank, int64_t *trace_fit, int64_t *res,
                             void *stream);
 
+/* lns_bqp_tabu_run_batch -- R independent searches of `iters` iterations each, run side by side
+ *   (restart r from x0s + r n; the paper's protocol runs every configuration 50 times, PAPER.md:
+ *   249-252): every iteration evaluates all R neighbourhoods in one launch (grid row r = restart r)
+ *   and applies the R moves in one launch, replayed from a CUDA graph. Each restart follows exactly
+ *   the trajectory lns_bqp_tabu_run gives from the same start. x0s: (host|device) R x n uint8 0/1;
+ *   x_outs: nullable (host|device) R x n uint8; res (host) R x 4 int64, row r as res of
+ *   lns_bqp_tabu_run. R in [1, 65535]; device memory R x C(n,k) x 4 bytes for the tabu lists.
+ *   Synchronous (ordered after `stream`). Errors: as lns_bqp_tabu_run; EINVAL also for R < 1,
+ *   ERANGE for R > 65535, ENOMEM when the R tabu lists do not fit. */
+lns_status lns_bqp_tabu_run_batch(lns_bqp *ctx, int32_t k, int32_t R, int64_t iters, int64_t tenure,
+                                  const uint8_t *x0s, uint8_t *x_outs, int64_t *res, void *stream);
+
 /* lns_bqp_last_kernel_ms -- device time (CUDA events) of the last eval_all / tabu_run (-1: NULL). */
 double lns_bqp_last_kernel_ms(const lns_bqp *ctx);
 

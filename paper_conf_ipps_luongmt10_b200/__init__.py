@@ -89,6 +89,7 @@ _SIGS = {
     "lns_bqp_destroy": (None, [_vp]),
     "lns_bqp_eval_all": (_i32, [_vp, _i32, _vp, _vp, _vp]),
     "lns_bqp_tabu_run": (_i32, [_vp, _i32, _i64, _i64, _vp, _vp, _vp, _vp, _vp, _vp]),
+    "lns_bqp_tabu_run_batch": (_i32, [_vp, _i32, _i32, _i64, _i64, _vp, _vp, _vp, _vp]),
     "lns_bqp_last_kernel_ms": (ctypes.c_double, [_vp]),
 }
 
@@ -424,6 +425,17 @@ def lns_bqp_tabu_run(ctx: int, k: int, iters: int, tenure: int = -1, x0=None, x_
     d = dict(zip(BQP_RESULT_FIELDS, (int(v) for v in res)))
     it = d["iters_done"]
     return (None if tr is None else tr[:it].copy()), (None if tf is None else tf[:it].copy()), x_out, d
+
+
+def lns_bqp_tabu_run_batch(ctx: int, k: int, x0s, iters: int, tenure: int = -1, x_outs=None, stream=None):
+    """R = len(x0s) independent tabu searches run side by side (x0s: R x n uint8 0/1); returns one
+    result dict per restart (the fields of lns_bqp_tabu_run); x_outs (R x n) receives the final x."""
+    R = int(tuple(x0s.shape)[0])
+    px, kx = _ptr(x0s, np.uint8)
+    res = np.zeros((max(R, 1), 4), dtype=np.int64)
+    _check(load().lns_bqp_tabu_run_batch(ctx, k, R, iters, tenure, px, _out_ptr(x_outs, np.uint8),
+                                         res.ctypes.data, _stream(stream)), "lns_bqp_tabu_run_batch")
+    return [dict(zip(BQP_RESULT_FIELDS, (int(v) for v in row))) for row in res[:R]]
 
 
 def lns_bqp_last_kernel_ms(ctx: int) -> float:

@@ -87,10 +87,13 @@ __device__ __forceinline__ unsigned long long bq_key(int32_t f, uint32_t r)
 }
 
 // g = Q x, f = x^T g, state reset; x entries must be 0 or 1.
+// Batched restarts (lns_bqp_tabu_run_batch): CTA r (init, apply) / grid row blockIdx.y = r (eval)
+// works on restart r's slice of x, g, st, until and key; a single search is the grid of one row.
 __global__ void __launch_bounds__(BQ_AT) k_bqp_init(const int32_t *__restrict__ Q, int n,
                                                     const uint8_t *__restrict__ x, int32_t *__restrict__ g,
                                                     int64_t *st)
 {
+    x += (size_t)blockIdx.x * n; g += (size_t)blockIdx.x * n; st += (size_t)blockIdx.x * BS_N;
     __shared__ unsigned long long s_f;
     __shared__ int s_bad;
     if (threadIdx.x == 0) { s_f = 0; s_bad = 0; }
@@ -122,7 +125,9 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     extern __shared__ int32_t s_h[];  // h_i = 2 d_i g_i + Q_ii, then d_i (n + n ints)
     int32_t *s_d = s_h + n;
     __shared__ unsigned long long s_key;
-    if (st[BS_ERR]) return;  // uniform over the grid
+    x += (size_t)blockIdx.y * n; g += (size_t)blockIdx.y * n; st += (size_t)blockIdx.y * BS_N; key += blockIdx.y;
+    if (until) until += (size_t)blockIdx.y * M;
+    if (st[BS_ERR]) return;  // uniform over the grid row
     for (int i = threadIdx.x; i < n; i += blockDim.x) {
         const int d = 1 - 2 * (int)x[i];
         s_d[i] = d;
@@ -190,6 +195,8 @@ __global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__
                                                      int64_t L, unsigned long long *key, int64_t *trace_r,
                                                      int64_t *trace_f)
 {
+    x += (size_t)blockIdx.x * n; g += (size_t)blockIdx.x * n; st += (size_t)blockIdx.x * BS_N; key += blockIdx.x;
+    until += (size_t)blockIdx.x * M;
     if (st[BS_ERR]) return;
     const unsigned long long kv = *key;
     if (kv == BQ_NONE) {
@@ -231,6 +238,12 @@ struct lns_bqp {
     uint32_t *d_until = nullptr;
     unsigned long long *d_key = nullptr;
     size_t fit_cap = 0, until_cap = 0, tr_cap = 0;
+    // batched restarts: R slices of x, g, state, key (until[] shares d_until: R x M entries)
+    uint8_t *d_bx = nullptr;
+    int32_t *d_bg = nullptr;
+    int64_t *d_bst = nullptr;
+    unsigned long long *d_bkey = nullptr;
+    size_t bx_cap = 0, bg_cap = 0, bst_cap = 0, bkey_cap = 0;
     cudaStream_t st = nullptr;
     cudaEvent_t ev0 = nullptr, ev1 = nullptr, evu = nullptr;
     float last_ms = 0;
@@ -254,28 +267,83 @@ int bqp_blocks(const lns_bqp *c, uint64_t M)
     return (int)std::max<uint64_t>(1, std::min<uint64_t>(want, (uint64_t)c->nsm * 8));
 }
 
-lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, const uint32_t *until, int32_t *fit)
+// The buffers one launch works on: a single search (the context's own) or R batched restarts.
+struct BqBufs {
+    uint8_t *x;
+    int32_t *g;
+    int64_t *st;
+    unsigned long long *key;
+    uint32_t *until;
+    int R;
+};
+
+BqBufs bq_single(lns_bqp *c) { return BqBufs{c->d_x, c->d_g, c->d_st, c->d_key, c->d_until, 1}; }
+
+lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, const BqBufs &b, const uint32_t *until, int32_t *fit)
 {
-    const int nb = bqp_blocks(c, M);
+    // one grid row per restart; R rows share the SMs (about 8 CTAs per SM in total)
+    const int nb = b.R == 1 ? bqp_blocks(c, M)
+                            : (int)std::max<uint64_t>(1, std::min<uint64_t>((M + BQ_NT - 1) / BQ_NT,
+                                                                            ((uint64_t)c->nsm * 8 + b.R - 1) / b.R));
+    const dim3 grid(nb, b.R);
     const size_t sm = 2 * sizeof(int32_t) * (size_t)c->n;
     switch (k) {
-    case 1: k_bqp_eval<1><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
-    case 2: k_bqp_eval<2><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
-    default: k_bqp_eval<3><<<nb, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, until, fit, c->d_key); break;
+    case 1: k_bqp_eval<1><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
+    case 2: k_bqp_eval<2><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
+    default: k_bqp_eval<3><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
     }
     CK(cudaGetLastError());
     return LNS_OK;
 }
 
-lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, int64_t L, bool trace)
+lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, int64_t L, const BqBufs &b, bool trace)
 {
     int64_t *tr = trace ? c->d_tr : nullptr, *tf = trace ? c->d_tf : nullptr;
     switch (k) {
-    case 1: k_bqp_apply<1><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
-    case 2: k_bqp_apply<2><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
-    default: k_bqp_apply<3><<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, c->d_x, c->d_g, c->d_st, c->d_until, L, c->d_key, tr, tf); break;
+    case 1: k_bqp_apply<1><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
+    case 2: k_bqp_apply<2><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
+    default: k_bqp_apply<3><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
     }
     CK(cudaGetLastError());
+    return LNS_OK;
+}
+
+// `iters` iterations of eval + apply on b: blocks of G = min(iters, 64) iterations captured once
+// into a CUDA graph and replayed (every launch reads the iteration number from the device state),
+// the remainder launched directly; ev0 is recorded after the graph is built (host work).
+lns_status bqp_iterate(lns_bqp *c, int k, uint64_t M, int64_t L, int64_t iters, const BqBufs &b, bool trace)
+{
+    lns_status s;
+    const int64_t G = std::min<int64_t>(iters, 64);
+    int64_t done = 0;
+    bool timing_started = false;
+    if (G > 0 && iters / G >= 2) {
+        cudaGraph_t graph = nullptr;
+        cudaGraphExec_t exec = nullptr;
+        CK(cudaStreamBeginCapture(c->st, cudaStreamCaptureModeThreadLocal));
+        for (int64_t q = 0; q < G; q++) {
+            lns_status e1 = bqp_launch_eval(c, k, M, b, b.until, nullptr);
+            lns_status e2 = e1 == LNS_OK ? bqp_launch_apply(c, k, M, L, b, trace) : e1;
+            if (e2 != LNS_OK) { cudaStreamEndCapture(c->st, &graph); if (graph) cudaGraphDestroy(graph); return e2; }
+        }
+        CK(cudaStreamEndCapture(c->st, &graph));
+        cudaError_t e = cudaGraphInstantiate(&exec, graph, 0);
+        cudaGraphDestroy(graph);
+        if (e != cudaSuccess) return fail(LNS_ECUDA, std::string("cudaGraphInstantiate: ") + cudaGetErrorString(e));
+        CK(cudaEventRecord(c->ev0, c->st));
+        timing_started = true;
+        for (; done + G <= iters; done += G) {
+            e = cudaGraphLaunch(exec, c->st);
+            if (e != cudaSuccess) { cudaGraphExecDestroy(exec); return fail(LNS_ECUDA, cudaGetErrorString(e)); }
+        }
+        cudaGraphExecDestroy(exec);
+    }
+    if (!timing_started) CK(cudaEventRecord(c->ev0, c->st));
+    for (; done < iters; done++) {
+        if ((s = bqp_launch_eval(c, k, M, b, b.until, nullptr)) != LNS_OK) return s;
+        if ((s = bqp_launch_apply(c, k, M, L, b, trace)) != LNS_OK) return s;
+    }
+    CK(cudaEventRecord(c->ev1, c->st));
     return LNS_OK;
 }
 
@@ -287,13 +355,12 @@ lns_status bqp_enter(lns_bqp *c, void *stream)
     return LNS_OK;
 }
 
-lns_status bqp_start(lns_bqp *c, const uint8_t *x)
+lns_status bqp_start(lns_bqp *c, const uint8_t *x, const BqBufs &b)
 {
-    CK(cudaMemcpyAsync(c->d_x, x, (size_t)c->n, cudaMemcpyDefault, c->st));
-    k_bqp_init<<<1, BQ_AT, 0, c->st>>>(c->d_Q, c->n, c->d_x, c->d_g, c->d_st);
+    CK(cudaMemcpyAsync(b.x, x, (size_t)c->n * b.R, cudaMemcpyDefault, c->st));
+    k_bqp_init<<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, b.x, b.g, b.st);
     CK(cudaGetLastError());
-    const unsigned long long none = BQ_NONE;
-    CK(cudaMemcpyAsync(c->d_key, &none, sizeof(none), cudaMemcpyHostToDevice, c->st));
+    CK(cudaMemsetAsync(b.key, 0xff, sizeof(unsigned long long) * b.R, c->st));  // BQ_NONE = all ones
     return LNS_OK;
 }
 
@@ -355,6 +422,7 @@ void lns_bqp_destroy(lns_bqp *c)
     if (c->st) cudaStreamSynchronize(c->st);
     pool_free(c->d_Q); pool_free(c->d_g); pool_free(c->d_x); pool_free(c->d_st); pool_free(c->d_key);
     pool_free(c->d_fit); pool_free(c->d_until); pool_free(c->d_tr); pool_free(c->d_tf);
+    pool_free(c->d_bx); pool_free(c->d_bg); pool_free(c->d_bst); pool_free(c->d_bkey);
     if (c->ev0) cudaEventDestroy(c->ev0);
     if (c->ev1) cudaEventDestroy(c->ev1);
     if (c->evu) cudaEventDestroy(c->evu);
@@ -371,9 +439,9 @@ lns_status lns_bqp_eval_all(lns_bqp *c, int32_t k, const uint8_t *x, int32_t *fi
     DeviceGuard dg(c->device);
     if ((s = grow(c->d_fit, c->fit_cap, M)) != LNS_OK) return s;
     if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
-    if ((s = bqp_start(c, x)) != LNS_OK) return s;
+    if ((s = bqp_start(c, x, bq_single(c))) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev0, c->st));
-    if ((s = bqp_launch_eval(c, k, M, nullptr, c->d_fit)) != LNS_OK) return s;
+    if ((s = bqp_launch_eval(c, k, M, bq_single(c), nullptr, c->d_fit)) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev1, c->st));
     int64_t hs[BS_N];
     CK(cudaMemcpyAsync(hs, c->d_st, sizeof(hs), cudaMemcpyDeviceToHost, c->st));
@@ -408,40 +476,8 @@ lns_status lns_bqp_tabu_run(lns_bqp *c, int32_t k, int64_t iters, int64_t tenure
     }
     if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
     CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * M, c->st));
-    if ((s = bqp_start(c, x0)) != LNS_OK) return s;
-    // Every launch reads the iteration number from the device state, so a block of G iterations
-    // is captured once into a CUDA graph and replayed (no host round trip per iteration).
-    const int64_t G = std::min<int64_t>(iters, 64);
-    int64_t done = 0;
-    bool timing_started = false;
-    if (G > 0 && iters / G >= 2) {
-        cudaGraph_t graph = nullptr;
-        cudaGraphExec_t exec = nullptr;
-        CK(cudaStreamBeginCapture(c->st, cudaStreamCaptureModeThreadLocal));
-        for (int64_t q = 0; q < G; q++) {
-            lns_status e1 = bqp_launch_eval(c, k, M, c->d_until, nullptr);
-            lns_status e2 = e1 == LNS_OK ? bqp_launch_apply(c, k, M, L, trace) : e1;
-            if (e2 != LNS_OK) { cudaStreamEndCapture(c->st, &graph); if (graph) cudaGraphDestroy(graph); return e2; }
-        }
-        CK(cudaStreamEndCapture(c->st, &graph));
-        cudaError_t e = cudaGraphInstantiate(&exec, graph, 0);
-        cudaGraphDestroy(graph);
-        if (e != cudaSuccess) return fail(LNS_ECUDA, std::string("cudaGraphInstantiate: ") + cudaGetErrorString(e));
-        // timed from here: the capture / instantiation above is host work, not search time
-        CK(cudaEventRecord(c->ev0, c->st));
-        timing_started = true;
-        for (; done + G <= iters; done += G) {
-            e = cudaGraphLaunch(exec, c->st);
-            if (e != cudaSuccess) { cudaGraphExecDestroy(exec); return fail(LNS_ECUDA, cudaGetErrorString(e)); }
-        }
-        cudaGraphExecDestroy(exec);
-    }
-    if (!timing_started) CK(cudaEventRecord(c->ev0, c->st));
-    for (; done < iters; done++) {
-        if ((s = bqp_launch_eval(c, k, M, c->d_until, nullptr)) != LNS_OK) return s;
-        if ((s = bqp_launch_apply(c, k, M, L, trace)) != LNS_OK) return s;
-    }
-    CK(cudaEventRecord(c->ev1, c->st));
+    if ((s = bqp_start(c, x0, bq_single(c))) != LNS_OK) return s;
+    if ((s = bqp_iterate(c, k, M, L, iters, bq_single(c), trace)) != LNS_OK) return s;
     int64_t hs[BS_N];
     CK(cudaMemcpyAsync(hs, c->d_st, sizeof(hs), cudaMemcpyDeviceToHost, c->st));
     if (x_out) CK(cudaMemcpyAsync(x_out, c->d_x, (size_t)c->n, cudaMemcpyDefault, c->st));
@@ -453,6 +489,47 @@ lns_status lns_bqp_tabu_run(lns_bqp *c, int32_t k, int64_t iters, int64_t tenure
     res[0] = nt; res[1] = hs[BS_F]; res[2] = hs[BS_BEST]; res[3] = hs[BS_BESTIT];
     if (hs[BS_ERR] == 1) return fail(LNS_EINVAL, "x0 must be 0/1");
     if (hs[BS_ERR] == 2) return fail(LNS_ENOADMISSIBLE, "every neighbour is tabu");
+    return LNS_OK;
+}
+
+lns_status lns_bqp_tabu_run_batch(lns_bqp *c, int32_t k, int32_t R, int64_t iters, int64_t tenure,
+                                  const uint8_t *x0s, uint8_t *x_outs, int64_t *res, void *stream)
+{
+    uint64_t M;
+    lns_status s = bqp_check_k(c, k, M);
+    if (s != LNS_OK) return s;
+    if (!x0s || !res) return fail(LNS_EINVAL, "null argument");
+    if (R < 1) return fail(LNS_EINVAL, "R must be >= 1");
+    if (R > 65535) return fail(LNS_ERANGE, "R > 65535 (grid rows)");
+    if (iters < 0 || iters >= ((int64_t)1 << 31)) return fail(LNS_EINVAL, "iters outside [0, 2^31)");
+    const int64_t L = tenure < 0 ? (int64_t)(M / 6) : tenure;
+    if ((uint64_t)L >= M) return fail(LNS_ERANGE, "tenure >= C(n,k)");
+    if (iters + L >= ((int64_t)1 << 32) - 1) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
+    DeviceGuard dg(c->device);
+    const size_t n = (size_t)c->n;
+    if ((s = grow(c->d_until, c->until_cap, M * (size_t)R)) != LNS_OK) return s;
+    if ((s = grow(c->d_bx, c->bx_cap, n * R)) != LNS_OK) return s;
+    if ((s = grow(c->d_bg, c->bg_cap, n * R)) != LNS_OK) return s;
+    if ((s = grow(c->d_bst, c->bst_cap, (size_t)BS_N * R)) != LNS_OK) return s;
+    if ((s = grow(c->d_bkey, c->bkey_cap, (size_t)R)) != LNS_OK) return s;
+    const BqBufs b{c->d_bx, c->d_bg, c->d_bst, c->d_bkey, c->d_until, R};
+    if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
+    CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * M * R, c->st));
+    if ((s = bqp_start(c, x0s, b)) != LNS_OK) return s;
+    if ((s = bqp_iterate(c, k, M, L, iters, b, false)) != LNS_OK) return s;
+    std::vector<int64_t> hs((size_t)BS_N * R);
+    CK(cudaMemcpyAsync(hs.data(), c->d_bst, sizeof(int64_t) * hs.size(), cudaMemcpyDeviceToHost, c->st));
+    if (x_outs) CK(cudaMemcpyAsync(x_outs, c->d_bx, n * R, cudaMemcpyDefault, c->st));
+    CK(cudaStreamSynchronize(c->st));
+    cudaEventElapsedTime(&c->last_ms, c->ev0, c->ev1);
+    int err = 0;
+    for (int r = 0; r < R; r++) {
+        const int64_t *h = hs.data() + (size_t)BS_N * r;
+        res[4 * r] = h[BS_T]; res[4 * r + 1] = h[BS_F]; res[4 * r + 2] = h[BS_BEST]; res[4 * r + 3] = h[BS_BESTIT];
+        if (h[BS_ERR] && !err) err = (int)h[BS_ERR];
+    }
+    if (err == 1) return fail(LNS_EINVAL, "x0s must be 0/1");
+    if (err == 2) return fail(LNS_ENOADMISSIBLE, "every neighbour is tabu");
     return LNS_OK;
 }
 

@@ -202,3 +202,53 @@ def test_errors(L):
         assert e.value.status == L.LNS_EINVAL
     finally:
         L.lns_bqp_destroy(tiny)
+
+
+@pytest.mark.parametrize("k,n,R,iters,tenure", [(1, 40, 7, 150, -1), (2, 33, 5, 130, 9), (2, 25, 1, 70, -1),
+                                                (3, 22, 12, 140, -1), (3, 18, 33, 40, 0), (3, 60, 4, 200, 300)])
+def test_batched_restarts_bit_exact(L, k, n, R, iters, tenure):
+    """lns_bqp_tabu_run_batch: every restart (one grid row each, graph blocks + remainder) ends where
+    the oracle's search from the same start ends: result fields and final x, restart by restart."""
+    Q = bi.random_q(n, 0.35, 70 + k + n)
+    X0 = np.stack([bi.start_x(n, 100 + r) for r in range(R)])
+    ctx = L.lns_bqp_create(Q, 0)
+    try:
+        Xo = np.empty_like(X0)
+        res = L.lns_bqp_tabu_run_batch(ctx, k, X0, iters, tenure, x_outs=Xo)
+        # the context's single-search state is untouched by a batch (and vice versa)
+        _, _, xo1, res1 = L.lns_bqp_tabu_run(ctx, k, iters, tenure, X0[R - 1])
+    finally:
+        L.lns_bqp_destroy(ctx)
+    for r in range(R):
+        _, _, oxo, ores = bqp.tabu_run(Q, X0[r], k, iters, tenure)
+        assert res[r] == ores, r
+        assert np.array_equal(Xo[r], oxo), r
+    assert res1 == res[R - 1] and np.array_equal(xo1, Xo[R - 1])
+
+
+def test_batched_restarts_device_buffers_and_errors(L):
+    import torch
+
+    n, k, R = 30, 3, 6
+    Q = bi.random_q(n, 0.3, 9)
+    X0 = np.stack([bi.start_x(n, 7 + r) for r in range(R)])
+    ctx = L.lns_bqp_create(Q, 0)
+    try:
+        Xo = torch.empty((R, n), dtype=torch.uint8, device="cuda")
+        res = L.lns_bqp_tabu_run_batch(ctx, k, torch.from_numpy(X0).cuda(), 90, -1, x_outs=Xo)
+        for r in (0, R - 1):
+            _, _, oxo, ores = bqp.tabu_run(Q, X0[r], k, 90, -1)
+            assert res[r] == ores and np.array_equal(Xo[r].cpu().numpy(), oxo)
+        bad = X0.copy()
+        bad[2, 5] = 3
+        with pytest.raises(L.LnsError) as e:
+            L.lns_bqp_tabu_run_batch(ctx, k, bad, 10)
+        assert e.value.status == L.LNS_EINVAL
+        with pytest.raises(L.LnsError) as e:
+            L.lns_bqp_tabu_run_batch(ctx, k, X0, 10, comb(n, k))
+        assert e.value.status == L.LNS_ERANGE
+        with pytest.raises(L.LnsError) as e:
+            L.lns_bqp_tabu_run_batch(ctx, k, X0[:0], 10)
+        assert e.value.status == L.LNS_EINVAL
+    finally:
+        L.lns_bqp_destroy(ctx)
