@@ -150,36 +150,59 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     if (lo < hi) {
         int idx[K];
         bq_unrank<K>(lo, n, M, idx);
-        // The prefix F \ {c} (all but the last index) changes only when the run wraps: its part of
-        // the delta (pre), its signs and its Q rows are kept in registers.
-        // Modular (u32) sums: every term fits int32 and so does f0 + delta (|f| <= sum |Q_ij| < 2^29),
-        // so the wrapped total is exact.
+        // Flip set (a, b, c) in registers (c = the last index; (a, b) the prefix, k = 3; a alone,
+        // k = 2). The prefix F \ {c} changes only when the run wraps: its part of the delta (pre),
+        // its signs and its Q rows are kept in registers. Modular (u32) sums: every term fits int32
+        // and so does f0 + delta (|f| <= sum |Q_ij| < 2^29), so the wrapped total is exact.
+        int a = K >= 2 ? idx[0] : 0, b = K == 3 ? idx[1] : 0, c = idx[K - 1];
         uint32_t pre = 0;
         int dp0 = 0, dp1 = 0;
         const int32_t *q0 = Q, *q1 = Q;
         auto load_prefix = [&]() {
-            if (K >= 2) { dp0 = s_d[idx[0]]; q0 = Q + (size_t)idx[0] * n; pre = (uint32_t)s_h[idx[0]]; }
+            if (K >= 2) { dp0 = s_d[a]; q0 = Q + (size_t)a * n; pre = (uint32_t)s_h[a]; }
             if (K == 3) {
-                dp1 = s_d[idx[1]]; q1 = Q + (size_t)idx[1] * n;
-                pre += (uint32_t)s_h[idx[1]] + (uint32_t)(2 * dp0 * dp1 * q0[idx[1]]);
+                dp1 = s_d[b]; q1 = Q + (size_t)b * n;
+                pre += (uint32_t)s_h[b] + (uint32_t)(2 * dp0 * dp1 * q0[b]);
             }
         };
         load_prefix();
+        // least admissible (biased fitness, rank) of this lane: ranks only grow along the run, so a
+        // strict "<" on the fitness keeps the lowest rank among equal fitnesses (reading R5)
+        uint32_t bf = 0xffffffffu, br = 0xffffffffu;
+        const uint32_t rhi = (uint32_t)hi;
+        const uint32_t *up = until ? until + lo : nullptr;  // until[r], advanced with r
         for (uint32_t r = (uint32_t)lo;;) {
-            const int c = idx[K - 1];
             uint32_t delta = pre + (uint32_t)s_h[c];
             if (K >= 2) {
                 const int dc2 = 2 * s_d[c];
                 delta += (uint32_t)(dc2 * dp0 * q0[c]);
                 if (K == 3) delta += (uint32_t)(dc2 * dp1 * q1[c]);
             }
-            const int32_t fr = (int32_t)((uint32_t)f0 + delta);
-            if (fit_out) fit_out[r] = fr;
-            if (!until || until[r] < t) best = min(best, bq_key(fr, r));
-            if ((uint64_t)r + 32 >= hi) break;
-            r += 32;
-            if (bq_advance<K>(n, idx, 32)) load_prefix();
+            const uint32_t fr = (uint32_t)f0 + delta;
+            if (fit_out) fit_out[r] = (int32_t)fr;
+            const uint32_t fb = fr ^ 0x80000000u;  // order-preserving for signed f
+            if ((!up || *up < t) && fb < bf) { bf = fb; br = r; }
+            if (rhi - r <= 32u) break;
+            r += 32u;
+            if (up) up += 32;
+            c += 32;
+            if (K >= 2 && c >= n) {
+                // the run passes the end of its prefix: the prefix takes its successor (a
+                // (k-1)-subset of [0, n - 2]) and the overshoot restarts after it
+                do {
+                    const int over = c - n;
+                    if (K == 2) {
+                        ++a;
+                        c = a + 1 + over;
+                    } else {
+                        if (b < n - 2) ++b; else { ++a; b = a + 1; }
+                        c = b + 1 + over;
+                    }
+                } while (c >= n);
+                load_prefix();
+            }
         }
+        if (br != 0xffffffffu) best = ((unsigned long long)bf << 32) | br;
     }
     best = warp_min_k(best);
     if ((threadIdx.x & 31) == 0 && best != BQ_NONE) atomicMin(&s_key, best);

@@ -1,8 +1,11 @@
 """Time the UBQP tabu search on a few shapes: device time of lns_bqp_tabu_run."""
+import os
+import sys
 from math import comb
 
-import paper_conf_ipps_luongmt10_b200 as L
-from ppp_inputs import bqp as bi
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import paper_conf_ipps_luongmt10_b200 as L  # noqa: E402
+from ppp_inputs import bqp as bi  # noqa: E402
 
 for k, n, dens, iters in [(1, 2500, 0.1, 2000), (2, 500, 0.1, 1000), (2, 2500, 0.1, 100), (3, 117, 0.1, 1000),
                           (3, 250, 0.1, 200), (3, 500, 0.1, 50)]:
