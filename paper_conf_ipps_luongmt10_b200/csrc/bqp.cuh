@@ -114,19 +114,24 @@ __global__ void __launch_bounds__(BQ_AT) k_bqp_init(const int32_t *__restrict__ 
     }
 }
 
+// Tabu state of one search (reading R3: the FIFO of the last L accepted ranks), `S` words per
+// restart: a bitmap of ceil(M/32) words (bit r set <=> rank r is tabu) followed by a ring of L
+// ranks (slot (s - 1) mod L = the rank accepted at iteration s). The same list as an until[] array
+// with until[r] = (iteration accepted) + L, at 1/32 of its memory traffic.
+
 // Every neighbour of iteration t = st[T] + 1: fitness (fit_out, optional) and the least admissible
-// key (until[r] < t; until == nullptr: all admissible) MIN-reduced into *key.
+// key (tabu bit clear; tabu == nullptr: all admissible) MIN-reduced into *key.
 template <int K>
 __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ Q, int n, uint64_t M,
                                                     const uint8_t *__restrict__ x, const int32_t *__restrict__ g,
-                                                    const int64_t *__restrict__ st, const uint32_t *__restrict__ until,
-                                                    int32_t *__restrict__ fit_out, unsigned long long *key)
+                                                    const int64_t *__restrict__ st, const uint32_t *__restrict__ tabu,
+                                                    uint64_t S, int32_t *__restrict__ fit_out, unsigned long long *key)
 {
     extern __shared__ int32_t s_h[];  // h_i = 2 d_i g_i + Q_ii, then d_i (n + n ints)
     int32_t *s_d = s_h + n;
     __shared__ unsigned long long s_key;
     x += (size_t)blockIdx.y * n; g += (size_t)blockIdx.y * n; st += (size_t)blockIdx.y * BS_N; key += blockIdx.y;
-    if (until) until += (size_t)blockIdx.y * M;
+    if (tabu) tabu += (size_t)blockIdx.y * S;
     if (st[BS_ERR]) return;  // uniform over the grid row
     for (int i = threadIdx.x; i < n; i += blockDim.x) {
         const int d = 1 - 2 * (int)x[i];
@@ -136,10 +141,9 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     if (threadIdx.x == 0) s_key = BQ_NONE;
     __syncthreads();
     const int32_t f0 = (int32_t)st[BS_F];
-    const uint32_t t = (uint32_t)(st[BS_T] + 1);
     // Warp-interleaved ranks: warp w owns [32 w per, 32 (w + 1) per) and lane l takes ranks
-    // base + l + 32 j, so consecutive lanes hold consecutive ranks: until[] and fit_out are
-    // coalesced, and (last index fastest) the Q row reads Q[a n + c], Q[b n + c] and the h[c], d[c]
+    // base + l + 32 j, so consecutive lanes hold consecutive ranks: the 32 ranks of a step are one
+    // bitmap word (bit = lane), fit_out is coalesced, and (last index fastest) the Q row reads Q[a n + c], Q[b n + c] and the h[c], d[c]
     // table reads hit consecutive addresses across the warp.
     const uint64_t T = (uint64_t)gridDim.x * blockDim.x;
     const uint64_t per = (M + T - 1) / T;
@@ -170,7 +174,8 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
         // strict "<" on the fitness keeps the lowest rank among equal fitnesses (reading R5)
         uint32_t bf = 0xffffffffu, br = 0xffffffffu;
         const uint32_t rhi = (uint32_t)hi;
-        const uint32_t *up = until ? until + lo : nullptr;  // until[r], advanced with r
+        const uint32_t *wp = tabu ? tabu + (lo >> 5) : nullptr;  // bitmap word of r, advanced with r
+        const unsigned lane = threadIdx.x & 31;
         for (uint32_t r = (uint32_t)lo;;) {
             uint32_t delta = pre + (uint32_t)s_h[c];
             if (K >= 2) {
@@ -181,10 +186,10 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
             const uint32_t fr = (uint32_t)f0 + delta;
             if (fit_out) fit_out[r] = (int32_t)fr;
             const uint32_t fb = fr ^ 0x80000000u;  // order-preserving for signed f
-            if ((!up || *up < t) && fb < bf) { bf = fb; br = r; }
+            if ((!wp || !((*wp >> lane) & 1u)) && fb < bf) { bf = fb; br = r; }
             if (rhi - r <= 32u) break;
             r += 32u;
-            if (up) up += 32;
+            if (wp) ++wp;
             c += 32;
             if (K >= 2 && c >= n) {
                 // the run passes the end of its prefix: the prefix takes its successor (a
@@ -210,16 +215,17 @@ __global__ void __launch_bounds__(BQ_NT) k_bqp_eval(const int32_t *__restrict__ 
     if (threadIdx.x == 0 && s_key != BQ_NONE) atomicMin(key, s_key);
 }
 
-// Apply the winning move of iteration t = st[T] + 1: x ^= F, g += sum_{i in F} d_i Q_i., until[r] =
-// t + L, trace, best; *key reset for the next iteration. One CTA.
+// Apply the winning move of iteration t = st[T] + 1: x ^= F, g += sum_{i in F} d_i Q_i., the tabu
+// list (the rank accepted at t - L leaves, r enters), trace, best; *key reset for the next
+// iteration. One CTA per search.
 template <int K>
 __global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__ Q, int n, uint64_t M,
-                                                     uint8_t *x, int32_t *g, int64_t *st, uint32_t *until,
-                                                     int64_t L, unsigned long long *key, int64_t *trace_r,
-                                                     int64_t *trace_f)
+                                                     uint8_t *x, int32_t *g, int64_t *st, uint32_t *tabu,
+                                                     uint64_t S, int64_t L, unsigned long long *key,
+                                                     int64_t *trace_r, int64_t *trace_f)
 {
     x += (size_t)blockIdx.x * n; g += (size_t)blockIdx.x * n; st += (size_t)blockIdx.x * BS_N; key += blockIdx.x;
-    until += (size_t)blockIdx.x * M;
+    tabu += (size_t)blockIdx.x * S;
     if (st[BS_ERR]) return;
     const unsigned long long kv = *key;
     if (kv == BQ_NONE) {
@@ -243,7 +249,18 @@ __global__ void __launch_bounds__(BQ_AT) k_bqp_apply(const int32_t *__restrict__
 #pragma unroll
         for (int q = 0; q < K; q++) x[idx[q]] ^= 1;
         const int64_t t = st[BS_T] + 1;
-        until[r] = (uint32_t)(t + L);
+        if (L > 0) {
+            // tabu at iteration t' <=> accepted at t' - L .. t' - 1: for t + 1 the rank of t - L
+            // leaves (it was tabu through t, so it is not r) and r enters; one writer per search
+            uint32_t *ring = tabu + (M + 31) / 32;
+            const size_t slot = (size_t)((t - 1) % L);
+            if (t > L) {
+                const uint32_t e = ring[slot];
+                tabu[e >> 5] &= ~(1u << (e & 31));
+            }
+            tabu[r >> 5] |= 1u << (r & 31);
+            ring[slot] = r;
+        }
         if (trace_r) { trace_r[t - 1] = r; trace_f[t - 1] = f; }
         st[BS_F] = f; st[BS_T] = t;
         if (f < st[BS_BEST]) { st[BS_BEST] = f; st[BS_BESTIT] = t; }
@@ -258,10 +275,10 @@ struct lns_bqp {
     int32_t *d_Q = nullptr, *d_g = nullptr, *d_fit = nullptr;
     uint8_t *d_x = nullptr;
     int64_t *d_st = nullptr, *d_tr = nullptr, *d_tf = nullptr;
-    uint32_t *d_until = nullptr;
+    uint32_t *d_until = nullptr;  // tabu state(s): bitmap + ring per search (bq_tabu_words)
     unsigned long long *d_key = nullptr;
     size_t fit_cap = 0, until_cap = 0, tr_cap = 0;
-    // batched restarts: R slices of x, g, state, key (until[] shares d_until: R x M entries)
+    // batched restarts: R slices of x, g, state, key (the tabu states share d_until: R x S words)
     uint8_t *d_bx = nullptr;
     int32_t *d_bg = nullptr;
     int64_t *d_bst = nullptr;
@@ -290,6 +307,9 @@ int bqp_blocks(const lns_bqp *c, uint64_t M)
     return (int)std::max<uint64_t>(1, std::min<uint64_t>(want, (uint64_t)c->nsm * 8));
 }
 
+// 32-bit words of one search's tabu state: the bitmap and the ring of L ranks.
+inline uint64_t bq_tabu_words(uint64_t M, int64_t L) { return (M + 31) / 32 + (uint64_t)L; }
+
 // The buffers one launch works on: a single search (the context's own) or R batched restarts.
 struct BqBufs {
     uint8_t *x;
@@ -302,7 +322,7 @@ struct BqBufs {
 
 BqBufs bq_single(lns_bqp *c) { return BqBufs{c->d_x, c->d_g, c->d_st, c->d_key, c->d_until, 1}; }
 
-lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, const BqBufs &b, const uint32_t *until, int32_t *fit)
+lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, uint64_t S, const BqBufs &b, const uint32_t *tabu, int32_t *fit)
 {
     // one grid row per restart; R rows share the SMs (about 8 CTAs per SM in total)
     const int nb = b.R == 1 ? bqp_blocks(c, M)
@@ -311,21 +331,21 @@ lns_status bqp_launch_eval(lns_bqp *c, int k, uint64_t M, const BqBufs &b, const
     const dim3 grid(nb, b.R);
     const size_t sm = 2 * sizeof(int32_t) * (size_t)c->n;
     switch (k) {
-    case 1: k_bqp_eval<1><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
-    case 2: k_bqp_eval<2><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
-    default: k_bqp_eval<3><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, until, fit, b.key); break;
+    case 1: k_bqp_eval<1><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, tabu, S, fit, b.key); break;
+    case 2: k_bqp_eval<2><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, tabu, S, fit, b.key); break;
+    default: k_bqp_eval<3><<<grid, BQ_NT, sm, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, tabu, S, fit, b.key); break;
     }
     CK(cudaGetLastError());
     return LNS_OK;
 }
 
-lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, int64_t L, const BqBufs &b, bool trace)
+lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, uint64_t S, int64_t L, const BqBufs &b, bool trace)
 {
     int64_t *tr = trace ? c->d_tr : nullptr, *tf = trace ? c->d_tf : nullptr;
     switch (k) {
-    case 1: k_bqp_apply<1><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
-    case 2: k_bqp_apply<2><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
-    default: k_bqp_apply<3><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, L, b.key, tr, tf); break;
+    case 1: k_bqp_apply<1><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, S, L, b.key, tr, tf); break;
+    case 2: k_bqp_apply<2><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, S, L, b.key, tr, tf); break;
+    default: k_bqp_apply<3><<<b.R, BQ_AT, 0, c->st>>>(c->d_Q, c->n, M, b.x, b.g, b.st, b.until, S, L, b.key, tr, tf); break;
     }
     CK(cudaGetLastError());
     return LNS_OK;
@@ -336,6 +356,7 @@ lns_status bqp_launch_apply(lns_bqp *c, int k, uint64_t M, int64_t L, const BqBu
 // the remainder launched directly; ev0 is recorded after the graph is built (host work).
 lns_status bqp_iterate(lns_bqp *c, int k, uint64_t M, int64_t L, int64_t iters, const BqBufs &b, bool trace)
 {
+    const uint64_t S = bq_tabu_words(M, L);
     lns_status s;
     const int64_t G = std::min<int64_t>(iters, 64);
     int64_t done = 0;
@@ -345,8 +366,8 @@ lns_status bqp_iterate(lns_bqp *c, int k, uint64_t M, int64_t L, int64_t iters, 
         cudaGraphExec_t exec = nullptr;
         CK(cudaStreamBeginCapture(c->st, cudaStreamCaptureModeThreadLocal));
         for (int64_t q = 0; q < G; q++) {
-            lns_status e1 = bqp_launch_eval(c, k, M, b, b.until, nullptr);
-            lns_status e2 = e1 == LNS_OK ? bqp_launch_apply(c, k, M, L, b, trace) : e1;
+            lns_status e1 = bqp_launch_eval(c, k, M, S, b, b.until, nullptr);
+            lns_status e2 = e1 == LNS_OK ? bqp_launch_apply(c, k, M, S, L, b, trace) : e1;
             if (e2 != LNS_OK) { cudaStreamEndCapture(c->st, &graph); if (graph) cudaGraphDestroy(graph); return e2; }
         }
         CK(cudaStreamEndCapture(c->st, &graph));
@@ -363,8 +384,8 @@ lns_status bqp_iterate(lns_bqp *c, int k, uint64_t M, int64_t L, int64_t iters, 
     }
     if (!timing_started) CK(cudaEventRecord(c->ev0, c->st));
     for (; done < iters; done++) {
-        if ((s = bqp_launch_eval(c, k, M, b, b.until, nullptr)) != LNS_OK) return s;
-        if ((s = bqp_launch_apply(c, k, M, L, b, trace)) != LNS_OK) return s;
+        if ((s = bqp_launch_eval(c, k, M, S, b, b.until, nullptr)) != LNS_OK) return s;
+        if ((s = bqp_launch_apply(c, k, M, S, L, b, trace)) != LNS_OK) return s;
     }
     CK(cudaEventRecord(c->ev1, c->st));
     return LNS_OK;
@@ -464,7 +485,7 @@ lns_status lns_bqp_eval_all(lns_bqp *c, int32_t k, const uint8_t *x, int32_t *fi
     if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
     if ((s = bqp_start(c, x, bq_single(c))) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev0, c->st));
-    if ((s = bqp_launch_eval(c, k, M, bq_single(c), nullptr, c->d_fit)) != LNS_OK) return s;
+    if ((s = bqp_launch_eval(c, k, M, 0, bq_single(c), nullptr, c->d_fit)) != LNS_OK) return s;
     CK(cudaEventRecord(c->ev1, c->st));
     int64_t hs[BS_N];
     CK(cudaMemcpyAsync(hs, c->d_st, sizeof(hs), cudaMemcpyDeviceToHost, c->st));
@@ -488,7 +509,8 @@ lns_status lns_bqp_tabu_run(lns_bqp *c, int32_t k, int64_t iters, int64_t tenure
     if (iters + L >= ((int64_t)1 << 32) - 1) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
     DeviceGuard dg(c->device);
     const bool trace = trace_rank || trace_fit;
-    if ((s = grow(c->d_until, c->until_cap, M)) != LNS_OK) return s;
+    const uint64_t S = bq_tabu_words(M, L);
+    if ((s = grow(c->d_until, c->until_cap, S)) != LNS_OK) return s;
     if (trace && c->tr_cap < (size_t)std::max<int64_t>(iters, 1)) {
         pool_free(c->d_tr); pool_free(c->d_tf);
         c->d_tr = c->d_tf = nullptr; c->tr_cap = 0;
@@ -498,7 +520,7 @@ lns_status lns_bqp_tabu_run(lns_bqp *c, int32_t k, int64_t iters, int64_t tenure
         c->tr_cap = cap;
     }
     if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
-    CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * M, c->st));
+    CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * ((M + 31) / 32), c->st));  // the bitmap (the ring fills first)
     if ((s = bqp_start(c, x0, bq_single(c))) != LNS_OK) return s;
     if ((s = bqp_iterate(c, k, M, L, iters, bq_single(c), trace)) != LNS_OK) return s;
     int64_t hs[BS_N];
@@ -530,14 +552,15 @@ lns_status lns_bqp_tabu_run_batch(lns_bqp *c, int32_t k, int32_t R, int64_t iter
     if (iters + L >= ((int64_t)1 << 32) - 1) return fail(LNS_ERANGE, "iters + tenure >= 2^32");
     DeviceGuard dg(c->device);
     const size_t n = (size_t)c->n;
-    if ((s = grow(c->d_until, c->until_cap, M * (size_t)R)) != LNS_OK) return s;
+    const uint64_t S = bq_tabu_words(M, L);
+    if ((s = grow(c->d_until, c->until_cap, S * (size_t)R)) != LNS_OK) return s;
     if ((s = grow(c->d_bx, c->bx_cap, n * R)) != LNS_OK) return s;
     if ((s = grow(c->d_bg, c->bg_cap, n * R)) != LNS_OK) return s;
     if ((s = grow(c->d_bst, c->bst_cap, (size_t)BS_N * R)) != LNS_OK) return s;
     if ((s = grow(c->d_bkey, c->bkey_cap, (size_t)R)) != LNS_OK) return s;
     const BqBufs b{c->d_bx, c->d_bg, c->d_bst, c->d_bkey, c->d_until, R};
     if ((s = bqp_enter(c, stream)) != LNS_OK) return s;
-    CK(cudaMemsetAsync(c->d_until, 0, sizeof(uint32_t) * M * R, c->st));
+    CK(cudaMemset2DAsync(c->d_until, 4 * S, 0, 4 * ((M + 31) / 32), R, c->st));  // each restart's bitmap
     if ((s = bqp_start(c, x0s, b)) != LNS_OK) return s;
     if ((s = bqp_iterate(c, k, M, L, iters, b, false)) != LNS_OK) return s;
     std::vector<int64_t> hs((size_t)BS_N * R);
