@@ -217,6 +217,7 @@ struct PlanScalars {
     // packed path, parity walks (build_plan_pk): records of walk 0 are [0, pkb1),
     // of walk 1 [pkb1, P); first row word of each walk
     int pkb1, pkw0[2];
+    const int *dtab;  // deep rows' per-column counts (cur[] after the plan, deep_table)
     unsigned long long key, gkey;
     int red[2 * NWARP + 2];
 };
@@ -885,8 +886,51 @@ __device__ void build_plan_seg(const DevInst &I, const uint32_t *Ar, unsigned ch
 // its walk -- is <= 255, and so is H_b of every walked bin; else the segment plan. Decided per
 // iteration by warp 0 after the shared counting sort.
 template <int K, bool XG = false, bool OVL = true>
+__device__ void build_plan_body(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                                uint32_t *Xarg, const Move &mv);
+
+// Deep rows' column table: the deep rows' cost is cneg - 240 sum t with
+// sum t = sum_{i in F} #{deep rows j : x_ji = 1}, a sum of per-column counts, so once the plan's X
+// is built every column's count D[c] is tabulated (in cur[], free between plans) and a neighbour
+// reads k entries instead of walking the deep row words. Only when the deep rows span at least
+// DEEP_TAB_MIN_W row words (one more barrier per plan).
+#ifndef DEEP_TAB_MIN_W
+#define DEEP_TAB_MIN_W 2
+#endif
+__device__ __forceinline__ bool deep_tab_on(int rneg) { return ((rneg + 31) >> 5) >= DEEP_TAB_MIN_W; }
+
+template <bool XG>
+__device__ __forceinline__ void deep_table(const DevInst &I, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                                           uint32_t *Xarg)
+{
+    const int rneg = ps.rneg;
+    if (!deep_tab_on(rneg)) return;
+    const uint32_t *X = XG ? Xarg : (const uint32_t *)(sm + L.X);
+    int *D = (int *)(sm + L.cur);
+    if (threadIdx.x == 0) ps.dtab = D;
+    const int nw = (rneg + 31) >> 5, n = I.n;
+    for (int col = threadIdx.x; col < n; col += NT) {
+        int cntc = 0;
+        for (int w = 0; w < nw; w++) {
+            const uint32_t mask = (w == nw - 1 && (rneg & 31)) ? ((1u << (rneg & 31)) - 1u) : FULL;
+            cntc += __popc(X[w * n + col] & mask);
+        }
+        D[col] = cntc;
+    }
+    __syncthreads();
+}
+
+template <int K, bool XG = false, bool OVL = true>
 __device__ void build_plan(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
                            uint32_t *Xarg, const Move &mv = Move{0, 0, 0, 0})
+{
+    build_plan_body<K, XG, OVL>(I, Ar, sm, L, ps, Xarg, mv);
+    deep_table<XG>(I, sm, L, ps, Xarg);
+}
+
+template <int K, bool XG, bool OVL>
+__device__ void build_plan_body(const DevInst &I, const uint32_t *Ar, unsigned char *sm, const Smem &L, PlanScalars &ps,
+                                uint32_t *Xarg, const Move &mv)
 {
     if (I.m <= PACKED_MAX_M) { build_plan_pk<K, XG, OVL>(I, Ar, sm, L, ps, Xarg, mv); return; }
     if (!I.pkw) { build_plan_seg<K, XG>(I, Ar, sm, L, ps, Xarg, mv, false); return; }
@@ -996,6 +1040,7 @@ struct EvalRange {
     int u0, u1;       // lattice points [u0, u1) go through the segment loop (u0 = uneg, u1 = utop)
     int rneg, cneg;   // deep-negative rows [0, rneg) and their constant part
     int p0;           // first piece of point u0
+    const int *dtab;  // deep rows' per-column counts (deep_table), used when deep_tab_on(rneg)
 };
 
 // Deep-negative rows: every destination is negative, cost sum_j 60(2K - Y_j - 4 t_j) - 1
@@ -1005,6 +1050,12 @@ __device__ __forceinline__ int deep_negative(const uint32_t *__restrict__ X, int
                                              int a, int b, int c)
 {
     int st = 0;
+    if (deep_tab_on(er.rneg)) {  // sum t = sum over the flipped columns of their deep-row counts
+        st = er.dtab[a];
+        if (K >= 2) st += er.dtab[b];
+        if (K == 3) st += er.dtab[c];
+        return (int)((unsigned)f + (unsigned)er.cneg - 240u * (unsigned)st);
+    }
     const int nw = (er.rneg + 31) >> 5;
     for (int w = 0; w < nw; w++) {
         const uint32_t mask = (w == nw - 1 && (er.rneg & 31)) ? ((1u << (er.rneg & 31)) - 1u) : FULL;
@@ -1210,7 +1261,7 @@ __device__ __forceinline__ int pk_deep(const uint32_t *__restrict__ X, int n, co
                                        int b, int c)
 {
     EvalRange er;
-    er.rneg = ps.rneg; er.cneg = ps.cneg;
+    er.rneg = ps.rneg; er.cneg = ps.cneg; er.dtab = ps.dtab;
     return deep_negative<K>(X, n, er, f, a, b, c);
 }
 
@@ -1253,7 +1304,7 @@ __device__ unsigned long long eval_range(const DevInst &I, const unsigned char *
     const uint32_t *T2 = (const uint32_t *)(sm + L.T2), *T3 = (const uint32_t *)(sm + L.T3);
     const bool packed = ps.pkok;
     EvalRange er;
-    er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg;
+    er.u0 = ps.uneg; er.u1 = ps.utop; er.rneg = ps.rneg; er.cneg = ps.cneg; er.dtab = (const int *)(sm + L.cur);
     er.p0 = ((const int *)(sm + L.pofs))[ps.uneg];
     // packed path, abs form: C = m - (H of the walked bins) + (rows above the top cut) - 8 (completed
     // bins); deep rows cost 60 |b| each (cneg, accumulated so by build_plan_pk)
