@@ -92,6 +92,36 @@ def test_eval_all_matches_oracle(L, orc, m, n, k):
         L.lns_destroy(ctx)
 
 
+@pytest.mark.parametrize("m,n,k", [(160, 41, 3), (240, 53, 2), (300, 61, 3), (600, 45, 3)])
+def test_deep_rows_table_boundary(L, orc, m, n, k):
+    """The deep rows' column table is used from two deep row words on: states whose
+    deep-negative rows (Y < -2k, every destination negative) number just below, at and above 32
+    and 64 (table off / on) give the oracle's fitness for every neighbour, on the packed path
+    (m <= 255) and the m > 255 path."""
+    inst = pi.planted_instance(m, n, 9100 + m + n)
+    rng = np.random.default_rng(m + k)
+    A = inst.A.astype(np.int32)
+    want_counts = {31, 32, 33, 63, 64, 65, 97}
+    seen = set()
+    ctx = L.lns_create(inst.A, inst.S)
+    try:
+        for trial in range(4000):
+            V = (-inst.secret).astype(np.int8)
+            flip = rng.choice(n, size=int(rng.integers(1, n)), replace=False)
+            V[flip] *= -1
+            deep = int(((A @ V.astype(np.int32)) < -2 * k).sum())
+            if deep not in want_counts or deep in seen:
+                continue
+            seen.add(deep)
+            got = L.lns_eval_all(ctx, k, V).astype(np.int64)
+            assert np.array_equal(got, orc.eval_all(inst.A, inst.S, V, k)), deep
+            if len(seen) == len(want_counts):
+                break
+    finally:
+        L.lns_destroy(ctx)
+    assert {31, 33}.issubset(seen) or {63, 65}.issubset(seen), seen  # both sides of a threshold
+
+
 def test_eval_all_forced_ties_duplicate_columns(L, orc):
     inst = pi.planted_instance(40, 30, 99)
     A = inst.A.copy()
